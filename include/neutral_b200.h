@@ -1,0 +1,180 @@
+/*
+ * neutral_b200.h -- C ABI of the B200-native neutral particle-history tracker.
+ *
+ * The method is the Monte Carlo neutral-particle transport mini-app "neutral" of
+ * Martineau & McIntosh-Smith, "Exploring On-Node Parallelism with Neutral, a Monte Carlo
+ * Neutral Particle Transport Mini-App", IEEE CLUSTER 2017.  "P:L1-L2 (§X)" cites lines of
+ * that paper's text.  The exact arithmetic is DESIGN.md §3; the readings of
+ * the paper it relies on are DESIGN.md §4.
+ *
+ * Conventions for every call:
+ *  - Every call returns nt_status; the library never aborts or exits.  On failure
+ *    nt_last_error(ctx) holds a one-line message (storage owned by ctx).
+ *  - Pointer arguments may be host or device memory (detected with
+ *    cudaPointerGetAttributes, copied with cudaMemcpyDefault).  Inputs are deep-copied
+ *    during the call: the caller keeps ownership and may free them on return.
+ *  - All device memory belongs to the context and is released by nt_destroy.
+ *  - All work is ordered on the context stream (the caller's stream if given).
+ *    nt_run_timestep, nt_read_tally and nt_read_particles synchronise that stream
+ *    before returning.
+ *  - Call order (state machine): nt_create -> nt_init_mesh -> nt_load_cross_sections
+ *    -> nt_inject_particles -> nt_run_timestep (repeatable) -> nt_read_*.
+ *    Out-of-order calls return NT_ERR_STATE.  Re-running an earlier stage
+ *    invalidates the later ones.
+ *  - One context per host thread; contexts are independent.
+ *  - Units: metres, seconds, kg/m^3, eV, barns.  The tally is eV x weight, raw.
+ */
+#ifndef NEUTRAL_B200_H
+#define NEUTRAL_B200_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define NT_ABI_VERSION 1
+
+typedef struct nt_ctx nt_ctx;
+
+typedef enum {
+    NT_OK = 0,
+    NT_ERR_ARG = 1,        /* invalid argument (message says which)                   */
+    NT_ERR_STATE = 2,      /* call out of order                                       */
+    NT_ERR_OOM = 3,        /* device allocation failed                                */
+    NT_ERR_CUDA = 4,       /* CUDA runtime error                                      */
+    NT_ERR_NCCL = 5,       /* NCCL error (nranks > 1)                                 */
+    NT_ERR_XS_RANGE = 6,   /* step completed; some energies were outside a table      */
+    NT_ERR_NONFINITE = 7,  /* step completed; some particle ended non-finite          */
+    NT_ERR_EVENT_CAP = 8,  /* step completed; some history hit max_events_per_history */
+    NT_ERR_UNSUPPORTED = 9 /* feature not available in this build / configuration     */
+} nt_status;
+
+enum { NT_MODE_HISTORY = 0, NT_MODE_EVENT = 1 };
+
+/* Context options.  Zero-initialise (or nt_options_default) and set what you need. */
+typedef struct {
+    int32_t device;            /* CUDA device ordinal                                     */
+    void *stream;              /* cudaStream_t to order work on, or NULL = own stream     */
+    int32_t mode;              /* NT_MODE_HISTORY: Over Particles (§V-A);
+                                  NT_MODE_EVENT: Over Events (§V-B)             */
+    int32_t deterministic;     /* 1: fixed-order tally = the oracle's (particle id, flush
+                                  sequence) order per cell; 0: fp64 atomics   */
+    int32_t rank, nranks;      /* this process's rank and the world size (0, 1 = 1 GPU)   */
+    const void *nccl_unique_id;/* 128-byte ncclUniqueId when nranks > 1 (nt_get_unique_id
+                                  on rank 0, broadcast by the caller)                     */
+    double A;                  /* target mass / neutron mass       (0 -> 1.0)            */
+    double molar_mass;         /* kg/mol                           (0 -> 1e-3)           */
+    double e_min;              /* energy cutoff, eV    (0 -> 1.0)            */
+    double w_min;              /* weight cutoff        (0 -> 1e-3)           */
+    int64_t max_events_per_history; /* guard per history per step  (0 -> 1e9)            */
+    int32_t block_size;        /* threads per CTA of the tracking kernel (0 -> default)   */
+    int32_t ctas_per_sm;       /* persistent CTAs per SM (0 -> occupancy maximum)         */
+    int64_t det_batch;         /* deterministic mode: particles per batch (0 -> 65536)    */
+} nt_options;
+
+/* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,
+ * all ranks -- tracked).  events = n_facets + n_collisions + n_census. */
+typedef struct {
+    uint64_t n_alive_start, n_facets, n_collisions, n_census, n_killed;
+    double tally_total;        /* sum of all deposits flushed this step                  */
+    double census_energy, census_weight;   /* sum of w*E, w over particles at census     */
+    double killed_energy, killed_weight;   /* sum of w*E, w over particles killed        */
+    double absorbed_weight;    /* weight removed by implicit capture          */
+    uint64_t n_xs_range, n_nonfinite, n_event_cap;
+    float track_ms;            /* device time of the tracking kernel(s)                   */
+    float reduce_ms;           /* device time of the cross-GPU tally reduction            */
+    float step_ms;             /* device time of the whole timestep                       */
+    uint32_t n_launches;       /* kernels this library launched for the step              */
+} nt_step_stats;
+
+/* Structure-of-arrays particle view used by nt_read_particles / nt_write_particles.
+ * Each pointer may be NULL (field skipped), a host pointer or a device pointer. */
+typedef struct {
+    double *x, *y;             /* position, m                                             */
+    double *ox, *oy;           /* direction cosines                                       */
+    double *e;                 /* energy, eV                                              */
+    double *w;                 /* weight                                      */
+    double *mfp;               /* mean free paths to the next collision                   */
+    int32_t *cx, *cy;          /* containing cell                                         */
+    uint32_t *ctr;             /* next RNG counter                            */
+    uint8_t *status;           /* 1 alive (at census), 0 dead                             */
+    uint32_t *nfac, *ncol, *ncen; /* cumulative facet / collision / census events         */
+    double *dep;               /* cumulative energy this particle deposited in the tally  */
+} nt_particles;
+
+/* Library identity. */
+int32_t nt_abi_version(void);
+const char *nt_build_info(void);       /* compile flags, arch, det/fmad settings          */
+const char *nt_status_string(nt_status s);
+
+/* Fill *opt with the defaults listed above. */
+nt_status nt_options_default(nt_options *opt);
+
+/* Write a fresh 128-byte ncclUniqueId into out[128] (rank 0 only; for nranks > 1). */
+nt_status nt_get_unique_id(void *out128);
+
+/* Create a context on opt->device.  For nranks > 1 this joins the NCCL communicator
+ * (collective over all ranks).  *out is NULL on failure. */
+nt_status nt_create(const nt_options *opt, nt_ctx **out);
+nt_status nt_destroy(nt_ctx *ctx);     /* NULL is a no-op                                 */
+const char *nt_last_error(const nt_ctx *ctx); /* never NULL                               */
+
+/* The structured 2D mesh of cell-centred mass densities:
+ * nx x ny uniform cells over [0,width] x [0,height], density[ny][nx] row-major, kg/m^3,
+ * finite and >= 0.  Cell edges are edge(i) = (i*width)/nx. */
+nt_status nt_init_mesh(nt_ctx *ctx, int32_t nx, int32_t ny, double width, double height,
+                       const double *density);
+
+/* The two microscopic cross-section tables of one material, scatter and capture
+ * (§IV-D): keys in eV strictly increasing and finite, values in barns finite and
+ * >= 0, n >= 2 each.  Lookup = bin search + linear interpolation. */
+nt_status nt_load_cross_sections(nt_ctx *ctx,
+                                 const double *scatter_keys, const double *scatter_vals,
+                                 int64_t n_scatter,
+                                 const double *capture_keys, const double *capture_vals,
+                                 int64_t n_capture);
+
+/* Create this rank's particles: global ids [first_id, first_id + n_local) of n_total,
+ * positions uniform in the source rectangle [src_x, src_x+src_w] x [src_y, src_y+src_h]
+ * (inside the mesh), isotropic directions, energy initial_energy, weight 1
+ * (§IV-F).  Random numbers: Threefry-2x64-20 keyed by (global id, seed)
+ * (P:296-300), so results do not depend on how ids are split across ranks. */
+nt_status nt_inject_particles(nt_ctx *ctx, int64_t n_total, int64_t first_id,
+                              int64_t n_local, double src_x, double src_y, double src_w,
+                              double src_h, double initial_energy, uint64_t seed);
+
+/* Track every alive particle for one timestep of length dt seconds until census or death
+ * (Listing 1, or Listing 2 P:362-373 in event mode).  Zeroes the tally first
+ * (the tally is per timestep), then accumulates every flushed deposit
+ * (P:391-401).  When nranks > 1 the tally and stats are summed over ranks (NCCL
+ * allreduce over NVLink) -- a collective call.  Device-side anomalies do not abort the
+ * step: it completes, stats are filled, and the return is NT_ERR_XS_RANGE,
+ * NT_ERR_NONFINITE or NT_ERR_EVENT_CAP.  stats may be NULL. */
+nt_status nt_run_timestep(nt_ctx *ctx, double dt, nt_step_stats *stats);
+
+/* Copy the per-cell tally [ny][nx] (f64) of the last step into dst (host or device).
+ * reduced = 1: the cross-rank sum (equal to the local tally when nranks == 1);
+ * reduced = 0: this rank's own partial tally (kept only when nranks > 1). */
+nt_status nt_read_tally(nt_ctx *ctx, double *dst, int32_t reduced);
+
+/* Copy local particles [first, first+count) (local indices) into dst's arrays. */
+nt_status nt_read_particles(nt_ctx *ctx, int64_t first, int64_t count,
+                            const nt_particles *dst);
+/* Overwrite local particles [first, first+count) from src (checkpoint / resume: the RNG
+ * is counter based, so a restored particle continues bit-exactly). */
+nt_status nt_write_particles(nt_ctx *ctx, int64_t first, int64_t count,
+                             const nt_particles *src);
+
+/* Verification entry points (run the device code paths in isolation). */
+/* out[2i], out[2i+1] = threefry2x64_20(ctr = {in[4i], in[4i+1]}, key = {in[4i+2], in[4i+3]}). */
+nt_status nt_debug_threefry(nt_ctx *ctx, const uint64_t *in, int64_t n, uint64_t *out);
+/* Microscopic XS from the loaded tables: out_s[i], out_a[i] at energies[i] (no clamp
+ * counting). */
+nt_status nt_debug_xs(nt_ctx *ctx, const double *energies, int64_t n, double *out_s,
+                      double *out_a);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* NEUTRAL_B200_H */

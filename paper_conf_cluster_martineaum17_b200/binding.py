@@ -1,0 +1,266 @@
+"""Thin ctypes binding of the C ABI in include/neutral_b200.h (argument marshalling only).
+
+Every step of the method runs in the CUDA kernels of ``lib/libneutral_b200.so``; this
+module only converts numpy arrays / torch tensors to pointers and status codes to
+exceptions.  There is no CPU fallback: if the library is missing, loading fails loudly.
+"""
+from __future__ import annotations
+
+import ctypes as C
+from pathlib import Path
+
+import numpy as np
+
+LIB_PATH = Path(__file__).resolve().parent / "lib" / "libneutral_b200.so"
+
+NT_OK = 0
+STATUS = {0: "NT_OK", 1: "NT_ERR_ARG", 2: "NT_ERR_STATE", 3: "NT_ERR_OOM", 4: "NT_ERR_CUDA",
+          5: "NT_ERR_NCCL", 6: "NT_ERR_XS_RANGE", 7: "NT_ERR_NONFINITE",
+          8: "NT_ERR_EVENT_CAP", 9: "NT_ERR_UNSUPPORTED"}
+STEP_ANOMALIES = {6, 7, 8}     # the step completed; stats are valid
+MODES = {"history": 0, "event": 1}
+
+# Every function the header declares (tests check the library exports all of them).
+EXPORTS = ["nt_abi_version", "nt_build_info", "nt_status_string", "nt_options_default",
+           "nt_get_unique_id", "nt_create", "nt_destroy", "nt_last_error", "nt_init_mesh",
+           "nt_load_cross_sections", "nt_inject_particles", "nt_run_timestep", "nt_read_tally",
+           "nt_read_particles", "nt_write_particles", "nt_debug_threefry", "nt_debug_xs"]
+
+
+class NeutralError(RuntimeError):
+    def __init__(self, status: int, msg: str):
+        super().__init__(f"{STATUS.get(status, status)}: {msg}")
+        self.status = status
+
+
+class Options(C.Structure):
+    _fields_ = [("device", C.c_int32), ("stream", C.c_void_p), ("mode", C.c_int32),
+                ("deterministic", C.c_int32), ("rank", C.c_int32), ("nranks", C.c_int32),
+                ("nccl_unique_id", C.c_void_p), ("A", C.c_double), ("molar_mass", C.c_double),
+                ("e_min", C.c_double), ("w_min", C.c_double),
+                ("max_events_per_history", C.c_int64), ("block_size", C.c_int32),
+                ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64)]
+
+
+class StepStats(C.Structure):
+    _fields_ = [("n_alive_start", C.c_uint64), ("n_facets", C.c_uint64),
+                ("n_collisions", C.c_uint64), ("n_census", C.c_uint64), ("n_killed", C.c_uint64),
+                ("tally_total", C.c_double), ("census_energy", C.c_double),
+                ("census_weight", C.c_double), ("killed_energy", C.c_double),
+                ("killed_weight", C.c_double), ("absorbed_weight", C.c_double),
+                ("n_xs_range", C.c_uint64), ("n_nonfinite", C.c_uint64),
+                ("n_event_cap", C.c_uint64), ("track_ms", C.c_float), ("reduce_ms", C.c_float),
+                ("step_ms", C.c_float), ("n_launches", C.c_uint32)]
+
+
+PARTICLE_FIELDS = [("x", np.float64), ("y", np.float64), ("ox", np.float64), ("oy", np.float64),
+                   ("e", np.float64), ("w", np.float64), ("mfp", np.float64), ("cx", np.int32),
+                   ("cy", np.int32), ("ctr", np.uint32), ("status", np.uint8),
+                   ("nfac", np.uint32), ("ncol", np.uint32), ("ncen", np.uint32),
+                   ("dep", np.float64)]
+
+
+class ParticlesView(C.Structure):
+    _fields_ = [(n, C.c_void_p) for n, _ in PARTICLE_FIELDS]
+
+
+_lib = None
+
+
+def lib():
+    """Load the CUDA library (fails loudly when it has not been built)."""
+    global _lib
+    if _lib is None:
+        if not LIB_PATH.exists():
+            raise ImportError(f"{LIB_PATH} is missing: run `python -m "
+                              "paper_conf_cluster_martineaum17_b200.build` (no CPU fallback)")
+        L = C.CDLL(str(LIB_PATH))
+        vp, i32, i64, u64, d = C.c_void_p, C.c_int32, C.c_int64, C.c_uint64, C.c_double
+        sigs = {
+            "nt_abi_version": ([], i32),
+            "nt_build_info": ([], C.c_char_p),
+            "nt_status_string": ([C.c_int], C.c_char_p),
+            "nt_options_default": ([C.POINTER(Options)], C.c_int),
+            "nt_get_unique_id": ([vp], C.c_int),
+            "nt_create": ([C.POINTER(Options), C.POINTER(vp)], C.c_int),
+            "nt_destroy": ([vp], C.c_int),
+            "nt_last_error": ([vp], C.c_char_p),
+            "nt_init_mesh": ([vp, i32, i32, d, d, vp], C.c_int),
+            "nt_load_cross_sections": ([vp, vp, vp, i64, vp, vp, i64], C.c_int),
+            "nt_inject_particles": ([vp, i64, i64, i64, d, d, d, d, d, u64], C.c_int),
+            "nt_run_timestep": ([vp, d, C.POINTER(StepStats)], C.c_int),
+            "nt_read_tally": ([vp, vp, i32], C.c_int),
+            "nt_read_particles": ([vp, i64, i64, C.POINTER(ParticlesView)], C.c_int),
+            "nt_write_particles": ([vp, i64, i64, C.POINTER(ParticlesView)], C.c_int),
+            "nt_debug_threefry": ([vp, vp, i64, vp], C.c_int),
+            "nt_debug_xs": ([vp, vp, i64, vp, vp], C.c_int),
+        }
+        for name, (args, res) in sigs.items():
+            f = getattr(L, name)
+            f.argtypes = args
+            f.restype = res
+        _lib = L
+    return _lib
+
+
+def get_unique_id() -> bytes:
+    buf = C.create_string_buffer(128)
+    st = lib().nt_get_unique_id(buf)
+    if st != NT_OK:
+        raise NeutralError(st, "ncclGetUniqueId failed")
+    return buf.raw
+
+
+def _ptr(a):
+    """(pointer, keepalive) for a numpy array or torch tensor (host or CUDA)."""
+    if a is None:
+        return None, None
+    if isinstance(a, np.ndarray):
+        if not a.flags["C_CONTIGUOUS"]:
+            a = np.ascontiguousarray(a)
+        return a.ctypes.data, a
+    if hasattr(a, "data_ptr"):
+        assert a.is_contiguous(), "tensor must be contiguous"
+        return a.data_ptr(), a
+    raise TypeError(f"unsupported array type {type(a)}")
+
+
+def _f64(a):
+    if isinstance(a, np.ndarray):
+        return np.ascontiguousarray(a, dtype=np.float64)
+    import torch
+    if isinstance(a, torch.Tensor):
+        assert a.dtype == torch.float64
+        return a.contiguous()
+    return np.ascontiguousarray(np.asarray(a, dtype=np.float64))
+
+
+class Tracker:
+    """One nt_ctx: a 2D mesh, two XS tables, this rank's particles, and its tally."""
+
+    def __init__(self, device: int = 0, stream=None, mode: str = "history",
+                 deterministic: bool = False, rank: int = 0, nranks: int = 1,
+                 unique_id: bytes | None = None, A: float = 1.0, molar_mass: float = 1e-3,
+                 e_min: float = 1.0, w_min: float = 1e-3, max_events: int = 0,
+                 ctas_per_sm: int = 0, det_batch: int = 0):
+        L = lib()
+        o = Options()
+        L.nt_options_default(C.byref(o))
+        o.device = device
+        o.stream = stream
+        o.mode = MODES[mode]
+        o.deterministic = int(bool(deterministic))
+        o.rank, o.nranks = rank, nranks
+        self._uid = C.create_string_buffer(unique_id, 128) if unique_id else None
+        o.nccl_unique_id = C.cast(self._uid, C.c_void_p) if self._uid else None
+        o.A, o.molar_mass, o.e_min, o.w_min = A, molar_mass, e_min, w_min
+        o.max_events_per_history = max_events
+        o.ctas_per_sm = ctas_per_sm
+        o.det_batch = det_batch
+        h = C.c_void_p()
+        st = L.nt_create(C.byref(o), C.byref(h))
+        if st != NT_OK:
+            raise NeutralError(st, "nt_create failed")
+        self._h = h
+        self.nx = self.ny = 0
+        self.n_local = 0
+
+    # -- helpers ---------------------------------------------------------------------------
+    def _check(self, st: int, what: str, allow=()):
+        if st != NT_OK and st not in allow:
+            raise NeutralError(st, f"{what}: {lib().nt_last_error(self._h).decode()}")
+        return st
+
+    def close(self):
+        if getattr(self, "_h", None):
+            lib().nt_destroy(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.close()
+
+    # -- the five calls of the boundary -------------------------------------------------------
+    def init_mesh(self, nx: int, ny: int, width: float, height: float, density):
+        p, keep = _ptr(_f64(density))
+        self._check(lib().nt_init_mesh(self._h, nx, ny, width, height, p), "nt_init_mesh")
+        self.nx, self.ny = nx, ny
+
+    def load_cross_sections(self, scatter_keys, scatter_vals, capture_keys, capture_vals):
+        arrs = [_f64(a) for a in (scatter_keys, scatter_vals, capture_keys, capture_vals)]
+        ps = [_ptr(a)[0] for a in arrs]
+        self._check(lib().nt_load_cross_sections(self._h, ps[0], ps[1], len(arrs[0]), ps[2], ps[3],
+                                                 len(arrs[2])), "nt_load_cross_sections")
+
+    def inject_particles(self, n_total: int, first_id: int, n_local: int, source, initial_energy: float,
+                         seed: int):
+        sx, sy, sw, sh = source
+        self._check(lib().nt_inject_particles(self._h, n_total, first_id, n_local, sx, sy, sw, sh,
+                                              initial_energy, seed), "nt_inject_particles")
+        self.n_local = n_local
+
+    def run_timestep(self, dt: float) -> dict:
+        s = StepStats()
+        st = self._check(lib().nt_run_timestep(self._h, dt, C.byref(s)), "nt_run_timestep",
+                         allow=STEP_ANOMALIES)
+        d = {n: getattr(s, n) for n, _ in StepStats._fields_}
+        d["status"] = st
+        d["events"] = d["n_facets"] + d["n_collisions"] + d["n_census"]
+        return d
+
+    def read_tally(self, out=None, reduced: bool = True):
+        if out is None:
+            out = np.empty((self.ny, self.nx), dtype=np.float64)
+        p, _ = _ptr(out)
+        self._check(lib().nt_read_tally(self._h, p, int(reduced)), "nt_read_tally")
+        return out
+
+    # -- verification / checkpoint ------------------------------------------------------------
+    def read_particles(self, first: int = 0, count: int | None = None) -> dict:
+        if count is None:
+            count = self.n_local - first
+        out = {n: np.empty(count, dtype=t) for n, t in PARTICLE_FIELDS}
+        v = ParticlesView(*[out[n].ctypes.data for n, _ in PARTICLE_FIELDS])
+        self._check(lib().nt_read_particles(self._h, first, count, C.byref(v)), "nt_read_particles")
+        return out
+
+    def write_particles(self, first: int, fields: dict):
+        count = len(next(iter(fields.values())))
+        keep = {n: np.ascontiguousarray(fields[n], dtype=t) for n, t in PARTICLE_FIELDS if n in fields}
+        v = ParticlesView(*[keep[n].ctypes.data if n in keep else None for n, _ in PARTICLE_FIELDS])
+        self._check(lib().nt_write_particles(self._h, first, count, C.byref(v)), "nt_write_particles")
+
+    def debug_threefry(self, inputs: np.ndarray) -> np.ndarray:
+        inp = np.ascontiguousarray(inputs, dtype=np.uint64).reshape(-1, 4)
+        out = np.empty((len(inp), 2), dtype=np.uint64)
+        self._check(lib().nt_debug_threefry(self._h, inp.ctypes.data, len(inp), out.ctypes.data),
+                    "nt_debug_threefry")
+        return out
+
+    def debug_xs(self, energies: np.ndarray):
+        e = np.ascontiguousarray(energies, dtype=np.float64)
+        os_, oa = np.empty_like(e), np.empty_like(e)
+        self._check(lib().nt_debug_xs(self._h, e.ctypes.data, len(e), os_.ctypes.data, oa.ctypes.data),
+                    "nt_debug_xs")
+        return os_, oa
+
+
+def setup(cfg, *, density=None, tables=None, first_id: int = 0, n_local: int | None = None,
+          **opts) -> Tracker:
+    """Create a Tracker for a workloads.Config: mesh, tables and injected particles."""
+    from . import workloads as wl
+    t = Tracker(A=cfg.A, molar_mass=cfg.molar_mass, e_min=cfg.e_min, w_min=cfg.w_min, **opts)
+    t.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, wl.density(cfg) if density is None else density)
+    t.load_cross_sections(*(wl.tables(cfg) if tables is None else tables))
+    if n_local is None:
+        n_local = cfg.n_particles - first_id
+    t.inject_particles(cfg.n_particles, first_id, n_local, cfg.source, cfg.e0, cfg.seed)
+    return t

@@ -1,0 +1,704 @@
+// nt_api.cu -- the C ABI (include/neutral_b200.h): context state machine, device
+// allocations, argument validation, step orchestration, NCCL reduction.
+//
+// Host-side orchestration only; every step of the method runs in the kernels of
+// nt_kernels.cu / nt_event.cu.
+#include <nccl.h>
+
+#include <cmath>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <string>
+#include <vector>
+
+#include "../../include/neutral_b200.h"
+#include "nt_event.h"
+#include "nt_internal.h"
+
+using namespace nt;
+
+namespace {
+
+enum Stage { ST_CREATED = 0, ST_MESH = 1, ST_XS = 2, ST_PARTICLES = 3, ST_STEPPED = 4 };
+
+struct DevBuf {
+  void* p = nullptr;
+  size_t bytes = 0;
+  cudaError_t ensure(size_t b) {
+    if (b <= bytes && p) return cudaSuccess;
+    if (p) cudaFree(p);
+    p = nullptr;
+    bytes = 0;
+    if (b == 0) return cudaSuccess;
+    cudaError_t e = cudaMalloc(&p, b);
+    if (e == cudaSuccess) bytes = b;
+    return e;
+  }
+  void release() {
+    if (p) cudaFree(p);
+    p = nullptr;
+    bytes = 0;
+  }
+  template <class T> T* as() const { return static_cast<T*>(p); }
+};
+
+}  // namespace
+
+struct nt_ctx {
+  nt_options opt{};
+  std::string err;
+  int stage = ST_CREATED;
+  int device = 0;
+  int sm_count = 0;
+  cudaStream_t stream = nullptr;
+  bool own_stream = false;
+  cudaEvent_t ev[6] = {};
+  ncclComm_t comm = nullptr;
+  Phys ph{};
+  // mesh
+  int32_t nx = 0, ny = 0;
+  double W = 0, H = 0;
+  DevBuf rho, tally, tally_local, ex, ey;
+  // tables
+  DevBuf xs;
+  Tables tables{};
+  // particles
+  int64_t n_total = 0, first_id = 0, n_local = 0;
+  uint64_t seed = 0;
+  DevBuf soa;
+  Soa p{};
+  // step scratch: [counter][stats_u][stats_f]
+  DevBuf scratch;
+  // deterministic mode
+  DevBuf rec_key, rec_val, rec_key2, rec_val2, sort_tmp, backup;
+  unsigned long long rec_cap = 0;
+  // event mode
+  EventState* evs = nullptr;
+};
+
+namespace {
+
+nt_status fail(nt_ctx* c, nt_status s, const char* fmt, ...) {
+  if (c) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof buf, fmt, ap);
+    va_end(ap);
+    c->err = buf;
+  }
+  return s;
+}
+
+#define NT_CUDA(c, call)                                                                \
+  do {                                                                                  \
+    cudaError_t e_ = (call);                                                            \
+    if (e_ != cudaSuccess)                                                              \
+      return fail((c), e_ == cudaErrorMemoryAllocation ? NT_ERR_OOM : NT_ERR_CUDA,      \
+                  "%s: %s (%s:%d)", #call, cudaGetErrorString(e_), __FILE__, __LINE__); \
+  } while (0)
+
+#define NT_NCCL(c, call)                                                                \
+  do {                                                                                  \
+    ncclResult_t r_ = (call);                                                           \
+    if (r_ != ncclSuccess)                                                              \
+      return fail((c), NT_ERR_NCCL, "%s: %s", #call, ncclGetErrorString(r_));           \
+  } while (0)
+
+bool is_fin(double v) { return std::isfinite(v); }
+
+// Copy n bytes from a host-or-device pointer into device memory.
+cudaError_t copy_in(void* dst, const void* src, size_t n, cudaStream_t s) {
+  if (n == 0) return cudaSuccess;
+  return cudaMemcpyAsync(dst, src, n, cudaMemcpyDefault, s);
+}
+
+// Read a host-or-device array into a host vector (for validation).
+template <class T>
+cudaError_t fetch(std::vector<T>& out, const T* src, int64_t n, cudaStream_t s) {
+  out.resize((size_t)n);
+  cudaError_t e = cudaMemcpyAsync(out.data(), src, sizeof(T) * (size_t)n, cudaMemcpyDefault, s);
+  if (e != cudaSuccess) return e;
+  return cudaStreamSynchronize(s);
+}
+
+size_t align256(size_t b) { return (b + 255) & ~(size_t)255; }
+
+void init_phys(nt_ctx* c) {
+  const double A = c->opt.A;
+  Phys& p = c->ph;
+  p.A = A;
+  p.AA = A * A;
+  p.twoA = 2.0 * A;
+  p.Ap1 = A + 1.0;
+  p.Am1 = A - 1.0;
+  p.Ap1sq = (A + 1.0) * (A + 1.0);
+  p.f = (A * A + 1.0) / ((A + 1.0) * (A + 1.0));
+  p.cn = kAvogadro / c->opt.molar_mass;
+  p.kv = (2.0 * kEv) / kNeutronMass;
+  p.e_min = c->opt.e_min;
+  p.w_min = c->opt.w_min;
+}
+
+}  // namespace
+
+// =========================================================================================
+extern "C" {
+
+int32_t nt_abi_version(void) { return NT_ABI_VERSION; }
+
+const char* nt_build_info(void) {
+  return "neutral_b200 sm_100a; nvcc -fmad=false -O3; history+event tracking; "
+         "fp64 RED tally / deterministic record-sort tally; NCCL allreduce";
+}
+
+const char* nt_status_string(nt_status s) {
+  switch (s) {
+    case NT_OK: return "NT_OK";
+    case NT_ERR_ARG: return "NT_ERR_ARG";
+    case NT_ERR_STATE: return "NT_ERR_STATE";
+    case NT_ERR_OOM: return "NT_ERR_OOM";
+    case NT_ERR_CUDA: return "NT_ERR_CUDA";
+    case NT_ERR_NCCL: return "NT_ERR_NCCL";
+    case NT_ERR_XS_RANGE: return "NT_ERR_XS_RANGE";
+    case NT_ERR_NONFINITE: return "NT_ERR_NONFINITE";
+    case NT_ERR_EVENT_CAP: return "NT_ERR_EVENT_CAP";
+    case NT_ERR_UNSUPPORTED: return "NT_ERR_UNSUPPORTED";
+  }
+  return "NT_ERR_UNKNOWN";
+}
+
+nt_status nt_options_default(nt_options* opt) {
+  if (!opt) return NT_ERR_ARG;
+  std::memset(opt, 0, sizeof *opt);
+  opt->nranks = 1;
+  opt->A = 1.0;
+  opt->molar_mass = 1.0e-3;
+  opt->e_min = 1.0;
+  opt->w_min = 1.0e-3;
+  opt->max_events_per_history = 1000000000ll;
+  opt->det_batch = 65536;
+  return NT_OK;
+}
+
+nt_status nt_get_unique_id(void* out128) {
+  if (!out128) return NT_ERR_ARG;
+  ncclUniqueId id;
+  if (ncclGetUniqueId(&id) != ncclSuccess) return NT_ERR_NCCL;
+  static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId size");
+  std::memcpy(out128, &id, sizeof id);
+  return NT_OK;
+}
+
+const char* nt_last_error(const nt_ctx* ctx) {
+  if (!ctx) return "null context";
+  return ctx->err.c_str();
+}
+
+nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
+  if (!out) return NT_ERR_ARG;
+  *out = nullptr;
+  nt_options def;
+  nt_options_default(&def);
+  nt_options opt = opt_in ? *opt_in : def;
+  if (opt.nranks <= 0) opt.nranks = 1;
+  if (opt.A == 0.0) opt.A = def.A;
+  if (opt.molar_mass == 0.0) opt.molar_mass = def.molar_mass;
+  if (opt.e_min == 0.0) opt.e_min = def.e_min;
+  if (opt.w_min == 0.0) opt.w_min = def.w_min;
+  if (opt.max_events_per_history <= 0) opt.max_events_per_history = def.max_events_per_history;
+  if (opt.det_batch <= 0) opt.det_batch = def.det_batch;
+  if (opt.det_batch > 65536) opt.det_batch = 65536;
+  if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
+      !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
+      opt.rank < 0 || opt.rank >= opt.nranks)
+    return NT_ERR_ARG;
+  if (opt.nranks > 1 && !opt.nccl_unique_id) return NT_ERR_ARG;
+
+  nt_ctx* c = new nt_ctx();
+  c->opt = opt;
+  c->device = opt.device;
+  cudaError_t e = cudaSetDevice(opt.device);
+  if (e != cudaSuccess) {
+    delete c;
+    return NT_ERR_CUDA;
+  }
+  cudaDeviceGetAttribute(&c->sm_count, cudaDevAttrMultiProcessorCount, opt.device);
+  if (opt.stream) {
+    c->stream = static_cast<cudaStream_t>(opt.stream);
+  } else {
+    if (cudaStreamCreateWithFlags(&c->stream, cudaStreamNonBlocking) != cudaSuccess) {
+      delete c;
+      return NT_ERR_CUDA;
+    }
+    c->own_stream = true;
+  }
+  for (auto& ev : c->ev) cudaEventCreate(&ev);
+  init_phys(c);
+  if (opt.nranks > 1) {
+    ncclUniqueId id;
+    std::memcpy(&id, opt.nccl_unique_id, sizeof id);
+    ncclResult_t r = ncclCommInitRank(&c->comm, opt.nranks, id, opt.rank);
+    if (r != ncclSuccess) {
+      nt_destroy(c);
+      return NT_ERR_NCCL;
+    }
+  }
+  *out = c;
+  return NT_OK;
+}
+
+nt_status nt_destroy(nt_ctx* c) {
+  if (!c) return NT_OK;
+  cudaSetDevice(c->device);
+  if (c->stream) cudaStreamSynchronize(c->stream);
+  if (c->evs) event_state_destroy(c->evs);
+  for (DevBuf* b : {&c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
+                    &c->scratch, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
+                    &c->sort_tmp, &c->backup})
+    b->release();
+  for (auto& ev : c->ev)
+    if (ev) cudaEventDestroy(ev);
+  if (c->comm) ncclCommDestroy(c->comm);
+  if (c->own_stream && c->stream) cudaStreamDestroy(c->stream);
+  delete c;
+  return NT_OK;
+}
+
+// ---- mesh ----------------------------------------------------------
+nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double height,
+                       const double* density) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (nx < 1 || ny < 1) return fail(c, NT_ERR_ARG, "nx, ny must be >= 1 (got %d, %d)", nx, ny);
+  if (!(width > 0.0) || !(height > 0.0) || !is_fin(width) || !is_fin(height))
+    return fail(c, NT_ERR_ARG, "width, height must be finite and > 0");
+  if (!density) return fail(c, NT_ERR_ARG, "density is NULL");
+  const size_t cells = (size_t)nx * (size_t)ny;
+  std::vector<double> h;
+  NT_CUDA(c, fetch(h, density, (int64_t)cells, c->stream));
+  for (size_t k = 0; k < cells; ++k)
+    if (!(h[k] >= 0.0) || !is_fin(h[k]))
+      return fail(c, NT_ERR_ARG, "density[%zu] = %g is not finite and >= 0", k, h[k]);
+  NT_CUDA(c, c->rho.ensure(cells * 8));
+  NT_CUDA(c, c->tally.ensure(cells * 8));
+  NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
+  NT_CUDA(c, c->ey.ensure(((size_t)ny + 1) * 8));
+  NT_CUDA(c, cudaMemcpyAsync(c->rho.p, h.data(), cells * 8, cudaMemcpyHostToDevice, c->stream));
+  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, cells * 8, c->stream));
+  launch_edges(c->ex.as<double>(), nx, width, c->ey.as<double>(), ny, height, c->stream);
+  NT_CUDA(c, cudaGetLastError());
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  c->nx = nx;
+  c->ny = ny;
+  c->W = width;
+  c->H = height;
+  c->stage = ST_MESH;
+  return NT_OK;
+}
+
+// ---- cross sections ---------------------------------------------------------
+nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, int64_t ns,
+                                 const double* ck, const double* cv, int64_t nc) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->stage < ST_MESH) return fail(c, NT_ERR_STATE, "nt_init_mesh must come first");
+  if (ns < 2 || nc < 2 || ns > (1ll << 30) || nc > (1ll << 30))
+    return fail(c, NT_ERR_ARG, "table sizes must be in [2, 2^30]");
+  if (!sk || !sv || !ck || !cv) return fail(c, NT_ERR_ARG, "table pointer is NULL");
+  const double* src[4] = {sk, sv, ck, cv};
+  const int64_t len[4] = {ns, ns, nc, nc};
+  std::vector<double> h[4];
+  for (int k = 0; k < 4; ++k) NT_CUDA(c, fetch(h[k], src[k], len[k], c->stream));
+  for (int k = 0; k < 4; k += 2) {
+    for (int64_t j = 0; j < len[k]; ++j) {
+      if (!is_fin(h[k][j])) return fail(c, NT_ERR_ARG, "table %d key %lld not finite", k / 2, (long long)j);
+      if (j > 0 && !(h[k][j] > h[k][j - 1]))
+        return fail(c, NT_ERR_ARG, "table %d keys not strictly increasing at %lld", k / 2, (long long)j);
+      if (!is_fin(h[k + 1][j]) || !(h[k + 1][j] >= 0.0))
+        return fail(c, NT_ERR_ARG, "table %d value %lld not finite and >= 0", k / 2, (long long)j);
+    }
+  }
+  size_t off[4], total = 0;
+  for (int k = 0; k < 4; ++k) {
+    off[k] = total;
+    total += align256((size_t)len[k] * 8);
+  }
+  NT_CUDA(c, c->xs.ensure(total));
+  for (int k = 0; k < 4; ++k)
+    NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k].data(), (size_t)len[k] * 8,
+                               cudaMemcpyHostToDevice, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  c->tables.sk = reinterpret_cast<const double*>(c->xs.as<char>() + off[0]);
+  c->tables.sv = reinterpret_cast<const double*>(c->xs.as<char>() + off[1]);
+  c->tables.ck = reinterpret_cast<const double*>(c->xs.as<char>() + off[2]);
+  c->tables.cv = reinterpret_cast<const double*>(c->xs.as<char>() + off[3]);
+  c->tables.ns = (int32_t)ns;
+  c->tables.nc = (int32_t)nc;
+  c->stage = ST_XS;
+  return NT_OK;
+}
+
+// ---- particles ------------------------------------------------------------
+static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
+  const size_t N = (size_t)(n > 0 ? n : 1);
+  const size_t b8 = align256(N * 8), b4 = align256(N * 4), b1 = align256(N);
+  cudaError_t e = c->soa.ensure(8 * b8 + 6 * b4 + b1);
+  if (e != cudaSuccess) return e;
+  char* q = c->soa.as<char>();
+  double** d8[8] = {&c->p.x, &c->p.y, &c->p.ox, &c->p.oy, &c->p.e, &c->p.w, &c->p.mfp, &c->p.dep};
+  for (auto d : d8) { *d = reinterpret_cast<double*>(q); q += b8; }
+  c->p.cx = reinterpret_cast<int32_t*>(q); q += b4;
+  c->p.cy = reinterpret_cast<int32_t*>(q); q += b4;
+  c->p.ctr = reinterpret_cast<uint32_t*>(q); q += b4;
+  c->p.nfac = reinterpret_cast<uint32_t*>(q); q += b4;
+  c->p.ncol = reinterpret_cast<uint32_t*>(q); q += b4;
+  c->p.ncen = reinterpret_cast<uint32_t*>(q); q += b4;
+  c->p.status = reinterpret_cast<uint8_t*>(q);
+  return cudaSuccess;
+}
+
+nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int64_t n_local,
+                              double sx, double sy, double sw, double sh, double e0,
+                              uint64_t seed) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->stage < ST_XS) return fail(c, NT_ERR_STATE, "mesh and cross sections must be loaded first");
+  if (n_total < 0 || first_id < 0 || n_local < 0 || first_id + n_local > n_total)
+    return fail(c, NT_ERR_ARG, "need 0 <= first_id, n_local and first_id + n_local <= n_total");
+  if (!(sw >= 0.0) || !(sh >= 0.0) || !(sx >= 0.0) || !(sy >= 0.0) || !(sx + sw <= c->W) ||
+      !(sy + sh <= c->H))
+    return fail(c, NT_ERR_ARG, "source rectangle must lie inside the mesh");
+  if (!(e0 > 0.0) || !is_fin(e0)) return fail(c, NT_ERR_ARG, "initial_energy must be finite and > 0");
+  NT_CUDA(c, alloc_soa(c, n_local));
+  InjectParams ip{};
+  ip.p = c->p;
+  ip.ex = c->ex.as<double>();
+  ip.ey = c->ey.as<double>();
+  ip.nx = c->nx;
+  ip.ny = c->ny;
+  ip.W = c->W;
+  ip.H = c->H;
+  ip.n_local = n_local;
+  ip.first_id = first_id;
+  ip.sx = sx;
+  ip.sy = sy;
+  ip.sw = sw;
+  ip.sh = sh;
+  ip.e0 = e0;
+  ip.seed = seed;
+  launch_inject(ip, c->stream);
+  NT_CUDA(c, cudaGetLastError());
+  c->n_total = n_total;
+  c->first_id = first_id;
+  c->n_local = n_local;
+  c->seed = seed;
+  if (c->evs) event_state_invalidate(c->evs);
+  c->stage = ST_PARTICLES;
+  return NT_OK;
+}
+
+// ---- timestep ---------------------------------------------------------------------------
+static TrackParams make_params(nt_ctx* c, double dt) {
+  TrackParams tp{};
+  tp.mesh.rho = c->rho.as<double>();
+  tp.mesh.tally = c->tally.as<double>();
+  tp.mesh.ex = c->ex.as<double>();
+  tp.mesh.ey = c->ey.as<double>();
+  tp.mesh.nx = c->nx;
+  tp.mesh.ny = c->ny;
+  tp.xs = c->tables;
+  tp.ph = c->ph;
+  tp.p = c->p;
+  tp.n = c->n_local;
+  tp.lo = 0;
+  tp.hi = c->n_local;
+  tp.first_id = c->first_id;
+  tp.seed = c->seed;
+  tp.dt = dt;
+  tp.max_events = c->opt.max_events_per_history;
+  char* s = c->scratch.as<char>();
+  tp.counter = reinterpret_cast<unsigned long long*>(s);
+  tp.stats_u = reinterpret_cast<unsigned long long*>(s + 256);
+  tp.stats_f = reinterpret_cast<double*>(s + 512);
+  return tp;
+}
+
+static int history_grid(nt_ctx* c, bool det) {
+  int per_sm = history_max_ctas_per_sm(det, kHistoryBlock);
+  if (per_sm < 1) per_sm = 1;
+  if (c->opt.ctas_per_sm > 0 && c->opt.ctas_per_sm < per_sm) per_sm = c->opt.ctas_per_sm;
+  return c->sm_count * per_sm;
+}
+
+// Deterministic mode: batches of <= 65536 particles, records sorted by (cell, particle,
+// sequence) and applied serially per cell, batch after batch -> the oracle's sum order.
+// A batch whose records overflow the buffer is restored (particles and statistics) and
+// re-run with a larger buffer or, at the buffer limit, half the particles.
+static nt_status det_snapshot(nt_ctx* c, int64_t lo, int64_t nb, bool restore) {
+  char* b = c->backup.as<char>();
+  auto mv = [&](void* col, size_t sz) -> cudaError_t {
+    char* d = static_cast<char*>(col) + (size_t)lo * sz;
+    cudaError_t e = restore ? cudaMemcpyAsync(d, b, (size_t)nb * sz, cudaMemcpyDeviceToDevice, c->stream)
+                            : cudaMemcpyAsync(b, d, (size_t)nb * sz, cudaMemcpyDeviceToDevice, c->stream);
+    b += align256((size_t)nb * sz);
+    return e;
+  };
+  void* d8[8] = {c->p.x, c->p.y, c->p.ox, c->p.oy, c->p.e, c->p.w, c->p.mfp, c->p.dep};
+  for (void* d : d8) NT_CUDA(c, mv(d, 8));
+  void* d4[6] = {c->p.cx, c->p.cy, c->p.ctr, c->p.nfac, c->p.ncol, c->p.ncen};
+  for (void* d : d4) NT_CUDA(c, mv(d, 4));
+  NT_CUDA(c, mv(c->p.status, 1));
+  // step statistics accumulated so far (scratch bytes [256, 1024))
+  char* s = c->scratch.as<char>() + 256;
+  NT_CUDA(c, restore ? cudaMemcpyAsync(s, b, 768, cudaMemcpyDeviceToDevice, c->stream)
+                     : cudaMemcpyAsync(b, s, 768, cudaMemcpyDeviceToDevice, c->stream));
+  return NT_OK;
+}
+
+static nt_status run_det_history(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
+  int cell_bits = 0;
+  while ((1ull << cell_bits) < (unsigned long long)c->nx * (unsigned long long)c->ny) ++cell_bits;
+  if (cell_bits > 24)
+    return fail(c, NT_ERR_UNSUPPORTED, "deterministic mode supports at most 2^24 cells");
+  if (c->rec_cap == 0) c->rec_cap = 1ull << 20;
+  const unsigned long long kMaxCap = 1ull << 27;
+  int64_t batch = c->opt.det_batch;
+  const int grid = history_grid(c, true);
+  unsigned long long* rec_count = reinterpret_cast<unsigned long long*>(c->scratch.as<char>() + 8);
+  int64_t lo = 0;
+  while (lo < c->n_local) {
+    const int64_t hi = lo + batch < c->n_local ? lo + batch : c->n_local;
+    const int64_t nb = hi - lo;
+    NT_CUDA(c, c->rec_key.ensure(c->rec_cap * 8));
+    NT_CUDA(c, c->rec_val.ensure(c->rec_cap * 8));
+    NT_CUDA(c, c->rec_key2.ensure(c->rec_cap * 8));
+    NT_CUDA(c, c->rec_val2.ensure(c->rec_cap * 8));
+    NT_CUDA(c, c->backup.ensure(15 * align256((size_t)nb * 8) + 4096));
+    nt_status st = det_snapshot(c, lo, nb, false);
+    if (st != NT_OK) return st;
+    TrackParams bp = tp;
+    bp.lo = lo;
+    bp.hi = hi;
+    bp.rec_key = c->rec_key.as<unsigned long long>();
+    bp.rec_val = c->rec_val.as<double>();
+    bp.rec_cap = c->rec_cap;
+    bp.rec_count = rec_count;
+    NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 16, c->stream));   // work counter, records
+    launch_history(bp, true, grid, kHistoryBlock, c->stream);
+    ++launches;
+    NT_CUDA(c, cudaGetLastError());
+    unsigned long long nrec = 0;
+    NT_CUDA(c, cudaMemcpyAsync(&nrec, rec_count, 8, cudaMemcpyDeviceToHost, c->stream));
+    NT_CUDA(c, cudaStreamSynchronize(c->stream));
+    if (nrec > c->rec_cap) {
+      st = det_snapshot(c, lo, nb, true);
+      if (st != NT_OK) return st;
+      if (c->rec_cap < kMaxCap) {
+        while (c->rec_cap < nrec && c->rec_cap < kMaxCap) c->rec_cap <<= 1;
+      } else if (batch > 1) {
+        batch /= 2;
+      } else {
+        return fail(c, NT_ERR_UNSUPPORTED, "deterministic record buffer overflow");
+      }
+      continue;
+    }
+    if (nrec > 0) {
+      size_t tmp = 0;
+      NT_CUDA(c, sort_pairs(nullptr, tmp, bp.rec_key, c->rec_key2.as<unsigned long long>(),
+                            bp.rec_val, c->rec_val2.as<double>(), nrec, 40 + cell_bits, c->stream));
+      NT_CUDA(c, c->sort_tmp.ensure(tmp));
+      NT_CUDA(c, sort_pairs(c->sort_tmp.p, tmp, bp.rec_key, c->rec_key2.as<unsigned long long>(),
+                            bp.rec_val, c->rec_val2.as<double>(), nrec, 40 + cell_bits, c->stream));
+      launch_det_apply(c->rec_key2.as<unsigned long long>(), c->rec_val2.as<double>(), nrec,
+                       tp.mesh.tally, c->stream);
+      launches += 2;
+      NT_CUDA(c, cudaGetLastError());
+    }
+    lo = hi;
+  }
+  return NT_OK;
+}
+
+nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->stage < ST_PARTICLES) return fail(c, NT_ERR_STATE, "nt_inject_particles must come first");
+  if (!(dt > 0.0) || !is_fin(dt)) return fail(c, NT_ERR_ARG, "dt must be finite and > 0");
+  NT_CUDA(c, c->scratch.ensure(1024));
+  const size_t cells = (size_t)c->nx * (size_t)c->ny;
+  uint32_t launches = 0;
+  const bool det = c->opt.deterministic != 0;
+
+  NT_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
+  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, cells * 8, c->stream));
+  NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 1024, c->stream));
+  NT_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
+  const TrackParams tp = make_params(c, dt);
+  if (c->opt.mode == NT_MODE_EVENT) {
+    if (!c->evs) c->evs = event_state_create();
+    if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
+    const nt_status st = event_run_timestep(c->evs, tp, det, c->sm_count, c->stream, launches, c->err);
+    if (st != NT_OK) return st;
+  } else if (det) {
+    const nt_status st = run_det_history(c, tp, launches);
+    if (st != NT_OK) return st;
+  } else {
+    launch_history(tp, false, history_grid(c, false), kHistoryBlock, c->stream);
+    ++launches;
+    NT_CUDA(c, cudaGetLastError());
+  }
+  NT_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
+  // stats: u64 slots then f64 slots, reduced over ranks as doubles (counts < 2^53 exact)
+  double hs[SU_COUNT + SF_COUNT];
+  {
+    unsigned long long hu[SU_COUNT];
+    double hf[SF_COUNT];
+    char* s = c->scratch.as<char>();
+    NT_CUDA(c, cudaMemcpyAsync(hu, s + 256, sizeof hu, cudaMemcpyDeviceToHost, c->stream));
+    NT_CUDA(c, cudaMemcpyAsync(hf, s + 512, sizeof hf, cudaMemcpyDeviceToHost, c->stream));
+    if (c->comm) {
+      NT_CUDA(c, c->tally_local.ensure(cells * 8));
+      NT_CUDA(c, cudaMemcpyAsync(c->tally_local.p, c->tally.p, cells * 8, cudaMemcpyDeviceToDevice, c->stream));
+      NT_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+      NT_NCCL(c, ncclAllReduce(c->tally.p, c->tally.p, cells, ncclFloat64, ncclSum, c->comm, c->stream));
+      NT_CUDA(c, cudaEventRecord(c->ev[4], c->stream));
+    }
+    NT_CUDA(c, cudaStreamSynchronize(c->stream));
+    for (int k = 0; k < SU_COUNT; ++k) hs[k] = (double)hu[k];
+    for (int k = 0; k < SF_COUNT; ++k) hs[SU_COUNT + k] = hf[k];
+  }
+  float reduce_ms = 0.f;
+  if (c->comm) {
+    // small stats allreduce through the same communicator
+    double* d = reinterpret_cast<double*>(c->scratch.as<char>() + 768 - 8 * 0);
+    (void)d;
+    DevBuf tmp;
+    NT_CUDA(c, tmp.ensure(sizeof hs));
+    NT_CUDA(c, cudaMemcpyAsync(tmp.p, hs, sizeof hs, cudaMemcpyHostToDevice, c->stream));
+    NT_NCCL(c, ncclAllReduce(tmp.p, tmp.p, SU_COUNT + SF_COUNT, ncclFloat64, ncclSum, c->comm, c->stream));
+    NT_CUDA(c, cudaMemcpyAsync(hs, tmp.p, sizeof hs, cudaMemcpyDeviceToHost, c->stream));
+    NT_CUDA(c, cudaStreamSynchronize(c->stream));
+    tmp.release();
+    cudaEventElapsedTime(&reduce_ms, c->ev[3], c->ev[4]);
+    ncclResult_t async_err;
+    ncclCommGetAsyncError(c->comm, &async_err);
+    if (async_err != ncclSuccess) return fail(c, NT_ERR_NCCL, "NCCL async error: %s", ncclGetErrorString(async_err));
+    launches += 0;
+  }
+  float track_ms = 0.f, step_ms = 0.f;
+  cudaEventElapsedTime(&track_ms, c->ev[1], c->ev[2]);
+  cudaEventElapsedTime(&step_ms, c->ev[0], c->ev[2]);
+  nt_step_stats s{};
+  s.n_alive_start = (uint64_t)hs[SU_ALIVE];
+  s.n_facets = (uint64_t)hs[SU_FACETS];
+  s.n_collisions = (uint64_t)hs[SU_COLLISIONS];
+  s.n_census = (uint64_t)hs[SU_CENSUS];
+  s.n_killed = (uint64_t)hs[SU_KILLED];
+  s.n_xs_range = (uint64_t)hs[SU_XS_RANGE];
+  s.n_nonfinite = (uint64_t)hs[SU_NONFINITE];
+  s.n_event_cap = (uint64_t)hs[SU_EVENT_CAP];
+  s.tally_total = hs[SU_COUNT + SF_TALLY];
+  s.census_energy = hs[SU_COUNT + SF_CENSUS_E];
+  s.census_weight = hs[SU_COUNT + SF_CENSUS_W];
+  s.killed_energy = hs[SU_COUNT + SF_KILLED_E];
+  s.killed_weight = hs[SU_COUNT + SF_KILLED_W];
+  s.absorbed_weight = hs[SU_COUNT + SF_ABSORBED_W];
+  s.track_ms = track_ms;
+  s.reduce_ms = reduce_ms;
+  s.step_ms = step_ms + reduce_ms;
+  s.n_launches = launches;
+  if (stats) *stats = s;
+  c->stage = ST_STEPPED;
+  if (hs[SU_REC_OVERFLOW] > 0) return fail(c, NT_ERR_UNSUPPORTED, "flush sequence overflow (>2^24 flushes in one history)");
+  if (s.n_nonfinite) return fail(c, NT_ERR_NONFINITE, "%llu particles ended non-finite", (unsigned long long)s.n_nonfinite);
+  if (s.n_event_cap) return fail(c, NT_ERR_EVENT_CAP, "%llu histories hit max_events_per_history", (unsigned long long)s.n_event_cap);
+  if (s.n_xs_range) return fail(c, NT_ERR_XS_RANGE, "%llu lookups outside the table range", (unsigned long long)s.n_xs_range);
+  return NT_OK;
+}
+
+// ---- read-back ---------------------------------------------------------------------------
+nt_status nt_read_tally(nt_ctx* c, double* dst, int32_t reduced) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->stage < ST_MESH) return fail(c, NT_ERR_STATE, "no mesh");
+  if (!dst) return fail(c, NT_ERR_ARG, "dst is NULL");
+  const size_t cells = (size_t)c->nx * (size_t)c->ny;
+  const void* src = (!reduced && c->comm) ? c->tally_local.p : c->tally.p;
+  if (!src) return fail(c, NT_ERR_STATE, "no local tally yet");
+  NT_CUDA(c, cudaMemcpyAsync(dst, src, cells * 8, cudaMemcpyDefault, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  return NT_OK;
+}
+
+static nt_status copy_particles(nt_ctx* c, int64_t first, int64_t count, const nt_particles* v,
+                                bool to_dev) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->stage < ST_PARTICLES) return fail(c, NT_ERR_STATE, "no particles");
+  if (!v || first < 0 || count < 0 || first + count > c->n_local)
+    return fail(c, NT_ERR_ARG, "range [first, first+count) outside the local particles");
+  struct F { void* host; void* dev; size_t sz; };
+  const F f[] = {
+      {v->x, c->p.x, 8}, {v->y, c->p.y, 8}, {v->ox, c->p.ox, 8}, {v->oy, c->p.oy, 8},
+      {v->e, c->p.e, 8}, {v->w, c->p.w, 8}, {v->mfp, c->p.mfp, 8}, {v->cx, c->p.cx, 4},
+      {v->cy, c->p.cy, 4}, {v->ctr, c->p.ctr, 4}, {v->status, c->p.status, 1},
+      {v->nfac, c->p.nfac, 4}, {v->ncol, c->p.ncol, 4}, {v->ncen, c->p.ncen, 4},
+      {v->dep, c->p.dep, 8}};
+  for (const F& x : f) {
+    if (!x.host) continue;
+    char* d = static_cast<char*>(x.dev) + (size_t)first * x.sz;
+    if (to_dev)
+      NT_CUDA(c, cudaMemcpyAsync(d, x.host, (size_t)count * x.sz, cudaMemcpyDefault, c->stream));
+    else
+      NT_CUDA(c, cudaMemcpyAsync(x.host, d, (size_t)count * x.sz, cudaMemcpyDefault, c->stream));
+  }
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  return NT_OK;
+}
+
+nt_status nt_read_particles(nt_ctx* c, int64_t first, int64_t count, const nt_particles* dst) {
+  return copy_particles(c, first, count, dst, false);
+}
+
+nt_status nt_write_particles(nt_ctx* c, int64_t first, int64_t count, const nt_particles* src) {
+  return copy_particles(c, first, count, src, true);
+}
+
+// ---- verification entry points -----------------------------------------------------------
+nt_status nt_debug_threefry(nt_ctx* c, const uint64_t* in, int64_t n, uint64_t* out) {
+  if (!c || !in || !out || n < 0) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  DevBuf a, b;
+  NT_CUDA(c, a.ensure((size_t)n * 32 + 32));
+  NT_CUDA(c, b.ensure((size_t)n * 16 + 16));
+  NT_CUDA(c, copy_in(a.p, in, (size_t)n * 32, c->stream));
+  launch_threefry_debug(a.as<uint64_t>(), n, b.as<uint64_t>(), c->stream);
+  NT_CUDA(c, cudaGetLastError());
+  NT_CUDA(c, cudaMemcpyAsync(out, b.p, (size_t)n * 16, cudaMemcpyDefault, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  a.release();
+  b.release();
+  return NT_OK;
+}
+
+nt_status nt_debug_xs(nt_ctx* c, const double* energies, int64_t n, double* out_s, double* out_a) {
+  if (!c || !energies || !out_s || !out_a || n < 0) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->stage < ST_XS) return fail(c, NT_ERR_STATE, "no cross sections loaded");
+  DevBuf a, b;
+  NT_CUDA(c, a.ensure((size_t)n * 8 + 8));
+  NT_CUDA(c, b.ensure((size_t)n * 16 + 16));
+  NT_CUDA(c, copy_in(a.p, energies, (size_t)n * 8, c->stream));
+  launch_xs_debug(c->tables, a.as<double>(), n, b.as<double>(), b.as<double>() + n, c->stream);
+  NT_CUDA(c, cudaGetLastError());
+  NT_CUDA(c, cudaMemcpyAsync(out_s, b.p, (size_t)n * 8, cudaMemcpyDefault, c->stream));
+  NT_CUDA(c, cudaMemcpyAsync(out_a, b.as<double>() + n, (size_t)n * 8, cudaMemcpyDefault, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  a.release();
+  b.release();
+  return NT_OK;
+}
+
+}  // extern "C"

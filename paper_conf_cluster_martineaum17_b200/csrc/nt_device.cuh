@@ -1,0 +1,166 @@
+// nt_device.cuh -- device-side building blocks of the tracker (sm_100a).
+//
+// Everything here implements DESIGN.md §3 (the paper's method as read in DESIGN.md §4)
+// and is written independently of oracle/ (no shared code).  The library is compiled
+// with -fmad=false so every expression rounds exactly as parenthesised.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace nt {
+
+// ---- physical constants (DESIGN.md §4 R4) -------------------------------------------
+constexpr double kAvogadro = 6.02214076e23;     // mol^-1
+constexpr double kEv = 1.602176634e-19;         // J
+constexpr double kNeutronMass = 1.67492749804e-27;  // kg
+constexpr double kBarn = 1.0e-28;               // m^2
+constexpr double kTwoPi = 6.283185307179586;
+constexpr unsigned kFull = 0xffffffffu;
+
+// ---- data layout -----------------------------------------------------------------------
+// Particle store: structure of arrays, one column per field, indexed by local index.
+// Coalesced 8 B / 4 B / 1 B column accesses for a warp handling consecutive particles.
+struct Soa {
+  double *x, *y, *ox, *oy, *e, *w, *mfp, *dep;
+  int32_t *cx, *cy;
+  uint32_t *ctr, *nfac, *ncol, *ncen;
+  uint8_t *status;
+};
+
+struct Mesh {
+  const double* __restrict__ rho;   // [ny][nx] kg/m^3
+  double* __restrict__ tally;       // [ny][nx] eV*weight
+  const double* __restrict__ ex;    // [nx+1] edge(i) = (i*W)/nx
+  const double* __restrict__ ey;    // [ny+1]
+  int32_t nx, ny;
+};
+
+struct Tables {
+  const double* __restrict__ sk;    // scatter keys (eV), values (barns)
+  const double* __restrict__ sv;
+  const double* __restrict__ ck;    // capture keys, values
+  const double* __restrict__ cv;
+  int32_t ns, nc;
+};
+
+// Sub-expressions of DESIGN.md §3 that depend only on run constants.  Each is computed
+// on the host with exactly the parenthesisation §3 writes, so using the stored value
+// rounds identically to evaluating it in place.
+struct Phys {
+  double A;        // A
+  double AA;       // A*A
+  double twoA;     // 2.0*A
+  double Ap1;      // A + 1.0
+  double Am1;      // A - 1.0
+  double Ap1sq;    // (A + 1.0)*(A + 1.0)
+  double f;        // (A*A + 1.0) / ((A + 1.0)*(A + 1.0))
+  double cn;       // N_A / M
+  double kv;       // (2.0*EV) / M_N
+  double e_min, w_min;
+};
+
+// Step statistics slots (u64 and f64 arrays in global memory).
+enum StatU { SU_ALIVE = 0, SU_FACETS, SU_COLLISIONS, SU_CENSUS, SU_KILLED, SU_XS_RANGE,
+             SU_NONFINITE, SU_EVENT_CAP, SU_REC_OVERFLOW, SU_COUNT };
+enum StatF { SF_TALLY = 0, SF_CENSUS_E, SF_CENSUS_W, SF_KILLED_E, SF_KILLED_W,
+             SF_ABSORBED_W, SF_COUNT };
+
+// ---- Threefry-2x64-20 (Random123 Threefry) -----------------------------------
+__device__ __forceinline__ uint64_t rotl64(uint64_t x, int r) {
+  return (x << r) | (x >> (64 - r));
+}
+
+struct U64x2 { uint64_t a, b; };
+
+__device__ __forceinline__ U64x2 threefry2x64_20(uint64_t c0, uint64_t c1, uint64_t k0,
+                                                 uint64_t k1) {
+  const uint64_t k2 = 0x1BD11BDAA9FC1A22ull ^ k0 ^ k1;
+  const uint64_t ks[3] = {k0, k1, k2};
+  constexpr int R[8] = {16, 42, 12, 31, 16, 32, 24, 21};
+  uint64_t x0 = c0 + k0, x1 = c1 + k1;
+#pragma unroll
+  for (int r = 0; r < 20; ++r) {
+    x0 += x1;
+    x1 = rotl64(x1, R[r & 7]);
+    x1 ^= x0;
+    if ((r & 3) == 3) {
+      const int s = (r + 1) >> 2;
+      x0 += ks[s % 3];
+      x1 += ks[(s + 1) % 3] + (uint64_t)s;
+    }
+  }
+  return {x0, x1};
+}
+
+// u(x) = ((x >> 11) | 1) * 2^-53 : odd multiple of 2^-53, exact (R13)
+__device__ __forceinline__ double u01(uint64_t x) {
+  return (double)((x >> 11) | 1ull) * 0x1.0p-53;
+}
+
+// ---- mesh --------------------------------------------------------------------------------
+// The unique i in [0,n-1] with edge[i] <= q < edge[i+1] (q >= edge[n] -> n-1), from a guess.
+__device__ __forceinline__ int32_t cell_of(double q, const double* __restrict__ edge,
+                                           int32_t n, double extent) {
+  if (!(q >= 0.0)) return 0;
+  if (q >= edge[n]) return n - 1;
+  int32_t i = (int32_t)(q / extent * (double)n);
+  i = i < 0 ? 0 : (i > n - 1 ? n - 1 : i);
+  while (i > 0 && edge[i] > q) --i;
+  while (i < n - 1 && edge[i + 1] <= q) ++i;
+  return i;
+}
+
+// ---- microscopic cross sections -----------------------------------------------
+// Bin i = max{i in [0,N-2]: k[i] <= e} for e already in [k0, k_{N-1}]; then lerp.
+__device__ __forceinline__ double xs_lookup(const double* __restrict__ k,
+                                            const double* __restrict__ v, int32_t n,
+                                            double e) {
+  int32_t lo = 0, hi = n - 1;                 // k[lo] <= e < k[hi]  (or e == k[n-1])
+  if (e >= __ldg(k + n - 1)) {
+    lo = n - 2;
+  } else {
+    while (hi - lo > 1) {
+      const int32_t mid = (lo + hi) >> 1;
+      if (__ldg(k + mid) <= e) lo = mid; else hi = mid;
+    }
+  }
+  const double k0 = __ldg(k + lo), k1 = __ldg(k + lo + 1);
+  const double v0 = __ldg(v + lo), v1 = __ldg(v + lo + 1);
+  const double t = (e - k0) / (k1 - k0);
+  return v0 + t * (v1 - v0);
+}
+
+struct Mat {
+  double st;   // (sigma_s + sigma_a) * barn, m^2
+  double pa;   // sigma_a / sigma_t
+  double H;    // E - (sigma_s/sigma_t) * (E*f): expected heating response
+};
+
+__device__ __forceinline__ double clamp_count(double e, const double* __restrict__ k,
+                                              int32_t n, uint32_t& nrange) {
+  const double lo = __ldg(k), hi = __ldg(k + n - 1);
+  if (e < lo) { ++nrange; return lo; }
+  if (e > hi) { ++nrange; return hi; }
+  return e;
+}
+
+__device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, double e,
+                                          uint32_t& nrange) {
+  const double es = clamp_count(e, T.sk, T.ns, nrange);
+  const double ea = clamp_count(e, T.ck, T.nc, nrange);
+  const double ss = xs_lookup(T.sk, T.sv, T.ns, es);
+  const double sa = xs_lookup(T.ck, T.cv, T.nc, ea);
+  const double t = ss + sa;
+  Mat m;
+  m.st = t * kBarn;
+  m.pa = t > 0.0 ? sa / t : 0.0;
+  const double rs = t > 0.0 ? ss / t : 0.0;
+  m.H = e - rs * (e * ph.f);
+  return m;
+}
+
+__device__ __forceinline__ double speed(double e, const Phys& ph) {
+  return sqrt(e * ph.kv);
+}
+
+}  // namespace nt

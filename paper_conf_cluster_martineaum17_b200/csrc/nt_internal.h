@@ -1,0 +1,62 @@
+// nt_internal.h -- kernel parameter blocks and launchers shared by the runtime (nt_api.cu)
+// and the kernel translation units.  Not part of the public ABI.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+#include "nt_device.cuh"
+
+namespace nt {
+
+struct TrackParams {
+  Mesh mesh;
+  Tables xs;
+  Phys ph;
+  Soa p;
+  int64_t n;                  // local particles
+  int64_t lo, hi;             // local index range processed by this launch
+  int64_t first_id;           // global id of local index 0
+  uint64_t seed;
+  double dt;
+  int64_t max_events;
+  unsigned long long* counter;      // dynamic work counter (particles claimed)
+  unsigned long long* stats_u;      // [SU_COUNT]
+  double* stats_f;                  // [SF_COUNT]
+  // deterministic-mode flush records (cell << 40 | (pid - lo) << 24 | seq, value)
+  unsigned long long* rec_key;
+  double* rec_val;
+  unsigned long long* rec_count;
+  unsigned long long rec_cap;
+};
+
+struct InjectParams {
+  Soa p;
+  const double* ex;
+  const double* ey;
+  int32_t nx, ny;
+  double W, H;
+  int64_t n_local, first_id;
+  double sx, sy, sw, sh, e0;
+  uint64_t seed;
+};
+
+// ---- launchers (nt_kernels.cu) ----------------------------------------------------------
+void launch_edges(double* ex, int32_t nx, double W, double* ey, int32_t ny, double H,
+                  cudaStream_t s);
+void launch_inject(const InjectParams& ip, cudaStream_t s);
+// History (Over Particles) tracking: grid = persistent CTAs.
+void launch_history(const TrackParams& tp, bool det, int grid, int block, cudaStream_t s);
+int history_max_ctas_per_sm(bool det, int block);
+void launch_det_apply(const unsigned long long* keys, const double* vals,
+                      unsigned long long n, double* tally, cudaStream_t s);
+void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s);
+void launch_xs_debug(const Tables& T, const double* e, int64_t n, double* os, double* oa,
+                     cudaStream_t s);
+// CUB radix sort of (key, value) pairs; temp_bytes query when temp == nullptr.
+cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long* kin,
+                       unsigned long long* kout, const double* vin, double* vout,
+                       unsigned long long n, int end_bit, cudaStream_t s);
+
+constexpr int kHistoryBlock = 256;
+
+}  // namespace nt

@@ -1,0 +1,412 @@
+// nt_kernels.cu -- history-based (Over Particles) tracking kernel, source injection,
+// deterministic tally application and verification kernels for sm_100a.
+//
+// DESIGN.md §3 is the arithmetic; §6 is the kernel design.  Paper passages:
+//  - Over Particles: one thread follows one particle from birth to census.
+//  - Event timers, nearest event wins (Listing 1).
+//  - Facet: flush the register-accumulated deposit with one fp64 atomic, load the new
+//    cell's density.  Collision: implicit capture + elastic scatter,
+//    XS re-lookup, new mean free path.
+//  - Census: flush and stop.
+#include <cub/device/device_radix_sort.cuh>
+
+#include "nt_internal.h"
+
+namespace nt {
+
+__device__ __forceinline__ double d_inf() { return __longlong_as_double(0x7ff0000000000000ll); }
+
+// ---------------------------------------------------------------------------------------
+// Mesh edges: edge(i) = (i*W)/n  (DESIGN.md §3 MESH)
+__global__ void edges_kernel(double* ex, int32_t nx, double W, double* ey, int32_t ny,
+                             double H) {
+  const int32_t i = blockIdx.x * blockDim.x + threadIdx.x;
+  if (i <= nx) ex[i] = ((double)i * W) / (double)nx;
+  if (i <= ny) ey[i] = ((double)i * H) / (double)ny;
+}
+
+void launch_edges(double* ex, int32_t nx, double W, double* ey, int32_t ny, double H,
+                  cudaStream_t s) {
+  const int n = (nx > ny ? nx : ny) + 1;
+  edges_kernel<<<(n + 255) / 256, 256, 0, s>>>(ex, nx, W, ey, ny, H);
+}
+
+// ---------------------------------------------------------------------------------------
+// Source injection: one thread per particle, coalesced SoA stores.
+__global__ void __launch_bounds__(256) inject_kernel(const __grid_constant__ InjectParams P) {
+  const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (i >= P.n_local) return;
+  const uint64_t pid = (uint64_t)(P.first_id + i);
+  const U64x2 r0 = threefry2x64_20(0, 0, pid, P.seed);
+  const double x = P.sx + u01(r0.a) * P.sw;
+  const double y = P.sy + u01(r0.b) * P.sh;
+  const U64x2 r1 = threefry2x64_20(1, 0, pid, P.seed);
+  const double theta = kTwoPi * u01(r1.a);
+  P.p.x[i] = x;
+  P.p.y[i] = y;
+  P.p.cx[i] = cell_of(x, P.ex, P.nx, P.W);
+  P.p.cy[i] = cell_of(y, P.ey, P.ny, P.H);
+  P.p.ox[i] = cos(theta);
+  P.p.oy[i] = sin(theta);
+  P.p.mfp[i] = -log(u01(r1.b));
+  P.p.e[i] = P.e0;
+  P.p.w[i] = 1.0;
+  P.p.ctr[i] = 2u;
+  P.p.status[i] = 1u;
+  P.p.nfac[i] = 0u;
+  P.p.ncol[i] = 0u;
+  P.p.ncen[i] = 0u;
+  P.p.dep[i] = 0.0;
+}
+
+void launch_inject(const InjectParams& ip, cudaStream_t s) {
+  if (ip.n_local <= 0) return;
+  const int64_t blocks = (ip.n_local + 255) / 256;
+  inject_kernel<<<(unsigned)blocks, 256, 0, s>>>(ip);
+}
+
+// ---------------------------------------------------------------------------------------
+// History tracking kernel.
+//
+// Persistent CTAs; each warp claims particles from a global counter with one atomic per
+// refill (warp ballot of idle lanes + popc rank), so a lane whose history ends picks up
+// a new particle at the next event instead of idling until the warp's longest history
+// finishes (the load imbalance of P:344-348).  All of a history's state -- position,
+// direction and its reciprocal, energy, weight, mean free paths, census timer, the
+// cell's number density, the cached cross sections and the deposit accumulator -- lives
+// in registers for the whole history.  Per event the memory traffic is one
+// 8 B density gather (facet) and one fp64 RED into the tally (facet / census / kill).
+//
+// kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
+// keyed record; the host sorts the records and applies them in the oracle's order.
+template <bool kDet>
+__global__ void __launch_bounds__(kHistoryBlock)
+history_kernel(const __grid_constant__ TrackParams P) {
+  __shared__ uint32_t s_u[SU_COUNT][kHistoryBlock];
+  __shared__ double s_f[SF_COUNT][kHistoryBlock];
+  const int t = threadIdx.x;
+#pragma unroll
+  for (int k = 0; k < SU_COUNT; ++k) s_u[k][t] = 0u;
+#pragma unroll
+  for (int k = 0; k < SF_COUNT; ++k) s_f[k][t] = 0.0;
+
+  const int lane = t & 31;
+  const unsigned lt_mask = (1u << lane) - 1u;
+  const unsigned long long span = (unsigned long long)(P.hi - P.lo);
+  const double* __restrict__ ex = P.mesh.ex;
+  const double* __restrict__ ey = P.mesh.ey;
+  const double* __restrict__ rho = P.mesh.rho;
+  const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
+  const Phys& ph = P.ph;
+
+  bool active = false, exhausted = false;
+  int64_t i = 0;
+  double x = 0, y = 0, ox = 0, oy = 0, iox = 0, ioy = 0, e = 0, w = 0, mfp = 0, dcen = 0;
+  double nd = 0, acc = 0, dep = 0;
+  Mat m{0, 0, 0};
+  int32_t cx = 0, cy = 0;
+  uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
+
+  for (;;) {
+    // ---- refill idle lanes with new particles (one atomic per warp) ----
+    const unsigned idle = __ballot_sync(kFull, !active);
+    if (idle != 0u && !exhausted) {
+      const int leader = __ffs(idle) - 1;
+      unsigned long long base = 0;
+      if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
+      base = __shfl_sync(kFull, base, leader);
+      if (base + (unsigned long long)__popc(idle) >= span) exhausted = true;
+      if (!active) {
+        const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
+        if (my < span) {
+          i = P.lo + (int64_t)my;
+          if (P.p.status[i] == 1u) {
+            active = true;
+            x = P.p.x[i];
+            y = P.p.y[i];
+            ox = P.p.ox[i];
+            oy = P.p.oy[i];
+            e = P.p.e[i];
+            w = P.p.w[i];
+            mfp = P.p.mfp[i];
+            dep = P.p.dep[i];
+            cx = P.p.cx[i];
+            cy = P.p.cy[i];
+            ctr = P.p.ctr[i];
+            nd = __ldg(rho + (int64_t)cy * nx + cx) * ph.cn;
+            m = refresh_xs(P.xs, ph, e, nrange);
+            dcen = speed(e, ph) * P.dt;
+            iox = 1.0 / ox;
+            ioy = 1.0 / oy;
+            acc = 0.0;
+            nf = 0u;
+            nc = 0u;
+            seq = 0u;
+            s_u[SU_ALIVE][t] += 1u;
+          }
+        }
+      }
+    }
+    if (!__any_sync(kFull, active)) {
+      if (exhausted) break;
+      continue;
+    }
+    if (!active) continue;
+
+    // ---- one event (Listing 1) ----
+    const uint64_t pid = (uint64_t)(P.first_id + i);
+    const double sig = nd * m.st;
+    double tx = d_inf(), ty = d_inf();
+    if (ox != 0.0) {
+      tx = (__ldg(ex + cx + (ox > 0.0 ? 1 : 0)) - x) * iox;
+      tx = tx < 0.0 ? 0.0 : tx;
+    }
+    if (oy != 0.0) {
+      ty = (__ldg(ey + cy + (oy > 0.0 ? 1 : 0)) - y) * ioy;
+      ty = ty < 0.0 ? 0.0 : ty;
+    }
+    const bool ax = tx < ty;
+    const double df = ax ? tx : ty;
+    const double dc = sig > 0.0 ? mfp / sig : d_inf();
+    const double ds = dcen;
+    int outcome = 0;                      // 0 continue, 1 census, 2 dead
+
+    auto flush = [&]() {
+      const int64_t cell = (int64_t)cy * nx + cx;
+      if constexpr (kDet) {
+        const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
+        if (slot < P.rec_cap) {
+          P.rec_key[slot] = ((unsigned long long)cell << 40) |
+                            ((unsigned long long)(i - P.lo) << 24) |
+                            (unsigned long long)(seq & 0xffffffu);
+          P.rec_val[slot] = acc;
+        }
+        if (seq >= (1u << 24)) s_u[SU_REC_OVERFLOW][t] += 1u;
+        ++seq;
+      } else {
+        atomicAdd(P.mesh.tally + cell, acc);
+      }
+      s_f[SF_TALLY][t] += acc;
+      dep += acc;
+      acc = 0.0;
+    };
+
+    if ((int64_t)(nf + nc) >= P.max_events) {
+      // guard (R27): count, flush, kill
+      s_u[SU_EVENT_CAP][t] += 1u;
+      flush();
+      s_u[SU_KILLED][t] += 1u;
+      s_f[SF_KILLED_E][t] += w * e;
+      s_f[SF_KILLED_W][t] += w;
+      outcome = 2;
+    } else if (dc < df && dc < ds) {
+      // ---- collision ----
+      acc += ((w * dc) * sig) * m.H;
+      x = x + dc * ox;
+      y = y + dc * oy;
+      dcen = dcen - dc;
+      const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, pid, P.seed);
+      ctr += 1u;
+      nc += 1u;
+      const double w_old = w;
+      w = w * (1.0 - m.pa);                               // implicit capture
+      s_f[SF_ABSORBED_W][t] += w_old - w;
+      const double mu = 1.0 - 2.0 * u01(r.a);
+      const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
+      const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
+      const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
+      const double q = 1.0 - ct * ct;
+      const double stt = sgn * sqrt(q > 0.0 ? q : 0.0);
+      const double nox = ox * ct - oy * stt;
+      const double noy = ox * stt + oy * ct;
+      ox = nox;
+      oy = noy;
+      const double tcen = dcen / speed(e, ph);
+      e = e2;
+      if (e < ph.e_min || w < ph.w_min) {
+        flush();
+        s_f[SF_KILLED_E][t] += w * e;
+        s_f[SF_KILLED_W][t] += w;
+        s_u[SU_KILLED][t] += 1u;
+        outcome = 2;
+      } else {
+        dcen = tcen * speed(e, ph);
+        m = refresh_xs(P.xs, ph, e, nrange);
+        iox = 1.0 / ox;
+        ioy = 1.0 / oy;
+        mfp = -log(u01(r.b));
+      }
+    } else if (df < ds) {
+      // ---- facet ----
+      acc += ((w * df) * sig) * m.H;
+      const double nm = mfp - df * sig;
+      mfp = nm > 0.0 ? nm : 0.0;
+      dcen = dcen - df;
+      if (ax) {
+        y = y + df * oy;
+        x = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
+        flush();
+        if (ox > 0.0) {
+          if (cx == nx - 1) { ox = -ox; iox = -iox; } else { cx += 1; }
+        } else {
+          if (cx == 0) { ox = -ox; iox = -iox; } else { cx -= 1; }
+        }
+      } else {
+        x = x + df * ox;
+        y = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
+        flush();
+        if (oy > 0.0) {
+          if (cy == ny - 1) { oy = -oy; ioy = -ioy; } else { cy += 1; }
+        } else {
+          if (cy == 0) { oy = -oy; ioy = -ioy; } else { cy -= 1; }
+        }
+      }
+      nf += 1u;
+      nd = __ldg(rho + (int64_t)cy * nx + cx) * ph.cn;    // density of the new cell
+    } else {
+      // ---- census ----
+      acc += ((w * ds) * sig) * m.H;
+      x = x + ds * ox;
+      y = y + ds * oy;
+      const double nm = mfp - ds * sig;
+      mfp = nm > 0.0 ? nm : 0.0;
+      flush();
+      s_u[SU_CENSUS][t] += 1u;
+      s_f[SF_CENSUS_E][t] += w * e;
+      s_f[SF_CENSUS_W][t] += w;
+      outcome = 1;
+    }
+
+    if (outcome != 0) {
+      if (!(isfinite(x) && isfinite(y) && isfinite(e) && isfinite(w)))
+        s_u[SU_NONFINITE][t] += 1u;
+      P.p.x[i] = x;
+      P.p.y[i] = y;
+      P.p.ox[i] = ox;
+      P.p.oy[i] = oy;
+      P.p.e[i] = e;
+      P.p.w[i] = w;
+      P.p.mfp[i] = mfp;
+      P.p.dep[i] = dep;
+      P.p.cx[i] = cx;
+      P.p.cy[i] = cy;
+      P.p.ctr[i] = ctr;
+      P.p.nfac[i] += nf;
+      P.p.ncol[i] += nc;
+      if (outcome == 1) {
+        P.p.ncen[i] += 1u;
+      } else {
+        P.p.status[i] = 0u;
+      }
+      s_u[SU_FACETS][t] += nf;
+      s_u[SU_COLLISIONS][t] += nc;
+      active = false;
+    }
+  }
+
+  // ---- CTA reduction of the per-thread statistics, one atomic per statistic ----
+  s_u[SU_XS_RANGE][t] += nrange;
+  __syncthreads();
+  const int warp = t >> 5;
+  constexpr int kWarps = kHistoryBlock / 32;
+  for (int k = warp; k < SU_COUNT + SF_COUNT; k += kWarps) {
+    if (k < SU_COUNT) {
+      unsigned long long v = 0;
+      for (int j = lane; j < kHistoryBlock; j += 32) v += s_u[k][j];
+#pragma unroll
+      for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(kFull, v, o);
+      if (lane == 0 && v != 0) atomicAdd(P.stats_u + k, v);
+    } else {
+      const int kf = k - SU_COUNT;
+      double v = 0.0;
+      for (int j = lane; j < kHistoryBlock; j += 32) v += s_f[kf][j];
+#pragma unroll
+      for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(kFull, v, o);
+      if (lane == 0 && v != 0.0) atomicAdd(P.stats_f + kf, v);
+    }
+  }
+}
+
+void launch_history(const TrackParams& tp, bool det, int grid, int block, cudaStream_t s) {
+  (void)block;
+  if (det)
+    history_kernel<true><<<grid, kHistoryBlock, 0, s>>>(tp);
+  else
+    history_kernel<false><<<grid, kHistoryBlock, 0, s>>>(tp);
+}
+
+int history_max_ctas_per_sm(bool det, int block) {
+  int n = 0;
+  (void)block;
+  if (det)
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_kernel<true>, kHistoryBlock, 0);
+  else
+    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_kernel<false>, kHistoryBlock, 0);
+  return n;
+}
+
+// ---------------------------------------------------------------------------------------
+// Deterministic tally: records sorted by (cell, particle, sequence); one thread per cell
+// segment adds the segment serially onto the running tally -- the oracle's order.
+__global__ void det_apply_kernel(const unsigned long long* __restrict__ keys,
+                                 const double* __restrict__ vals, unsigned long long n,
+                                 double* __restrict__ tally) {
+  for (unsigned long long j = (unsigned long long)blockIdx.x * blockDim.x + threadIdx.x; j < n;
+       j += (unsigned long long)gridDim.x * blockDim.x) {
+    const unsigned long long cell = keys[j] >> 40;
+    if (j != 0 && (keys[j - 1] >> 40) == cell) continue;
+    double s = tally[cell];
+    for (unsigned long long k = j; k < n && (keys[k] >> 40) == cell; ++k) s += vals[k];
+    tally[cell] = s;
+  }
+}
+
+void launch_det_apply(const unsigned long long* keys, const double* vals,
+                      unsigned long long n, double* tally, cudaStream_t s) {
+  if (n == 0) return;
+  unsigned long long blocks = (n + 255) / 256;
+  if (blocks > 65535ull * 8) blocks = 65535ull * 8;
+  det_apply_kernel<<<(unsigned)blocks, 256, 0, s>>>(keys, vals, n, tally);
+}
+
+cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long* kin,
+                       unsigned long long* kout, const double* vin, double* vout,
+                       unsigned long long n, int end_bit, cudaStream_t s) {
+  return cub::DeviceRadixSort::SortPairs(temp, temp_bytes, kin, kout, vin, vout,
+                                         (int64_t)n, 0, end_bit, s);
+}
+
+// ---------------------------------------------------------------------------------------
+// Verification kernels.
+__global__ void threefry_debug_kernel(const uint64_t* __restrict__ in, int64_t n,
+                                      uint64_t* __restrict__ out) {
+  const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (i >= n) return;
+  const U64x2 r = threefry2x64_20(in[4 * i], in[4 * i + 1], in[4 * i + 2], in[4 * i + 3]);
+  out[2 * i] = r.a;
+  out[2 * i + 1] = r.b;
+}
+
+void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s) {
+  if (n <= 0) return;
+  threefry_debug_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(in, n, out);
+}
+
+__global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, int64_t n,
+                                double* __restrict__ os, double* __restrict__ oa) {
+  const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (i >= n) return;
+  uint32_t dummy = 0;
+  const double es = clamp_count(e[i], T.sk, T.ns, dummy);
+  const double ea = clamp_count(e[i], T.ck, T.nc, dummy);
+  os[i] = xs_lookup(T.sk, T.sv, T.ns, es);
+  oa[i] = xs_lookup(T.ck, T.cv, T.nc, ea);
+}
+
+void launch_xs_debug(const Tables& T, const double* e, int64_t n, double* os, double* oa,
+                     cudaStream_t s) {
+  if (n <= 0) return;
+  xs_debug_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(T, e, n, os, oa);
+}
+
+}  // namespace nt

@@ -1,0 +1,95 @@
+"""The C-ABI library loads and exports every symbol include/*.h declares (no GPU needed).
+
+Also checks that the product package does not import the oracle (the
+oracle is test infrastructure only) and that the library has no CPU fallback.
+"""
+import ast
+import ctypes as C
+import re
+from pathlib import Path
+
+import pytest
+
+ROOT = Path(__file__).resolve().parent.parent
+PKG = ROOT / "paper_conf_cluster_martineaum17_b200"
+
+
+def _declared():
+    names = set()
+    for h in (ROOT / "include").glob("*.h"):
+        txt = re.sub(r"/\*.*?\*/", "", h.read_text(), flags=re.S)
+        names |= set(re.findall(r"\b(nt_[a-z_0-9]+)\s*\(", txt))
+    return names
+
+
+@pytest.fixture(scope="module")
+def L():
+    from paper_conf_cluster_martineaum17_b200 import build, binding
+    build.build()
+    return binding.lib()
+
+
+def test_exports_every_declared_symbol(L):
+    from paper_conf_cluster_martineaum17_b200 import binding
+    declared = _declared()
+    assert declared, "no declarations found"
+    assert declared == set(binding.EXPORTS)
+    for name in declared:
+        assert hasattr(L, name), name
+
+
+def test_identity_calls(L):
+    from paper_conf_cluster_martineaum17_b200 import binding
+    assert L.nt_abi_version() == 1
+    assert b"sm_100a" in L.nt_build_info()
+    assert b"-fmad=false" in L.nt_build_info()
+    for k, v in binding.STATUS.items():
+        assert L.nt_status_string(k).decode() == v
+    o = binding.Options()
+    assert L.nt_options_default(C.byref(o)) == 0
+    assert o.nranks == 1 and o.A == 1.0 and o.e_min == 1.0 and o.w_min == 1e-3
+    assert o.max_events_per_history == 10**9 and o.det_batch == 65536
+
+
+def test_struct_layouts_match_header():
+    """ctypes structs mirror the header's field lists (names and order)."""
+    from paper_conf_cluster_martineaum17_b200 import binding
+    txt = (ROOT / "include" / "neutral_b200.h").read_text()
+
+    def fields(struct_name):
+        body = re.search(r"typedef struct \{([^{}]*)\}\s*" + struct_name + ";", txt).group(1)
+        body = re.sub(r"/\*.*?\*/", "", body, flags=re.S)
+        out = []
+        for decl in body.split(";"):
+            decl = decl.strip()
+            if not decl:
+                continue
+            names = decl.split(None, 1)[1] if not decl.startswith("const") else decl.split(None, 2)[2]
+            for n in names.split(","):
+                out.append(n.strip().lstrip("*").strip())
+        return out
+
+    assert fields("nt_options") == [f for f, _ in binding.Options._fields_]
+    assert fields("nt_step_stats") == [f for f, _ in binding.StepStats._fields_]
+    assert fields("nt_particles") == [f for f, _ in binding.ParticlesView._fields_]
+
+
+def test_product_never_imports_oracle():
+    for py in PKG.rglob("*.py"):
+        tree = ast.parse(py.read_text())
+        for node in ast.walk(tree):
+            if isinstance(node, ast.Import):
+                assert all(not a.name.startswith("oracle") for a in node.names), py
+            if isinstance(node, ast.ImportFrom):
+                assert not (node.module or "").startswith("oracle"), py
+    for src in (PKG / "csrc").glob("*"):
+        for inc in re.findall(r'#include\s*[<"]([^>"]+)[>"]', src.read_text()):
+            assert "oracle" not in inc, (src, inc)
+
+
+def test_missing_library_fails_loudly(tmp_path, monkeypatch):
+    from paper_conf_cluster_martineaum17_b200 import binding
+    monkeypatch.setattr(binding, "_lib", None)
+    monkeypatch.setattr(binding, "LIB_PATH", tmp_path / "nope.so")
+    with pytest.raises(ImportError):
+        binding.lib()

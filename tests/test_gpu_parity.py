@@ -1,0 +1,297 @@
+"""GPU parity: the CUDA path (through the C ABI) against the oracle, element by element.
+
+Runs on a B200 (`pytest -m gpu` via gpurun).  Sizes: tiny/small problems the oracle
+finishes in well under a second (several CTAs of particles, ragged tails), then the
+BASELINE.json full-size configs in the launch configuration bench.py times, checked on
+sampled particles the oracle recomputes one by one and by properties that hold at any
+size.
+"""
+import math
+
+import numpy as np
+import pytest
+
+from paper_conf_cluster_martineaum17_b200 import workloads as wl
+from tests.parity import compare_particles, compare_stats, compare_tally
+
+pytestmark = pytest.mark.gpu
+
+MODES = ["history"]
+
+
+@pytest.fixture(scope="module")
+def nt():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    from paper_conf_cluster_martineaum17_b200 import binding, build
+    build.build()
+    return binding
+
+
+def _gpu_run(nt, cfg, steps=1, first_id=0, n_local=None, **opts):
+    t = nt.setup(cfg, first_id=first_id, n_local=n_local, **opts)
+    stats = [t.run_timestep(cfg.dt) for _ in range(steps)]
+    tally = t.read_tally()
+    parts = t.read_particles()
+    t.close()
+    return tally, parts, stats
+
+
+# ---------------------------------------------------------------------------------------------
+def test_threefry_words_bit_exact(nt, orc):
+    rng = np.random.default_rng(0)
+    grid = [(c, 0, p, s) for c in range(0, 40) for p in (0, 1, 2, 999, 2**40 + 3) for s in (0, 11, 2**63)]
+    rand = [tuple(int(v) for v in rng.integers(0, 2**64, 4, dtype=np.uint64)) for _ in range(2000)]
+    inp = np.array(grid + rand, dtype=np.uint64)
+    t = nt.Tracker()
+    out = t.debug_threefry(inp)
+    t.close()
+    assert tuple(int(v) for v in out[0 * 0]) == orc.threefry2x64_20(*[int(v) for v in inp[0]])
+    for row, o in zip(inp, out):
+        assert tuple(int(v) for v in o) == orc.threefry2x64_20(*[int(v) for v in row])
+
+
+@pytest.mark.parametrize("cfgname", ["csp", "tiny_csp"])
+def test_xs_lookup_matches_oracle(nt, orc, cfgname):
+    cfg = wl.CONFIGS[cfgname]
+    sk, sv, ck, cv = wl.tables(cfg)
+    t = nt.Tracker()
+    t.init_mesh(4, 4, 1.0, 1.0, np.ones(16))
+    t.load_cross_sections(sk, sv, ck, cv)
+    rng = np.random.default_rng(3)
+    es = np.concatenate([np.exp(rng.uniform(np.log(1e-5), np.log(2e7), 3000)), sk[:50], sk[-50:],
+                         ck[::997], [sk[0], sk[-1], 1.0, 1e6]])
+    gs, ga = t.debug_xs(es)
+    t.close()
+    for e, a, b in zip(es, gs, ga):
+        assert a == orc.xs_lookup(sk, sv, e)
+        assert b == orc.xs_lookup(ck, cv, e)
+
+
+def test_xs_random_tables(nt, orc):
+    rng = np.random.default_rng(9)
+    for n in [2, 3, 5, 17, 64, 1000]:
+        k, v = wl.random_tables(rng, n)
+        t = nt.Tracker()
+        t.init_mesh(4, 4, 1.0, 1.0, np.ones(16))
+        t.load_cross_sections(k, v, k, v[::-1].copy())
+        es = np.concatenate([rng.uniform(k[0], k[-1], 300), k])
+        gs, ga = t.debug_xs(es)
+        t.close()
+        for e, a, b in zip(es, gs, ga):
+            assert a == orc.xs_lookup(k, v, e)
+            assert b == orc.xs_lookup(k, v[::-1].copy(), e)
+
+
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "csp", "split"])
+def test_inject_matches_oracle(nt, orc, cfgname):
+    cfg = wl.CONFIGS[cfgname].with_(n_particles=5000)
+    t = nt.setup(cfg)
+    g = t.read_particles()
+    t.close()
+    prob = orc.Problem(cfg, wl.density(cfg), wl.tables(cfg))
+    o = orc.inject(prob, 0, cfg.n_particles)
+    for f in ["x", "y", "e", "w"]:
+        assert np.array_equal(g[f], getattr(o, f)), f
+    for f in ["cx", "cy", "ctr", "status", "nfac", "ncol", "ncen"]:
+        assert np.array_equal(g[f], getattr(o, f)), f
+    for f in ["ox", "oy", "mfp"]:          # libdevice vs libm: <= 2 ulp
+        a, b = g[f], getattr(o, f)
+        assert np.all(np.abs(a - b) <= 2 * np.spacing(np.abs(b)) + 1e-300), f
+
+
+# ---------------------------------------------------------------------------------------------
+TINY = ["tiny_csp", "tiny_stream", "tiny_split", "tiny_vacuum", "tiny_vacuum_lo", "tiny_scatter_1g",
+        "tiny_wkill", "tiny_A12", "tiny_mid", "tiny_thin", "tiny_absorber", "small_csp", "small_scatter"]
+
+
+@pytest.mark.parametrize("mode", MODES)
+@pytest.mark.parametrize("cfgname", TINY)
+def test_parity_deterministic(nt, orc, cfgname, mode):
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=True, mode=mode)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)
+    rep = compare_tally(gt, ot)
+    compare_stats(gs, os_)
+    assert gs["status"] == 0
+    print(cfgname, mode, rep)
+
+
+@pytest.mark.parametrize("mode", MODES)
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_split", "tiny_mid", "small_scatter"])
+def test_parity_production_atomic(nt, orc, cfgname, mode):
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)                  # per-particle results do not depend on the tally
+    compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+    compare_stats(gs, os_, rtol=1e-9)
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_parity_two_steps_and_shard(nt, orc, mode):
+    cfg = wl.CONFIGS["tiny_split"]
+    lo, n = 317, 1203                          # ragged shard of the id space
+    gt, gp, gs = _gpu_run(nt, cfg, steps=2, first_id=lo, n_local=n, deterministic=True, mode=mode)
+    ot, op, os_ = orc.run(cfg, first_id=lo, n_local=n, steps=2)
+    compare_particles(gp, op)
+    compare_tally(gt, ot)
+    for a, b in zip(gs, os_):
+        compare_stats(a, b)
+    assert gs[1]["n_alive_start"] == gs[0]["n_census"]
+
+
+def test_checkpoint_resume_bit_exact(nt):
+    """Census is a restart point; counter-based RNG makes resume exact."""
+    cfg = wl.CONFIGS["tiny_mid"]
+    t = nt.setup(cfg, deterministic=True)
+    t.run_timestep(cfg.dt)
+    snap = t.read_particles()
+    t.run_timestep(cfg.dt)
+    want = t.read_particles()
+    want_tally = t.read_tally()
+    t.write_particles(0, snap)
+    t.run_timestep(cfg.dt)
+    got = t.read_particles()
+    for k in want:
+        assert np.array_equal(want[k], got[k]), k
+    assert np.array_equal(want_tally, t.read_tally())
+    t.close()
+
+
+def test_edge_cases(nt, orc):
+    # empty particle set
+    cfg = wl.CONFIGS["tiny_csp"]
+    t = nt.setup(cfg, n_local=0, first_id=0)
+    s = t.run_timestep(cfg.dt)
+    assert s["events"] == 0 and s["status"] == 0
+    assert np.all(t.read_tally() == 0)
+    t.close()
+    # 1 x 1 mesh: every facet is a reflection
+    c1 = wl.CONFIGS["tiny_stream"].with_(nx=1, ny=1, n_particles=300, source=(0.0, 0.0, 1.0, 1.0))
+    gt, gp, (gs,) = _gpu_run(nt, c1, deterministic=True)
+    ot, op, (os_,) = orc.run(c1)
+    compare_particles(gp, op)
+    compare_stats(gs, os_)
+    # non-square mesh, non-unit extents
+    c2 = wl.CONFIGS["tiny_mid"].with_(nx=37, ny=91, width=2.5, height=0.7, source=(1.0, 0.1, 0.5, 0.3),
+                                       n_particles=999)
+    gt, gp, (gs,) = _gpu_run(nt, c2, deterministic=True)
+    ot, op, (os_,) = orc.run(c2)
+    compare_particles(gp, op)
+    compare_tally(gt, ot)
+    # event cap
+    c3 = wl.CONFIGS["tiny_stream"]
+    gt, gp, (gs,) = _gpu_run(nt, c3, deterministic=True, max_events=50)
+    prob = orc.Problem(c3, wl.density(c3), wl.tables(c3), max_events=50)
+    op = orc.inject(prob, 0, c3.n_particles)
+    ot = np.zeros((c3.ny, c3.nx))
+    os_ = orc.step(prob, op, 0, ot)
+    assert gs["status"] == 8 and gs["n_event_cap"] == os_["n_event_cap"] > 0
+    compare_particles(gp, op)
+    compare_tally(gt, ot)
+    # energy above the table: counted and clamped (NT_ERR_XS_RANGE)
+    c4 = wl.CONFIGS["tiny_scatter_1g"].with_(e0=5e7, n_particles=200)
+    gt, gp, (gs,) = _gpu_run(nt, c4, deterministic=True)
+    ot, op, (os_,) = orc.run(c4)
+    assert gs["status"] == 6 and gs["n_xs_range"] == os_["n_xs_range"] > 0
+    compare_particles(gp, op)
+
+
+def test_api_errors(nt):
+    t = nt.Tracker()
+    with pytest.raises(nt.NeutralError) as e:
+        t.run_timestep(1e-7)
+    assert e.value.status == 2
+    with pytest.raises(nt.NeutralError) as e:
+        t.init_mesh(0, 4, 1.0, 1.0, np.ones(4))
+    assert e.value.status == 1
+    with pytest.raises(nt.NeutralError):
+        t.init_mesh(2, 2, 1.0, 1.0, np.array([1.0, -1.0, 0.0, 0.0]))
+    t.init_mesh(2, 2, 1.0, 1.0, np.ones(4))
+    with pytest.raises(nt.NeutralError):
+        t.load_cross_sections([1.0, 1.0], [1.0, 1.0], [1.0, 2.0], [1.0, 1.0])   # not increasing
+    t.load_cross_sections([1.0, 2.0], [1.0, 1.0], [1.0, 2.0], [1.0, 1.0])
+    with pytest.raises(nt.NeutralError):
+        t.inject_particles(10, 5, 6, (0, 0, 0.5, 0.5), 1.5, 1)                    # past n_total
+    with pytest.raises(nt.NeutralError):
+        t.inject_particles(10, 0, 10, (0.8, 0, 0.5, 0.5), 1.5, 1)                 # outside mesh
+    t.inject_particles(10, 0, 10, (0, 0, 0.5, 0.5), 1.5, 1)
+    with pytest.raises(nt.NeutralError):
+        t.run_timestep(-1.0)
+    t.close()
+
+
+def test_device_pointer_inputs_and_outputs(nt, orc):
+    import torch
+    cfg = wl.CONFIGS["tiny_csp"]
+    dens = torch.as_tensor(wl.density(cfg), device="cuda")
+    tabs = [torch.as_tensor(a, device="cuda") for a in wl.tables(cfg)]
+    t = nt.Tracker(deterministic=True)
+    t.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, dens)
+    t.load_cross_sections(*tabs)
+    t.inject_particles(cfg.n_particles, 0, cfg.n_particles, cfg.source, cfg.e0, cfg.seed)
+    t.run_timestep(cfg.dt)
+    out = torch.empty((cfg.ny, cfg.nx), dtype=torch.float64, device="cuda")
+    t.read_tally(out)
+    ot, _, _ = orc.run(cfg)
+    compare_tally(out.cpu().numpy(), ot)
+    t.close()
+
+
+# ---------------------------------------------------------------------------------------------
+# Full BASELINE.json sizes, production launch configuration (what bench.py times).
+SCALE = ["csp", "stream", "scatter", "split"]
+
+
+def _sample_ids(n, k=48):
+    ids = np.unique(np.concatenate([np.arange(8), np.linspace(0, n - 1, k).astype(np.int64), [n - 1]]))
+    return ids
+
+
+@pytest.mark.parametrize("mode", MODES)
+@pytest.mark.parametrize("cfgname", SCALE)
+def test_scale_sampled_parity_and_properties(nt, orc, cfgname, mode):
+    cfg = wl.CONFIGS[cfgname]
+    t = nt.setup(cfg, mode=mode)
+    s = t.run_timestep(cfg.dt)
+    tally = t.read_tally()
+    g = t.read_particles()
+    t.close()
+    assert s["status"] == 0
+    n = cfg.n_particles
+    # properties at any size
+    assert s["n_alive_start"] == n and s["n_census"] + s["n_killed"] == n          # P5
+    assert s["n_facets"] == int(g["nfac"].astype(np.int64).sum())
+    assert s["n_collisions"] == int(g["ncol"].astype(np.int64).sum())
+    assert np.array_equal(g["ctr"].astype(np.int64), 2 + g["ncol"].astype(np.int64))
+    tot = tally.sum()
+    assert abs(tot - s["tally_total"]) <= 1e-9 * abs(tot)
+    assert abs(tot - g["dep"].sum()) <= 1e-9 * abs(tot)
+    r = g["dep"] + g["w"] * g["e"] - cfg.e0                                       # P10
+    assert abs(r.mean()) < 5 * r.std() / math.sqrt(n) + 1e-9 * cfg.e0
+    wl_ = s["census_weight"] + s["killed_weight"] + s["absorbed_weight"]
+    assert abs(wl_ - n) <= 1e-9 * n
+    # sampled per-particle parity: the oracle recomputes these ids one by one
+    prob = orc.Problem(cfg, wl.density(cfg), wl.tables(cfg))
+    ids = _sample_ids(n)
+    for pid in ids:
+        op = orc.inject(prob, int(pid), 1)
+        orc.step(prob, op, int(pid), np.zeros(cfg.nx * cfg.ny))
+        gp = {k: v[pid:pid + 1] for k, v in g.items()}
+        compare_particles(gp, op)
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_scale_deterministic_subrange(nt, orc, mode):
+    """Paper-size mesh, id subrange [0, K): the deterministic tally equals the oracle's."""
+    cfg = wl.CONFIGS["csp"]
+    K = 6000
+    gt, gp, (gs,) = _gpu_run(nt, cfg, n_local=K, deterministic=True, mode=mode)
+    ot, op, (os_,) = orc.run(cfg, n_local=K)
+    compare_particles(gp, op)
+    rep = compare_tally(gt, ot)
+    compare_stats(gs, os_)
+    print(rep)
