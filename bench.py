@@ -1,0 +1,359 @@
+#!/usr/bin/env python
+"""Benchmark: particle events/s per timestep of the B200 neutral tracker (BASELINE.json metric).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config csp] [--mode history]
+    python -m torch.distributed.run --nproc-per-node N --master-addr 127.0.0.1 bench.py --gpus N
+    python bench.py --impl reference ...      # the oracle on the host cores (reference arm)
+
+A step is one pass of the whole hot path over one batch of synthetic input:
+nt_inject_particles + nt_run_timestep (tally zero, tracking kernel, statistics, and the NCCL
+tally allreduce when N > 1).  Inputs (mesh, tables) are resident in HBM; the working set
+(128 MB density + 128 MB tally + particle store) exceeds the 126 MB L2, so no explicit L2
+flush is needed.  Weak scaling: every rank tracks the config's full particle count with
+its own global id range.  Rank 0 prints one JSON line.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import statistics
+import subprocess
+import sys
+import time
+from pathlib import Path
+
+import numpy as np
+
+ROOT = Path(__file__).resolve().parent
+sys.path.insert(0, str(ROOT))
+
+from paper_conf_cluster_martineaum17_b200 import workloads as wl  # noqa: E402
+
+METRIC = "particle events/sec per timestep at 1/2/4/8 B200; % of HBM roofline"
+UNIT = "events/s"
+
+# Algorithmic HBM bytes of the method: a facet reads the
+# entered cell's density (8 B) and read-modify-writes the exited cell's tally (16 B); a
+# census or kill flush is one tally RMW (16 B); every particle's state (x, y, ωx, ωy, E, w,
+# n_mfp, cx, cy, ctr, status = 69 B) is read and written once per step.
+B_FACET, B_FLUSH, B_PARTICLE = 24, 16, 138
+
+
+def algorithmic_bytes(s: dict) -> int:
+    return (B_FACET * s["n_facets"] + B_FLUSH * (s["n_census"] + s["n_killed"])
+            + B_PARTICLE * s["n_alive_start"])
+
+
+def measured_peaks() -> dict:
+    p = ROOT / "MEASURED_PEAKS.json"
+    if p.exists():
+        d = json.loads(p.read_text())
+        return {"hbm_gbs": d["hbm_gbs"], "source": "measured (MEASURED_PEAKS.json)"}
+    return {"hbm_gbs": 6650.0, "source": "fallback (B200_PROFILING.md)"}
+
+
+def ncu_traffic(config: str, mode: str):
+    """Per-launch DRAM bytes of the tracking kernel from a committed ncu --set full capture."""
+    p = ROOT / "profiles" / "ncu_traffic.json"
+    if not p.exists():
+        return None
+    d = json.loads(p.read_text())
+    return d.get(f"{config}/{mode}")
+
+
+# ---- clocks sampled during the timed region ------------------------------------------------
+class ClockSampler:
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, gpu_index: int):
+        self.idx = gpu_index
+        self.proc = None
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-i", str(self.idx), "-lms", "200"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+        except Exception:
+            self.proc = None
+        time.sleep(0.3)
+        return self
+
+    def __exit__(self, *a):
+        self.out = ""
+        if self.proc:
+            time.sleep(0.25)
+            self.proc.terminate()
+            try:
+                self.out, _ = self.proc.communicate(timeout=5)
+            except Exception:
+                self.proc.kill()
+
+    def summary(self) -> dict:
+        rows = []
+        for line in (getattr(self, "out", "") or "").splitlines():
+            f = [x.strip() for x in line.split(",")]
+            if len(f) < 9:
+                continue
+            try:
+                rows.append((float(f[1]), float(f[2]), f[5:9]))
+            except ValueError:
+                continue
+        if not rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unavailable"], "samples": 0}
+        smax = max(r[1] for r in rows)
+        loaded = [r for r in rows if r[0] > 0.5 * smax] or rows
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in loaded for i, v in enumerate(r[2]) if v.lower() == "active"})
+        return {"sm_mhz": statistics.median(r[0] for r in loaded), "sm_max_mhz": smax,
+                "reasons": reasons, "samples": len(rows)}
+
+
+# ---- the oracle on the host cores (cpu_baseline leg and --impl reference) ----------------------
+_ORC_STATE = {}
+
+
+def _oracle_worker(args):
+    lo, n = args
+    import oracle
+    prob = _ORC_STATE["prob"]
+    t0 = time.perf_counter()
+    p = oracle.inject(prob, lo, n)
+    tally = np.zeros(prob.cfg.nx * prob.cfg.ny)
+    st = oracle.step(prob, p, lo, tally)
+    dt = time.perf_counter() - t0
+    return st["n_facets"] + st["n_collisions"] + st["n_census"], dt
+
+
+def oracle_host_rate(cfg, budget_s: float = 12.0, max_procs: int | None = None) -> dict:
+    """Events/s of the unmodified oracle on the host's cores: one process per core, each on
+    a disjoint id range of the workload (ids are iid, so events/s is intensive)."""
+    import multiprocessing as mp
+
+    import oracle
+    oracle.build()
+    prob = oracle.Problem(cfg, wl.density(cfg), wl.tables(cfg))
+    _ORC_STATE["prob"] = prob
+    cores = len(os.sched_getaffinity(0)) if hasattr(os, "sched_getaffinity") else os.cpu_count()
+    procs = max(1, min(cores, max_procs or cores))
+    # calibrate on one core
+    ev, dt = _oracle_worker((0, 64))
+    per_particle = max(dt / 64, 1e-7)
+    n_per = max(1, int(budget_s / per_particle))
+    n_per = min(n_per, max(1, cfg.n_particles // procs))
+    ranges = [(r * n_per, n_per) for r in range(procs)]
+    ctx = mp.get_context("fork")
+    t0 = time.perf_counter()
+    with ctx.Pool(procs) as pool:
+        res = pool.map(_oracle_worker, ranges)
+    wall = time.perf_counter() - t0
+    events = sum(r[0] for r in res)
+    slowest = max(r[1] for r in res)
+    return {"value": events / slowest, "unit": UNIT, "cores": procs, "kind": "oracle",
+            "sample": f"{cfg.name}: ids [0, {procs * n_per}) as {procs} processes x {n_per} particles "
+                      f"(1 step each, {events} events, slowest process {slowest:.2f} s, wall {wall:.2f} s)"}
+
+
+# ---- main --------------------------------------------------------------------------------------
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--config", default="csp", choices=sorted(wl.CONFIGS))
+    ap.add_argument("--mode", default="history", choices=["history", "event"])
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--ctas-per-sm", type=int, default=0)
+    ap.add_argument("--json-out", default=None)
+    return ap.parse_args()
+
+
+def dist_env():
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return rank, world, local
+
+
+def emit(d: dict, path: str | None):
+    line = json.dumps(d)
+    print(line, flush=True)
+    if path:
+        Path(path).parent.mkdir(parents=True, exist_ok=True)
+        Path(path).write_text(line + "\n")
+
+
+def run_reference(a):
+    rank, world, _ = dist_env()
+    if rank != 0:
+        return
+    cfg = wl.CONFIGS[a.config]
+    n_gpus = max(a.gpus, world)
+    budget = max(3.0, min(20.0, 120.0 / max(1, a.steps + a.warmup)))
+    vals = []
+    last = None
+    for k in range(a.warmup + a.steps):
+        r = oracle_host_rate(cfg, budget_s=budget)
+        if k >= a.warmup:
+            vals.append(r["value"])
+            last = r
+    v = statistics.median(vals)
+    cpu = dict(last)
+    cpu["value"] = v
+    emit({"impl": "reference", "metric": METRIC, "value": v, "unit": UNIT, "n_gpus": n_gpus,
+          "steps": a.steps, "warmup": a.warmup, "ms_per_step": None, "higher_is_better": True,
+          "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+          "config": {"workload": cfg.name, "mode": "oracle (Listing 1, single-threaded per process)",
+                     "nx": cfg.nx, "ny": cfg.ny, "particles_per_gpu": cfg.n_particles},
+          "cpu_baseline": cpu,
+          "e2e": {"value": v, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}},
+         a.json_out)
+
+
+def main():
+    a = parse()
+    if a.impl == "reference":
+        return run_reference(a)
+    import torch
+    import torch.distributed as dist
+
+    from paper_conf_cluster_martineaum17_b200 import binding
+
+    rank, world, local = dist_env()
+    if world > 1 and not dist.is_initialized():
+        torch.cuda.set_device(local)
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    torch.cuda.set_device(local)
+    cfg = wl.CONFIGS[a.config]
+    n_per = cfg.n_particles
+    n_total = n_per * world
+    first_id = rank * n_per
+    uid = None
+    if world > 1:
+        obj = [binding.get_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        uid = obj[0]
+    stream = torch.cuda.current_stream()
+    tr = binding.Tracker(device=local, stream=stream.cuda_stream, mode=a.mode, rank=rank,
+                         nranks=world, unique_id=uid, A=cfg.A, molar_mass=cfg.molar_mass,
+                         e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm)
+    density = wl.density(cfg)
+    tables = wl.tables(cfg)
+    tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
+    tr.load_cross_sections(*tables)
+
+    def step():
+        tr.inject_particles(n_total, first_id, n_per, cfg.source, cfg.e0, cfg.seed)
+        return tr.run_timestep(cfg.dt)
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+
+    for _ in range(a.warmup):
+        step()
+    barrier()
+    vis = os.environ.get("CUDA_VISIBLE_DEVICES", "").split(",")
+    gidx = int(vis[local]) if len(vis) > local and vis[local].strip().isdigit() else local
+    stats = []
+    with ClockSampler(gidx) as clk:
+        barrier()
+        e0 = torch.cuda.Event(enable_timing=True)
+        e1 = torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        for _ in range(a.steps):
+            stats.append(step())
+        e1.record(stream)
+        barrier()
+    ms = e0.elapsed_time(e1)
+    t = torch.tensor([ms], dtype=torch.float64, device="cuda")
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    ms = float(t.item())
+    # events: the step statistics are already summed over ranks when world > 1
+    events = sum(s["events"] for s in stats)
+    value = events / (ms / 1e3)
+    track_ms = statistics.mean(s["track_ms"] for s in stats)
+    ab = statistics.mean(algorithmic_bytes(s) for s in stats) / world   # per rank launch
+    peaks = measured_peaks()
+    achieved = ab / (track_ms / 1e3) / 1e9
+    traffic = ncu_traffic(cfg.name, a.mode)
+    status = {s["status"] for s in stats}
+    launches = sum(s["n_launches"] + 1 for s in stats)          # + inject kernel per step
+
+    e2e = None
+    if not a.no_e2e:
+        pin_d = torch.from_numpy(density).pin_memory()
+        pin_t = [torch.from_numpy(np.ascontiguousarray(x)).pin_memory() for x in tables]
+        out = torch.empty((cfg.ny, cfg.nx), dtype=torch.float64).pin_memory()
+        h2d = pin_d.numel() * 8 + sum(x.numel() * 8 for x in pin_t)
+        d2h = out.numel() * 8 + 160          # tally + step statistics
+        barrier()
+        f0 = torch.cuda.Event(enable_timing=True)
+        f1 = torch.cuda.Event(enable_timing=True)
+        ev_e2e = 0
+        f0.record(stream)
+        for _ in range(a.steps):
+            tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, pin_d)
+            tr.load_cross_sections(*pin_t)
+            s = step()
+            tr.read_tally(out)
+            ev_e2e += s["events"]
+        f1.record(stream)
+        barrier()
+        ms2 = f0.elapsed_time(f1)
+        t2 = torch.tensor([ms2], dtype=torch.float64, device="cuda")
+        if world > 1:
+            dist.all_reduce(t2, op=dist.ReduceOp.MAX)
+        e2e = {"value": ev_e2e / (float(t2.item()) / 1e3), "unit": UNIT, "h2d_bytes_per_step": h2d,
+               "d2h_bytes_per_step": d2h, "ms_per_step": float(t2.item()) / a.steps,
+               "path": "C ABI with pinned host buffers: init_mesh + load_cross_sections + inject + "
+                       "run_timestep + read_tally"}
+    tr.close()
+
+    cpu = None
+    if rank == 0 and world == 1 and not a.no_cpu_baseline:
+        cpu = oracle_host_rate(cfg)
+
+    if rank == 0:
+        s0 = stats[-1]
+        emit({
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": a.steps,
+            "warmup": a.warmup, "ms_per_step": ms / a.steps, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+            "config": {"workload": cfg.name, "mode": a.mode, "nx": cfg.nx, "ny": cfg.ny,
+                       "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
+                       "tables": [len(tables[0]), len(tables[2])],
+                       "parallelism": f"dp{world} (particle id shards, tally NCCL allreduce)",
+                       "l2": "no flush: working set (128 MB density + 128 MB tally + particles) > 126 MB L2",
+                       "step": "inject_particles + run_timestep"},
+            "events_per_step": events / a.steps,
+            "event_mix": {"facets": s0["n_facets"], "collisions": s0["n_collisions"],
+                          "census": s0["n_census"], "killed": s0["n_killed"]},
+            "status": sorted(status),
+            "roofline": {"bound": "hbm", "kernel": f"history_kernel<false>" if a.mode == "history" else "event kernels",
+                         "achieved": achieved, "peak": peaks["hbm_gbs"], "unit": "GB/s",
+                         "frac": achieved / peaks["hbm_gbs"], "traffic": traffic,
+                         "algorithmic_bytes_per_launch": ab, "kernel_ms": track_ms,
+                         "kernel_share_of_step": track_ms / (ms / a.steps),
+                         "peak_source": peaks["source"]},
+            "cpu_baseline": cpu,
+            "e2e": e2e,
+            "gpu_launches": launches,
+            "clocks": clk.summary(),
+        }, a.json_out)
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

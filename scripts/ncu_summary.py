@@ -1,0 +1,108 @@
+#!/usr/bin/env python
+"""Summarise an ncu --set full capture (run here, on the CPU box, with ncu -i).
+
+    python scripts/ncu_summary.py gpurun_out/r01/prof.ncu-rep profiles/r01_csp_history_ncu.md \
+        [--traffic-key csp/history]
+
+Writes the key metrics (time, DRAM bytes, hit rates, REDs, occupancy, divergence, FP64 pipe,
+stall reasons) and the top stall-sampled SASS lines; with --traffic-key also records
+dram read+write bytes per launch into profiles/ncu_traffic.json (bench.py's roofline.traffic).
+"""
+from __future__ import annotations
+
+import argparse
+import csv
+import io
+import json
+import re
+import subprocess
+from pathlib import Path
+
+KEYS = [
+    "gpu__time_duration.sum", "dram__bytes_read.sum", "dram__bytes_write.sum",
+    "dram__throughput.avg.pct_of_peak_sustained_elapsed", "lts__t_sector_hit_rate.pct",
+    "l1tex__t_sector_hit_rate.pct", "lts__t_requests_srcunit_tex_op_red.sum",
+    "smsp__inst_executed_op_global_red.sum", "lts__throughput.avg.pct_of_peak_sustained_elapsed",
+    "l1tex__throughput.avg.pct_of_peak_sustained_elapsed", "sm__warps_active.avg.pct_of_peak_sustained_active",
+    "launch__registers_per_thread", "launch__occupancy_limit_registers", "launch__grid_size",
+    "launch__block_size", "smsp__thread_inst_executed_per_inst_executed.ratio",
+    "sm__pipe_fp64_cycles_active.avg.pct_of_peak_sustained_active", "smsp__inst_executed.sum",
+    "smsp__issue_active.avg.pct_of_peak_sustained_active", "sm__throughput.avg.pct_of_peak_sustained_elapsed",
+]
+STALL = re.compile(r"^smsp__pcsamp_warps_issue_stalled_([a-z_]+)$")
+
+
+def ncu(args):
+    return subprocess.run(["ncu", *args], capture_output=True, text=True, check=True).stdout
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("rep")
+    ap.add_argument("out")
+    ap.add_argument("--traffic-key", default=None)
+    ap.add_argument("--top", type=int, default=25)
+    a = ap.parse_args()
+    raw = list(csv.reader(io.StringIO(ncu(["-i", a.rep, "--page", "raw", "--csv"]))))
+    hdr, units, rows = raw[0], raw[1], raw[2:]
+    lines = [f"# ncu summary: {Path(a.rep).name}", ""]
+    traffic = None
+    for r in rows:
+        d = dict(zip(hdr, r))
+        u = dict(zip(hdr, units))
+        lines.append(f"## kernel `{d.get('Kernel Name', '?')}`")
+        lines.append("")
+        lines.append("| metric | value | unit |")
+        lines.append("|---|---|---|")
+        for k in KEYS:
+            if k in d:
+                lines.append(f"| {k} | {d[k]} | {u[k]} |")
+        stalls = {}
+        for k, v in d.items():
+            m = STALL.match(k)
+            if m and v not in ("", "0"):
+                try:
+                    stalls[m.group(1)] = float(v.replace(",", ""))
+                except ValueError:
+                    pass
+        tot = sum(stalls.values()) or 1.0
+        lines.append("")
+        lines.append("| stall reason (pc sampling) | share |")
+        lines.append("|---|---|")
+        for k, v in sorted(stalls.items(), key=lambda kv: -kv[1])[:12]:
+            lines.append(f"| {k} | {100 * v / tot:.1f}% |")
+        def num(k, scale):
+            s = d.get(k, "").replace(",", "")
+            f = float(s) if s else 0.0
+            un = u.get(k, "")
+            mult = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "Tbyte": 1e12}.get(un, 1)
+            return f * mult
+        traffic = num("dram__bytes_read.sum", 1) + num("dram__bytes_write.sum", 1)
+        lines.append("")
+        lines.append(f"DRAM traffic per launch (read + write): {traffic:.4g} B")
+    # source page: top stall-sampled SASS lines
+    try:
+        src = list(csv.reader(io.StringIO(ncu(["-i", a.rep, "--page", "source", "--csv",
+                                                "--print-source", "sass"]))))
+        h = src[1]
+        body = src[2:]
+        iS, iW = h.index("Source"), h.index("Warp Stall Sampling (All Samples)")
+        iE, iT = h.index("Instructions Executed"), h.index("Avg. Threads Executed")
+        tot = sum(int(x[iW]) for x in body) or 1
+        lines += ["", f"### top {a.top} stall-sampled SASS instructions", "",
+                  "| # | share | executed | avg threads | SASS |", "|---|---|---|---|---|"]
+        for k, x in sorted(enumerate(body), key=lambda kx: -int(kx[1][iW]))[:a.top]:
+            lines.append(f"| {k} | {100 * int(x[iW]) / tot:.1f}% | {x[iE]} | {x[iT]} | `{x[iS].strip()}` |")
+    except Exception as e:  # noqa: BLE001
+        lines.append(f"(source page unavailable: {e})")
+    Path(a.out).write_text("\n".join(lines) + "\n")
+    if a.traffic_key and traffic:
+        p = Path(a.out).parent / "ncu_traffic.json"
+        d = json.loads(p.read_text()) if p.exists() else {}
+        d[a.traffic_key] = traffic
+        p.write_text(json.dumps(d, indent=1, sort_keys=True) + "\n")
+    print(f"wrote {a.out}")
+
+
+if __name__ == "__main__":
+    main()
