@@ -171,6 +171,7 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--ctas-per-sm", type=int, default=0)
+    ap.add_argument("--refill-min", type=int, default=0)
     ap.add_argument("--json-out", default=None)
     return ap.parse_args()
 
@@ -243,7 +244,8 @@ def main():
     stream = torch.cuda.current_stream()
     tr = binding.Tracker(device=local, stream=stream.cuda_stream, mode=a.mode, rank=rank,
                          nranks=world, unique_id=uid, A=cfg.A, molar_mass=cfg.molar_mass,
-                         e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm)
+                         e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm,
+                         refill_min=a.refill_min)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)

@@ -71,6 +71,11 @@ typedef struct {
     int32_t block_size;        /* threads per CTA of the tracking kernel (0 -> default)   */
     int32_t ctas_per_sm;       /* persistent CTAs per SM (0 -> occupancy maximum)         */
     int64_t det_batch;         /* deterministic mode: particles per batch (0 -> 65536)    */
+    int32_t refill_min;        /* history mode: a warp refills its idle lanes once at least
+                                  this many are idle (0 -> 1)                              */
+    int32_t density_format;    /* 0: lossless u8/u16 material codes when the density map
+                                  holds <= 256 / 65536 distinct values, else f64;
+                                  1: always the f64 map                                    */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

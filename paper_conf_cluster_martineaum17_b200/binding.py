@@ -39,7 +39,8 @@ class Options(C.Structure):
                 ("nccl_unique_id", C.c_void_p), ("A", C.c_double), ("molar_mass", C.c_double),
                 ("e_min", C.c_double), ("w_min", C.c_double),
                 ("max_events_per_history", C.c_int64), ("block_size", C.c_int32),
-                ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64)]
+                ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64),
+                ("refill_min", C.c_int32), ("density_format", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -142,7 +143,8 @@ class Tracker:
                  deterministic: bool = False, rank: int = 0, nranks: int = 1,
                  unique_id: bytes | None = None, A: float = 1.0, molar_mass: float = 1e-3,
                  e_min: float = 1.0, w_min: float = 1e-3, max_events: int = 0,
-                 ctas_per_sm: int = 0, det_batch: int = 0):
+                 ctas_per_sm: int = 0, det_batch: int = 0, refill_min: int = 0,
+                 density_format: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -157,6 +159,8 @@ class Tracker:
         o.max_events_per_history = max_events
         o.ctas_per_sm = ctas_per_sm
         o.det_batch = det_batch
+        o.refill_min = refill_min
+        o.density_format = density_format
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:

@@ -60,6 +60,8 @@ struct nt_ctx {
   int32_t nx = 0, ny = 0;
   double W = 0, H = 0;
   DevBuf rho, tally, tally_local, ex, ey;
+  DevBuf rho_code, nd_tab, enc_keys;     // lossless density encoding
+  int dens_fmt = kDensF64, dens_codes = 0;
   // tables
   DevBuf xs;
   Tables tables{};
@@ -179,6 +181,7 @@ nt_status nt_options_default(nt_options* opt) {
   opt->w_min = 1.0e-3;
   opt->max_events_per_history = 1000000000ll;
   opt->det_batch = 65536;
+  opt->refill_min = 1;
   return NT_OK;
 }
 
@@ -210,6 +213,8 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.max_events_per_history <= 0) opt.max_events_per_history = def.max_events_per_history;
   if (opt.det_batch <= 0) opt.det_batch = def.det_batch;
   if (opt.det_batch > 65536) opt.det_batch = 65536;
+  if (opt.refill_min <= 0) opt.refill_min = def.refill_min;
+  if (opt.refill_min > 32) opt.refill_min = 32;
   if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
       opt.rank < 0 || opt.rank >= opt.nranks)
@@ -254,7 +259,7 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
-  for (DevBuf* b : {&c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
+  for (DevBuf* b : {&c->rho_code, &c->nd_tab, &c->enc_keys, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup})
     b->release();
@@ -267,29 +272,65 @@ nt_status nt_destroy(nt_ctx* c) {
 }
 
 // ---- mesh ----------------------------------------------------------
+// The density is copied straight into device memory, validated there, and -- when the map
+// holds few distinct values (density_format 0) -- encoded losslessly as u8/u16 material
+// codes plus a number-density table, so the tracker's per-facet gather is 1-2 B instead of
+// 8 B and the map stays L2-resident.
 nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double height,
                        const double* density) {
   if (!c) return NT_ERR_ARG;
   cudaSetDevice(c->device);
   if (nx < 1 || ny < 1) return fail(c, NT_ERR_ARG, "nx, ny must be >= 1 (got %d, %d)", nx, ny);
+  if ((int64_t)nx * (int64_t)ny > (1ll << 31))
+    return fail(c, NT_ERR_ARG, "nx * ny must be <= 2^31");
   if (!(width > 0.0) || !(height > 0.0) || !is_fin(width) || !is_fin(height))
     return fail(c, NT_ERR_ARG, "width, height must be finite and > 0");
   if (!density) return fail(c, NT_ERR_ARG, "density is NULL");
-  const size_t cells = (size_t)nx * (size_t)ny;
-  std::vector<double> h;
-  NT_CUDA(c, fetch(h, density, (int64_t)cells, c->stream));
-  for (size_t k = 0; k < cells; ++k)
-    if (!(h[k] >= 0.0) || !is_fin(h[k]))
-      return fail(c, NT_ERR_ARG, "density[%zu] = %g is not finite and >= 0", k, h[k]);
-  NT_CUDA(c, c->rho.ensure(cells * 8));
-  NT_CUDA(c, c->tally.ensure(cells * 8));
+  const int64_t cells = (int64_t)nx * (int64_t)ny;
+  c->stage = ST_CREATED;
+  NT_CUDA(c, c->rho.ensure((size_t)cells * 8));
+  NT_CUDA(c, c->tally.ensure((size_t)cells * 8));
   NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
   NT_CUDA(c, c->ey.ensure(((size_t)ny + 1) * 8));
-  NT_CUDA(c, cudaMemcpyAsync(c->rho.p, h.data(), cells * 8, cudaMemcpyHostToDevice, c->stream));
-  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, cells * 8, c->stream));
+  NT_CUDA(c, c->scratch.ensure(1024));
+  NT_CUDA(c, cudaMemcpyAsync(c->rho.p, density, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
+  unsigned long long* bad = c->scratch.as<unsigned long long>();
+  NT_CUDA(c, cudaMemsetAsync(bad, 0, 16, c->stream));
+  NT_CUDA(c, launch_density_check(c->rho.as<double>(), cells, bad, c->stream));
+  // distinct density values (for the lossless encoding)
+  int fmt = kDensF64, nu = 0;
+  if (c->opt.density_format == 0) {
+    size_t tmp = 0;
+    NT_CUDA(c, c->enc_keys.ensure((size_t)cells * 16));
+    unsigned long long* k0 = c->enc_keys.as<unsigned long long>();
+    unsigned long long* k1 = k0 + cells;
+    int* d_count = reinterpret_cast<int*>(c->scratch.as<char>() + 8);
+    NT_CUDA(c, density_distinct(c->rho.as<double>(), cells, k0, k1, nullptr, tmp, d_count, c->stream));
+    NT_CUDA(c, c->sort_tmp.ensure(tmp));
+    NT_CUDA(c, density_distinct(c->rho.as<double>(), cells, k0, k1, c->sort_tmp.p, tmp, d_count, c->stream));
+  }
+  unsigned long long hb[2] = {0, 0};
+  NT_CUDA(c, cudaMemcpyAsync(hb, bad, 16, cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  if (hb[0] != 0)
+    return fail(c, NT_ERR_ARG, "%llu density values are not finite and >= 0", hb[0]);
+  if (c->opt.density_format == 0) {
+    nu = (int)(hb[1] & 0xffffffffu);
+    if (nu <= 256) fmt = kDensU8;
+    else if (nu <= 65536) fmt = kDensU16;
+  }
+  if (fmt != kDensF64) {
+    NT_CUDA(c, c->rho_code.ensure((size_t)cells * (fmt == kDensU8 ? 1 : 2)));
+    NT_CUDA(c, c->nd_tab.ensure((size_t)nu * 8));
+    NT_CUDA(c, launch_encode(c->rho.as<double>(), cells, c->enc_keys.as<unsigned long long>(), nu,
+                             c->ph.cn, fmt, c->rho_code.p, c->nd_tab.as<double>(), c->stream));
+  }
+  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, (size_t)cells * 8, c->stream));
   launch_edges(c->ex.as<double>(), nx, width, c->ey.as<double>(), ny, height, c->stream);
   NT_CUDA(c, cudaGetLastError());
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  c->dens_fmt = fmt;
+  c->dens_codes = nu;
   c->nx = nx;
   c->ny = ny;
   c->W = width;
@@ -320,22 +361,71 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
         return fail(c, NT_ERR_ARG, "table %d value %lld not finite and >= 0", k / 2, (long long)j);
     }
   }
-  size_t off[4], total = 0;
+  // bucket indexes over the IEEE bit patterns of the (positive) keys
+  std::vector<uint32_t> idx[2];
+  uint64_t base[2] = {0, 0};
+  int32_t shift[2] = {0, 0}, nbk[2] = {0, 0};
+  for (int t = 0; t < 2; ++t) {
+    const std::vector<double>& k = h[2 * t];
+    const int64_t n = len[2 * t];
+    if (!(k[0] > 0.0)) continue;                       // index needs positive keys
+    uint64_t b0, b1;
+    std::memcpy(&b0, &k[0], 8);
+    std::memcpy(&b1, &k[n - 1], 8);
+    const uint64_t range = b1 - b0;
+    int64_t target = n / 4;
+    if (target < 1) target = 1;
+    if (target > 16384) target = 16384;
+    int s = 0;
+    while ((range >> s) >= (uint64_t)target) ++s;
+    const int64_t nb = (int64_t)(range >> s) + 1;
+    idx[t].resize((size_t)nb + 1);
+    for (int64_t b = 0; b <= nb; ++b) {
+      const uint64_t bits = b0 + ((uint64_t)b << s);
+      double v;
+      if (bits >= 0x7ff0000000000000ull) v = INFINITY; else std::memcpy(&v, &bits, 8);
+      // bin of v: max{i in [0, n-2] : k[i] <= v}
+      int64_t lo = 0, hi = n - 1;
+      if (v >= k[n - 1]) lo = n - 2;
+      else
+        while (hi - lo > 1) {
+          const int64_t mid = (lo + hi) / 2;
+          if (k[mid] <= v) lo = mid; else hi = mid;
+        }
+      idx[t][(size_t)b] = (uint32_t)lo;
+    }
+    base[t] = b0;
+    shift[t] = s;
+    nbk[t] = (int32_t)nb;
+  }
+  size_t off[6], total = 0;
   for (int k = 0; k < 4; ++k) {
     off[k] = total;
     total += align256((size_t)len[k] * 8);
+  }
+  for (int t = 0; t < 2; ++t) {
+    off[4 + t] = total;
+    total += align256(idx[t].size() * 4 + 4);
   }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k].data(), (size_t)len[k] * 8,
                                cudaMemcpyHostToDevice, c->stream));
+  for (int t = 0; t < 2; ++t)
+    if (!idx[t].empty())
+      NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[4 + t], idx[t].data(), idx[t].size() * 4,
+                                 cudaMemcpyHostToDevice, c->stream));
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
-  c->tables.sk = reinterpret_cast<const double*>(c->xs.as<char>() + off[0]);
-  c->tables.sv = reinterpret_cast<const double*>(c->xs.as<char>() + off[1]);
-  c->tables.ck = reinterpret_cast<const double*>(c->xs.as<char>() + off[2]);
-  c->tables.cv = reinterpret_cast<const double*>(c->xs.as<char>() + off[3]);
-  c->tables.ns = (int32_t)ns;
-  c->tables.nc = (int32_t)nc;
+  Table* T[2] = {&c->tables.s, &c->tables.c};
+  for (int t = 0; t < 2; ++t) {
+    T[t]->k = reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t]);
+    T[t]->v = reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t + 1]);
+    T[t]->idx = reinterpret_cast<const uint32_t*>(c->xs.as<char>() + off[4 + t]);
+    T[t]->n = (int32_t)len[2 * t];
+    T[t]->nb = nbk[t];
+    T[t]->shift = shift[t];
+    T[t]->base = base[t];
+  }
   c->stage = ST_XS;
   return NT_OK;
 }
@@ -403,6 +493,11 @@ nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int6
 static TrackParams make_params(nt_ctx* c, double dt) {
   TrackParams tp{};
   tp.mesh.rho = c->rho.as<double>();
+  tp.mesh.rho8 = c->rho_code.as<uint8_t>();
+  tp.mesh.rho16 = c->rho_code.as<uint16_t>();
+  tp.mesh.nd_tab = c->nd_tab.as<double>();
+  tp.mesh.fmt = c->dens_fmt;
+  tp.mesh.ncodes = c->dens_codes;
   tp.mesh.tally = c->tally.as<double>();
   tp.mesh.ex = c->ex.as<double>();
   tp.mesh.ey = c->ey.as<double>();
@@ -418,6 +513,7 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.seed = c->seed;
   tp.dt = dt;
   tp.max_events = c->opt.max_events_per_history;
+  tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 1;
   char* s = c->scratch.as<char>();
   tp.counter = reinterpret_cast<unsigned long long*>(s);
   tp.stats_u = reinterpret_cast<unsigned long long*>(s + 256);
@@ -425,10 +521,16 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   return tp;
 }
 
+// Register budget / CTAs per SM of the production history kernel: ctas_per_sm option
+// (3: <= 80 registers, no spills; 4: <= 64 registers, spills; 0 -> 3), persistent grid =
+// SMs x resident CTAs.
+static int history_min_blocks(nt_ctx* c) {
+  return c->opt.ctas_per_sm >= 4 ? 4 : 3;
+}
+
 static int history_grid(nt_ctx* c, bool det) {
-  int per_sm = history_max_ctas_per_sm(det, kHistoryBlock);
+  int per_sm = history_max_ctas_per_sm(det, det ? 3 : history_min_blocks(c), c->dens_fmt);
   if (per_sm < 1) per_sm = 1;
-  if (c->opt.ctas_per_sm > 0 && c->opt.ctas_per_sm < per_sm) per_sm = c->opt.ctas_per_sm;
   return c->sm_count * per_sm;
 }
 
@@ -486,7 +588,7 @@ static nt_status run_det_history(nt_ctx* c, const TrackParams& tp, uint32_t& lau
     bp.rec_cap = c->rec_cap;
     bp.rec_count = rec_count;
     NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 16, c->stream));   // work counter, records
-    launch_history(bp, true, grid, kHistoryBlock, c->stream);
+    launch_history(bp, true, grid, 3, c->stream);
     ++launches;
     NT_CUDA(c, cudaGetLastError());
     unsigned long long nrec = 0;
@@ -545,7 +647,7 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
     const nt_status st = run_det_history(c, tp, launches);
     if (st != NT_OK) return st;
   } else {
-    launch_history(tp, false, history_grid(c, false), kHistoryBlock, c->stream);
+    launch_history(tp, false, history_grid(c, false), history_min_blocks(c), c->stream);
     ++launches;
     NT_CUDA(c, cudaGetLastError());
   }

@@ -27,20 +27,39 @@ struct Soa {
   uint8_t *status;
 };
 
+// Density storage (lossless): the f64 map, or -- when the map holds <= 256 (65536) distinct
+// values -- a u8 (u16) material code per cell plus a table of each code's number density
+// rho_k * cn (the product DESIGN.md §3 forms first, computed on the host with the same
+// single rounding).  Either way the kernel obtains nd = rho[cell] * cn bit-identically.
+enum DensFmt { kDensF64 = 0, kDensU16 = 1, kDensU8 = 2 };
+
 struct Mesh {
-  const double* __restrict__ rho;   // [ny][nx] kg/m^3
-  double* __restrict__ tally;       // [ny][nx] eV*weight
-  const double* __restrict__ ex;    // [nx+1] edge(i) = (i*W)/nx
-  const double* __restrict__ ey;    // [ny+1]
+  const double* __restrict__ rho;     // [ny][nx] kg/m^3            (kDensF64)
+  const uint8_t* __restrict__ rho8;   // [ny][nx] material code     (kDensU8)
+  const uint16_t* __restrict__ rho16; // [ny][nx] material code     (kDensU16)
+  const double* __restrict__ nd_tab;  // [codes] rho_k * cn, atoms/m^3
+  double* __restrict__ tally;         // [ny][nx] eV*weight
+  const double* __restrict__ ex;      // [nx+1] edge(i) = (i*W)/nx
+  const double* __restrict__ ey;      // [ny+1]
   int32_t nx, ny;
+  int32_t fmt, ncodes;
+};
+
+// One microscopic cross-section table with its bucket index: bucket b covers the IEEE bit
+// patterns [base + (b << shift), base + ((b+1) << shift)) of positive energies (monotone in
+// the value), and idx[b] is the bin holding the bucket's first value, so the bin of any
+// energy in bucket b lies in [idx[b], idx[b+1]].  nb = 0 disables the index (keys <= 0).
+struct Table {
+  const double* __restrict__ k;     // keys, eV, strictly increasing
+  const double* __restrict__ v;     // values, barns
+  const uint32_t* __restrict__ idx; // [nb + 1]
+  uint64_t base;
+  int32_t n, nb, shift, pad;
 };
 
 struct Tables {
-  const double* __restrict__ sk;    // scatter keys (eV), values (barns)
-  const double* __restrict__ sv;
-  const double* __restrict__ ck;    // capture keys, values
-  const double* __restrict__ cv;
-  int32_t ns, nc;
+  Table s;   // scatter
+  Table c;   // capture
 };
 
 // Sub-expressions of DESIGN.md §3 that depend only on run constants.  Each is computed
@@ -110,22 +129,44 @@ __device__ __forceinline__ int32_t cell_of(double q, const double* __restrict__ 
   return i;
 }
 
+// Number density of a cell: rho[cell] * cn.
+template <int kFmt>
+__device__ __forceinline__ double number_density(const Mesh& M, const double* __restrict__ tab,
+                                                 int64_t cell, double cn) {
+  if constexpr (kFmt == kDensU8) {
+    return tab[__ldg(M.rho8 + cell)];
+  } else if constexpr (kFmt == kDensU16) {
+    return __ldg(tab + __ldg(M.rho16 + cell));
+  } else {
+    return __ldg(M.rho + cell) * cn;
+  }
+}
+
 // ---- microscopic cross sections -----------------------------------------------
-// Bin i = max{i in [0,N-2]: k[i] <= e} for e already in [k0, k_{N-1}]; then lerp.
-__device__ __forceinline__ double xs_lookup(const double* __restrict__ k,
-                                            const double* __restrict__ v, int32_t n,
-                                            double e) {
-  int32_t lo = 0, hi = n - 1;                 // k[lo] <= e < k[hi]  (or e == k[n-1])
+// Bin i = max{i in [0,N-2]: k[i] <= e} for e already in [k0, k_{N-1}] (the energy-bin
+// search), then linear interpolation.  The bucket index narrows the binary search to a
+// few keys; it returns the same bin as a full binary search by construction.
+__device__ __forceinline__ double xs_lookup(const Table& T, double e) {
+  const double* __restrict__ k = T.k;
+  const int32_t n = T.n;
+  int32_t lo, hi;                             // k[lo] <= e < k[hi]
   if (e >= __ldg(k + n - 1)) {
     lo = n - 2;
+    hi = n - 1;
+  } else if (T.nb > 0) {
+    const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
+    lo = (int32_t)__ldg(T.idx + b);
+    hi = (int32_t)__ldg(T.idx + b + 1) + 1;
   } else {
-    while (hi - lo > 1) {
-      const int32_t mid = (lo + hi) >> 1;
-      if (__ldg(k + mid) <= e) lo = mid; else hi = mid;
-    }
+    lo = 0;
+    hi = n - 1;
+  }
+  while (hi - lo > 1) {
+    const int32_t mid = (lo + hi) >> 1;
+    if (__ldg(k + mid) <= e) lo = mid; else hi = mid;
   }
   const double k0 = __ldg(k + lo), k1 = __ldg(k + lo + 1);
-  const double v0 = __ldg(v + lo), v1 = __ldg(v + lo + 1);
+  const double v0 = __ldg(T.v + lo), v1 = __ldg(T.v + lo + 1);
   const double t = (e - k0) / (k1 - k0);
   return v0 + t * (v1 - v0);
 }
@@ -146,10 +187,10 @@ __device__ __forceinline__ double clamp_count(double e, const double* __restrict
 
 __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, double e,
                                           uint32_t& nrange) {
-  const double es = clamp_count(e, T.sk, T.ns, nrange);
-  const double ea = clamp_count(e, T.ck, T.nc, nrange);
-  const double ss = xs_lookup(T.sk, T.sv, T.ns, es);
-  const double sa = xs_lookup(T.ck, T.cv, T.nc, ea);
+  const double es = clamp_count(e, T.s.k, T.s.n, nrange);
+  const double ea = clamp_count(e, T.c.k, T.c.n, nrange);
+  const double ss = xs_lookup(T.s, es);
+  const double sa = xs_lookup(T.c, ea);
   const double t = ss + sa;
   Mat m;
   m.st = t * kBarn;

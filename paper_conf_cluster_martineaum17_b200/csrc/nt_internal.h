@@ -19,6 +19,7 @@ struct TrackParams {
   uint64_t seed;
   double dt;
   int64_t max_events;
+  int32_t refill_min;         // refill a warp's idle lanes once at least this many are idle
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]
@@ -45,8 +46,10 @@ void launch_edges(double* ex, int32_t nx, double W, double* ey, int32_t ny, doub
                   cudaStream_t s);
 void launch_inject(const InjectParams& ip, cudaStream_t s);
 // History (Over Particles) tracking: grid = persistent CTAs.
-void launch_history(const TrackParams& tp, bool det, int grid, int block, cudaStream_t s);
-int history_max_ctas_per_sm(bool det, int block);
+// min_blocks selects the register budget: 4 -> <= 64 regs (1024 threads/SM), 3 -> <= 80;
+// the density format (tp.mesh.fmt) selects the instantiation.
+void launch_history(const TrackParams& tp, bool det, int grid, int min_blocks, cudaStream_t s);
+int history_max_ctas_per_sm(bool det, int min_blocks, int fmt);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);
 void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s);
@@ -59,4 +62,17 @@ cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long*
 
 constexpr int kHistoryBlock = 256;
 
+}  // namespace nt
+
+namespace nt {
+// Mesh preparation (nt_kernels.cu).
+cudaError_t launch_density_check(const double* rho, int64_t n, unsigned long long* bad,
+                                 cudaStream_t s);
+// Sort the density bit patterns (k0 -> k1) and write the distinct ones to k0, their count to
+// *d_count.  temp == nullptr: query temp_bytes.
+cudaError_t density_distinct(const double* rho, int64_t n, unsigned long long* k0,
+                             unsigned long long* k1, void* temp, size_t& temp_bytes,
+                             int* d_count, cudaStream_t s);
+cudaError_t launch_encode(const double* rho, int64_t n, const unsigned long long* uniq, int nu,
+                          double cn, int fmt, void* code, double* nd_tab, cudaStream_t s);
 }  // namespace nt

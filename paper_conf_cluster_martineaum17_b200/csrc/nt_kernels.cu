@@ -79,38 +79,48 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet>
-__global__ void __launch_bounds__(kHistoryBlock)
+template <bool kDet, int kMinBlocks, int kFmt>
+__global__ void __launch_bounds__(kHistoryBlock, kMinBlocks)
 history_kernel(const __grid_constant__ TrackParams P) {
   __shared__ uint32_t s_u[SU_COUNT][kHistoryBlock];
   __shared__ double s_f[SF_COUNT][kHistoryBlock];
+  __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
   const int t = threadIdx.x;
 #pragma unroll
   for (int k = 0; k < SU_COUNT; ++k) s_u[k][t] = 0u;
 #pragma unroll
   for (int k = 0; k < SF_COUNT; ++k) s_f[k][t] = 0.0;
+  if constexpr (kFmt == kDensU8) {
+    for (int k = t; k < 256; k += kHistoryBlock) s_nd[k] = k < P.mesh.ncodes ? P.mesh.nd_tab[k] : 0.0;
+    __syncthreads();
+  }
+  const double* __restrict__ ndtab = (kFmt == kDensU8) ? s_nd : P.mesh.nd_tab;
 
   const int lane = t & 31;
   const unsigned lt_mask = (1u << lane) - 1u;
   const unsigned long long span = (unsigned long long)(P.hi - P.lo);
   const double* __restrict__ ex = P.mesh.ex;
   const double* __restrict__ ey = P.mesh.ey;
-  const double* __restrict__ rho = P.mesh.rho;
   const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
   const Phys& ph = P.ph;
+  const int refill_min = P.refill_min;
 
   bool active = false, exhausted = false;
-  int64_t i = 0;
+  int32_t i = 0;                 // local particle index (< 2^31)
+  // register-resident history state
   double x = 0, y = 0, ox = 0, oy = 0, iox = 0, ioy = 0, e = 0, w = 0, mfp = 0, dcen = 0;
-  double nd = 0, acc = 0, dep = 0;
+  double nd = 0;      // number density of the current cell: Sigma_t = nd * st
+  double exn = 0, eyn = 0;  // edge each axis is heading to (facet distance, snap value)
+  double acc = 0;     // deposit accumulated in the current cell
+  double dstep = 0;   // deposits this particle flushed this step
   Mat m{0, 0, 0};
   int32_t cx = 0, cy = 0;
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
 
   for (;;) {
-    // ---- refill idle lanes with new particles (one atomic per warp) ----
+    // ---- refill idle lanes with new particles: one atomic per warp ----
     const unsigned idle = __ballot_sync(kFull, !active);
-    if (idle != 0u && !exhausted) {
+    if (!exhausted && idle != 0u && (__popc(idle) >= refill_min || idle == kFull)) {
       const int leader = __ffs(idle) - 1;
       unsigned long long base = 0;
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
@@ -119,7 +129,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       if (!active) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
         if (my < span) {
-          i = P.lo + (int64_t)my;
+          i = (int32_t)(P.lo + (int64_t)my);
           if (P.p.status[i] == 1u) {
             active = true;
             x = P.p.x[i];
@@ -129,16 +139,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
             e = P.p.e[i];
             w = P.p.w[i];
             mfp = P.p.mfp[i];
-            dep = P.p.dep[i];
             cx = P.p.cx[i];
             cy = P.p.cy[i];
             ctr = P.p.ctr[i];
-            nd = __ldg(rho + (int64_t)cy * nx + cx) * ph.cn;
+            nd = number_density<kFmt>(P.mesh, ndtab, (int64_t)cy * nx + cx, ph.cn);
+            exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
+            eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             m = refresh_xs(P.xs, ph, e, nrange);
             dcen = speed(e, ph) * P.dt;
             iox = 1.0 / ox;
             ioy = 1.0 / oy;
             acc = 0.0;
+            dstep = 0.0;
             nf = 0u;
             nc = 0u;
             seq = 0u;
@@ -154,17 +166,13 @@ history_kernel(const __grid_constant__ TrackParams P) {
     if (!active) continue;
 
     // ---- one event (Listing 1) ----
-    const uint64_t pid = (uint64_t)(P.first_id + i);
     const double sig = nd * m.st;
-    double tx = d_inf(), ty = d_inf();
-    if (ox != 0.0) {
-      tx = (__ldg(ex + cx + (ox > 0.0 ? 1 : 0)) - x) * iox;
-      tx = tx < 0.0 ? 0.0 : tx;
-    }
-    if (oy != 0.0) {
-      ty = (__ldg(ey + cy + (oy > 0.0 ? 1 : 0)) - y) * ioy;
-      ty = ty < 0.0 ? 0.0 : ty;
-    }
+    double tx = (exn - x) * iox;
+    tx = tx < 0.0 ? 0.0 : tx;
+    tx = ox != 0.0 ? tx : d_inf();
+    double ty = (eyn - y) * ioy;
+    ty = ty < 0.0 ? 0.0 : ty;
+    ty = oy != 0.0 ? ty : d_inf();
     const bool ax = tx < ty;
     const double df = ax ? tx : ty;
     const double dc = sig > 0.0 ? mfp / sig : d_inf();
@@ -177,17 +185,16 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
         if (slot < P.rec_cap) {
           P.rec_key[slot] = ((unsigned long long)cell << 40) |
-                            ((unsigned long long)(i - P.lo) << 24) |
+                            ((unsigned long long)((int64_t)i - P.lo) << 24) |
                             (unsigned long long)(seq & 0xffffffu);
           P.rec_val[slot] = acc;
         }
         if (seq >= (1u << 24)) s_u[SU_REC_OVERFLOW][t] += 1u;
         ++seq;
       } else {
-        atomicAdd(P.mesh.tally + cell, acc);
+        atomicAdd(P.mesh.tally + cell, acc);      // fire-and-forget fp64 RED at L2
       }
-      s_f[SF_TALLY][t] += acc;
-      dep += acc;
+      dstep += acc;
       acc = 0.0;
     };
 
@@ -200,16 +207,16 @@ history_kernel(const __grid_constant__ TrackParams P) {
       s_f[SF_KILLED_W][t] += w;
       outcome = 2;
     } else if (dc < df && dc < ds) {
-      // ---- collision ----
+      // ---- collision (implicit capture + elastic scatter) ----
       acc += ((w * dc) * sig) * m.H;
       x = x + dc * ox;
       y = y + dc * oy;
       dcen = dcen - dc;
-      const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, pid, P.seed);
+      const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
       ctr += 1u;
       nc += 1u;
       const double w_old = w;
-      w = w * (1.0 - m.pa);                               // implicit capture
+      w = w * (1.0 - m.pa);
       s_f[SF_ABSORBED_W][t] += w_old - w;
       const double mu = 1.0 - 2.0 * u01(r.a);
       const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
@@ -230,6 +237,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
         s_u[SU_KILLED][t] += 1u;
         outcome = 2;
       } else {
+        exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
+        eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
         dcen = tcen * speed(e, ph);
         m = refresh_xs(P.xs, ph, e, nrange);
         iox = 1.0 / ox;
@@ -237,32 +246,34 @@ history_kernel(const __grid_constant__ TrackParams P) {
         mfp = -log(u01(r.b));
       }
     } else if (df < ds) {
-      // ---- facet ----
+      // ---- facet: one code path for both axes (no X/Y divergence) ----
       acc += ((w * df) * sig) * m.H;
       const double nm = mfp - df * sig;
       mfp = nm > 0.0 ? nm : 0.0;
       dcen = dcen - df;
-      if (ax) {
-        y = y + df * oy;
-        x = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
-        flush();
-        if (ox > 0.0) {
-          if (cx == nx - 1) { ox = -ox; iox = -iox; } else { cx += 1; }
-        } else {
-          if (cx == 0) { ox = -ox; iox = -iox; } else { cx -= 1; }
-        }
-      } else {
-        x = x + df * ox;
-        y = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
-        flush();
-        if (oy > 0.0) {
-          if (cy == ny - 1) { oy = -oy; ioy = -ioy; } else { cy += 1; }
-        } else {
-          if (cy == 0) { oy = -oy; ioy = -ioy; } else { cy -= 1; }
-        }
-      }
+      const double xm = x + df * ox, ym = y + df * oy;
+      x = ax ? exn : xm;                          // snap the crossed coordinate
+      y = ax ? ym : eyn;
+      flush();                                    // deposit of the cell being left
+      const int32_t c = ax ? cx : cy;
+      const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
+      const int32_t last = (ax ? nx : ny) - 1;
+      const bool refl = pos ? (c == last) : (c == 0);   // reflective boundary
+      const int32_t c2 = refl ? c : (pos ? c + 1 : c - 1);
+      cx = ax ? c2 : cx;
+      cy = ax ? cy : c2;
+      const bool fx = refl && ax, fy = refl && !ax;
+      ox = fx ? -ox : ox;
+      iox = fx ? -iox : iox;
+      oy = fy ? -oy : oy;
+      ioy = fy ? -ioy : ioy;
+      // next edge on the crossed axis and the new cell's density: two independent loads
+      const bool pos2 = refl ? !pos : pos;
+      const double ev = __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
+      nd = number_density<kFmt>(P.mesh, ndtab, (int64_t)cy * nx + cx, ph.cn);
+      exn = ax ? ev : exn;
+      eyn = ax ? eyn : ev;
       nf += 1u;
-      nd = __ldg(rho + (int64_t)cy * nx + cx) * ph.cn;    // density of the new cell
     } else {
       // ---- census ----
       acc += ((w * ds) * sig) * m.H;
@@ -287,7 +298,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       P.p.e[i] = e;
       P.p.w[i] = w;
       P.p.mfp[i] = mfp;
-      P.p.dep[i] = dep;
+      P.p.dep[i] += dstep;
       P.p.cx[i] = cx;
       P.p.cy[i] = cy;
       P.p.ctr[i] = ctr;
@@ -300,6 +311,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       }
       s_u[SU_FACETS][t] += nf;
       s_u[SU_COLLISIONS][t] += nc;
+      s_f[SF_TALLY][t] += dstep;
       active = false;
     }
   }
@@ -327,21 +339,29 @@ history_kernel(const __grid_constant__ TrackParams P) {
   }
 }
 
-void launch_history(const TrackParams& tp, bool det, int grid, int block, cudaStream_t s) {
-  (void)block;
-  if (det)
-    history_kernel<true><<<grid, kHistoryBlock, 0, s>>>(tp);
-  else
-    history_kernel<false><<<grid, kHistoryBlock, 0, s>>>(tp);
+template <bool kDet, int kMinBlocks>
+static void* history_fn(int fmt) {
+  if (fmt == kDensU8) return (void*)history_kernel<kDet, kMinBlocks, kDensU8>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kMinBlocks, kDensU16>;
+  return (void*)history_kernel<kDet, kMinBlocks, kDensF64>;
 }
 
-int history_max_ctas_per_sm(bool det, int block) {
+static void* history_select(bool det, int min_blocks, int fmt) {
+  if (det) return history_fn<true, 3>(fmt);
+  if (min_blocks >= 4) return history_fn<false, 4>(fmt);
+  return history_fn<false, 3>(fmt);
+}
+
+void launch_history(const TrackParams& tp, bool det, int grid, int min_blocks, cudaStream_t s) {
+  void* fn = history_select(det, min_blocks, tp.mesh.fmt);
+  void* args[] = {const_cast<TrackParams*>(&tp)};
+  cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
+}
+
+int history_max_ctas_per_sm(bool det, int min_blocks, int fmt) {
   int n = 0;
-  (void)block;
-  if (det)
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_kernel<true>, kHistoryBlock, 0);
-  else
-    cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_kernel<false>, kHistoryBlock, 0);
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, min_blocks, fmt),
+                                                kHistoryBlock, 0);
   return n;
 }
 
@@ -397,10 +417,10 @@ __global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, in
   const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
   if (i >= n) return;
   uint32_t dummy = 0;
-  const double es = clamp_count(e[i], T.sk, T.ns, dummy);
-  const double ea = clamp_count(e[i], T.ck, T.nc, dummy);
-  os[i] = xs_lookup(T.sk, T.sv, T.ns, es);
-  oa[i] = xs_lookup(T.ck, T.cv, T.nc, ea);
+  const double es = clamp_count(e[i], T.s.k, T.s.n, dummy);
+  const double ea = clamp_count(e[i], T.c.k, T.c.n, dummy);
+  os[i] = xs_lookup(T.s, es);
+  oa[i] = xs_lookup(T.c, ea);
 }
 
 void launch_xs_debug(const Tables& T, const double* e, int64_t n, double* os, double* oa,

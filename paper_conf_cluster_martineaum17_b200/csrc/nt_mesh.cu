@@ -1,0 +1,92 @@
+// nt_mesh.cu -- mesh preparation on the device: density validation and the lossless
+// density encoding (u8 / u16 material codes + number-density table) used by the tracker.
+#include <cub/device/device_radix_sort.cuh>
+#include <cub/device/device_select.cuh>
+
+#include "nt_internal.h"
+
+namespace nt {
+
+// Count cells whose density is not finite or < 0 (nt_init_mesh validation).
+__global__ void density_check_kernel(const double* __restrict__ rho, int64_t n,
+                                     unsigned long long* bad) {
+  unsigned long long local = 0;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+       i += (int64_t)gridDim.x * blockDim.x) {
+    const double v = rho[i];
+    if (!(v >= 0.0) || !isfinite(v)) ++local;
+  }
+  for (int o = 16; o > 0; o >>= 1) local += __shfl_xor_sync(kFull, local, o);
+  if ((threadIdx.x & 31) == 0 && local) atomicAdd(bad, local);
+}
+
+__global__ void bits_kernel(const double* __restrict__ rho, int64_t n,
+                            unsigned long long* __restrict__ out) {
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+       i += (int64_t)gridDim.x * blockDim.x)
+    out[i] = (unsigned long long)__double_as_longlong(rho[i]);
+}
+
+// code[i] = index of rho[i]'s bit pattern among the sorted distinct patterns uniq[0..nu)
+template <class T>
+__global__ void encode_kernel(const double* __restrict__ rho, int64_t n,
+                              const unsigned long long* __restrict__ uniq, int nu,
+                              T* __restrict__ code) {
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+       i += (int64_t)gridDim.x * blockDim.x) {
+    const unsigned long long b = (unsigned long long)__double_as_longlong(rho[i]);
+    int lo = 0, hi = nu;                         // uniq[lo] <= b < uniq[hi]
+    while (hi - lo > 1) {
+      const int mid = (lo + hi) >> 1;
+      if (uniq[mid] <= b) lo = mid; else hi = mid;
+    }
+    code[i] = (T)lo;
+  }
+}
+
+// nd_tab[k] = rho_k * cn: the first product of DESIGN.md §3 MAT, rounded once, as in place.
+__global__ void nd_table_kernel(const unsigned long long* __restrict__ uniq, int nu, double cn,
+                                double* __restrict__ tab) {
+  const int k = blockIdx.x * blockDim.x + threadIdx.x;
+  if (k < nu) tab[k] = __longlong_as_double((long long)uniq[k]) * cn;
+}
+
+static unsigned grid_for(int64_t n) {
+  const int64_t b = (n + 255) / 256;
+  return (unsigned)(b > 148 * 32 ? 148 * 32 : (b < 1 ? 1 : b));
+}
+
+cudaError_t launch_density_check(const double* rho, int64_t n, unsigned long long* bad,
+                                 cudaStream_t s) {
+  density_check_kernel<<<grid_for(n), 256, 0, s>>>(rho, n, bad);
+  return cudaGetLastError();
+}
+
+cudaError_t density_distinct(const double* rho, int64_t n, unsigned long long* k0,
+                             unsigned long long* k1, void* temp, size_t& temp_bytes,
+                             int* d_count, cudaStream_t s) {
+  if (temp == nullptr) {
+    size_t a = 0, b = 0;
+    cudaError_t e = cub::DeviceRadixSort::SortKeys(nullptr, a, k0, k1, n, 0, 64, s);
+    if (e != cudaSuccess) return e;
+    e = cub::DeviceSelect::Unique(nullptr, b, k1, k0, d_count, n, s);
+    temp_bytes = a > b ? a : b;
+    return e;
+  }
+  bits_kernel<<<grid_for(n), 256, 0, s>>>(rho, n, k0);
+  cudaError_t e = cub::DeviceRadixSort::SortKeys(temp, temp_bytes, k0, k1, n, 0, 64, s);
+  if (e != cudaSuccess) return e;
+  return cub::DeviceSelect::Unique(temp, temp_bytes, k1, k0, d_count, n, s);
+}
+
+cudaError_t launch_encode(const double* rho, int64_t n, const unsigned long long* uniq, int nu,
+                          double cn, int fmt, void* code, double* nd_tab, cudaStream_t s) {
+  if (fmt == kDensU8)
+    encode_kernel<uint8_t><<<grid_for(n), 256, 0, s>>>(rho, n, uniq, nu, (uint8_t*)code);
+  else
+    encode_kernel<uint16_t><<<grid_for(n), 256, 0, s>>>(rho, n, uniq, nu, (uint16_t*)code);
+  nd_table_kernel<<<(nu + 255) / 256, 256, 0, s>>>(uniq, nu, cn, nd_tab);
+  return cudaGetLastError();
+}
+
+}  // namespace nt

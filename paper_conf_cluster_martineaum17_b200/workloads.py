@@ -100,6 +100,9 @@ CONFIGS: dict[str, Config] = {
                                    sigma_a_1g=20000.0), rho=0.0177),
     # thin medium: mfp ~ 0.3 m at E0, so census segments carry high-energy deposits
     "tiny_thin": Config("tiny_thin", 64, 64, "uniform", (0.4, 0.4, 0.2, 0.2), 10_000, 15, _SINGLE, rho=0.02),
+    # heterogeneous maps exercising the u16 and f64 density layouts
+    "tiny_levels": Config("tiny_levels", 64, 64, "levels", (0.3, 0.3, 0.4, 0.4), 3000, 16, _SINGLE, rho=2.0),
+    "small_random": Config("small_random", 300, 300, "random", (0.3, 0.3, 0.4, 0.4), 3000, 17, rho=2.0),
     "tiny_stream": Config("tiny_stream", 64, 64, "uniform_lo", (0.45, 0.45, 0.1, 0.1), 2000, 8),
     "tiny_split": Config("tiny_split", 64, 64, "split", (0.0, 0.0, 1.0, 1.0), 2000, 9),
     "small_csp": Config("small_csp", 256, 256, "csp", (0.0, 0.0, 0.1, 0.1), 4096, 10),
@@ -120,6 +123,12 @@ def density(cfg: Config) -> np.ndarray:
         return np.full((ny, nx), RHO_HI)
     if cfg.density == "uniform":
         return np.full((ny, nx), cfg.rho)
+    if cfg.density == "levels":      # 1000 distinct levels in [0, rho]: u16 material codes
+        rng = np.random.default_rng(cfg.seed)
+        return rng.integers(0, 1000, (ny, nx)) * (cfg.rho / 1000.0)
+    if cfg.density == "random":      # continuous random densities: no lossless code fits
+        rng = np.random.default_rng(cfg.seed)
+        return rng.uniform(0.0, cfg.rho, (ny, nx))
     if cfg.density == "csp":
         inx = (xc >= 0.25 * cfg.width) & (xc <= 0.75 * cfg.width)
         iny = (yc >= 0.25 * cfg.height) & (yc <= 0.75 * cfg.height)

@@ -103,7 +103,8 @@ def test_inject_matches_oracle(nt, orc, cfgname):
 
 # ---------------------------------------------------------------------------------------------
 TINY = ["tiny_csp", "tiny_stream", "tiny_split", "tiny_vacuum", "tiny_vacuum_lo", "tiny_scatter_1g",
-        "tiny_wkill", "tiny_A12", "tiny_mid", "tiny_thin", "tiny_absorber", "small_csp", "small_scatter"]
+        "tiny_wkill", "tiny_A12", "tiny_mid", "tiny_thin", "tiny_absorber", "small_csp", "small_scatter",
+        "tiny_levels", "small_random"]
 
 
 @pytest.mark.parametrize("mode", MODES)
@@ -120,10 +121,11 @@ def test_parity_deterministic(nt, orc, cfgname, mode):
 
 
 @pytest.mark.parametrize("mode", MODES)
-@pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_split", "tiny_mid", "small_scatter"])
-def test_parity_production_atomic(nt, orc, cfgname, mode):
+@pytest.mark.parametrize("density_format", [0, 1])
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_split", "tiny_mid", "small_scatter", "tiny_levels"])
+def test_parity_production_atomic(nt, orc, cfgname, mode, density_format):
     cfg = wl.CONFIGS[cfgname]
-    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode)
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, density_format=density_format)
     ot, op, (os_,) = orc.run(cfg)
     compare_particles(gp, op)                  # per-particle results do not depend on the tally
     compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
@@ -255,7 +257,7 @@ def _sample_ids(n, k=48):
 @pytest.mark.parametrize("cfgname", SCALE)
 def test_scale_sampled_parity_and_properties(nt, orc, cfgname, mode):
     cfg = wl.CONFIGS[cfgname]
-    t = nt.setup(cfg, mode=mode)
+    t = nt.setup(cfg, mode=mode)      # bench.py's launch configuration (defaults)
     s = t.run_timestep(cfg.dt)
     tally = t.read_tally()
     g = t.read_particles()
