@@ -559,7 +559,20 @@ static nt_status det_snapshot(nt_ctx* c, int64_t lo, int64_t nb, bool restore) {
   return NT_OK;
 }
 
-static nt_status run_det_history(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
+// Track one batch [bp.lo, bp.hi) in the context's mode (history kernel or event loop).
+static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_t& launches) {
+  if (c->opt.mode == NT_MODE_EVENT) {
+    if (!c->evs) c->evs = event_state_create();
+    if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
+    return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
+  }
+  launch_history(bp, det, history_grid(c, det), det ? 3 : history_min_blocks(c), c->stream);
+  ++launches;
+  NT_CUDA(c, cudaGetLastError());
+  return NT_OK;
+}
+
+static nt_status run_det(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
   int cell_bits = 0;
   while ((1ull << cell_bits) < (unsigned long long)c->nx * (unsigned long long)c->ny) ++cell_bits;
   if (cell_bits > 24)
@@ -567,7 +580,6 @@ static nt_status run_det_history(nt_ctx* c, const TrackParams& tp, uint32_t& lau
   if (c->rec_cap == 0) c->rec_cap = 1ull << 20;
   const unsigned long long kMaxCap = 1ull << 27;
   int64_t batch = c->opt.det_batch;
-  const int grid = history_grid(c, true);
   unsigned long long* rec_count = reinterpret_cast<unsigned long long*>(c->scratch.as<char>() + 8);
   int64_t lo = 0;
   while (lo < c->n_local) {
@@ -588,9 +600,8 @@ static nt_status run_det_history(nt_ctx* c, const TrackParams& tp, uint32_t& lau
     bp.rec_cap = c->rec_cap;
     bp.rec_count = rec_count;
     NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 16, c->stream));   // work counter, records
-    launch_history(bp, true, grid, 3, c->stream);
-    ++launches;
-    NT_CUDA(c, cudaGetLastError());
+    st = track_range(c, bp, true, launches);
+    if (st != NT_OK) return st;
     unsigned long long nrec = 0;
     NT_CUDA(c, cudaMemcpyAsync(&nrec, rec_count, 8, cudaMemcpyDeviceToHost, c->stream));
     NT_CUDA(c, cudaStreamSynchronize(c->stream));
@@ -638,18 +649,9 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 1024, c->stream));
   NT_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
   const TrackParams tp = make_params(c, dt);
-  if (c->opt.mode == NT_MODE_EVENT) {
-    if (!c->evs) c->evs = event_state_create();
-    if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
-    const nt_status st = event_run_timestep(c->evs, tp, det, c->sm_count, c->stream, launches, c->err);
+  {
+    const nt_status st = det ? run_det(c, tp, launches) : track_range(c, tp, false, launches);
     if (st != NT_OK) return st;
-  } else if (det) {
-    const nt_status st = run_det_history(c, tp, launches);
-    if (st != NT_OK) return st;
-  } else {
-    launch_history(tp, false, history_grid(c, false), history_min_blocks(c), c->stream);
-    ++launches;
-    NT_CUDA(c, cudaGetLastError());
   }
   NT_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
   // stats: u64 slots then f64 slots, reduced over ranks as doubles (counts < 2^53 exact)

@@ -11,8 +11,12 @@ namespace nt {
 struct EventState;
 EventState* event_state_create();
 void event_state_destroy(EventState* s);
-void event_state_invalidate(EventState* s);   // particles re-injected: drop cached buffers
-nt_status event_run_timestep(EventState* s, const TrackParams& tp, bool det, int sm_count,
-                             cudaStream_t stream, uint32_t& launches, std::string& err);
+void event_state_invalidate(EventState* s);
+// Track local particles [tp.lo, tp.hi) for one timestep with the event queues; adds the
+// range's statistics into tp.stats_*.  Deterministic mode (det) writes flush records.
+nt_status event_run_range(EventState* s, const TrackParams& tp, bool det, int sm_count,
+                          cudaStream_t stream, uint32_t& launches, std::string& err);
+// Iterations the device loop ran for the last range (synchronises the stream).
+unsigned event_iterations(EventState* s, cudaStream_t stream);
 
 }  // namespace nt

@@ -16,7 +16,7 @@ from tests.parity import compare_particles, compare_stats, compare_tally
 
 pytestmark = pytest.mark.gpu
 
-MODES = ["history"]
+MODES = ["history", "event"]
 
 
 @pytest.fixture(scope="module")
