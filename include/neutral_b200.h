@@ -61,8 +61,11 @@ typedef struct {
     int32_t deterministic;     /* 1: fixed-order tally = the oracle's (particle id, flush
                                   sequence) order per cell; 0: fp64 atomics   */
     int32_t rank, nranks;      /* this process's rank and the world size (0, 1 = 1 GPU)   */
-    const void *nccl_unique_id;/* 128-byte ncclUniqueId when nranks > 1 (nt_get_unique_id
-                                  on rank 0, broadcast by the caller)                     */
+    const void *nccl_unique_id;/* 128-byte ncclUniqueId (nt_get_unique_id on rank 0,
+                                  broadcast by the caller); required when nranks > 1.  When
+                                  given, the context joins that NCCL communicator and every
+                                  timestep allreduces the tally and statistics (also for
+                                  nranks == 1, which exercises the same path on one GPU)  */
     double A;                  /* target mass / neutron mass       (0 -> 1.0)            */
     double molar_mass;         /* kg/mol                           (0 -> 1e-3)           */
     double e_min;              /* energy cutoff, eV    (0 -> 1.0)            */
@@ -72,7 +75,7 @@ typedef struct {
     int32_t ctas_per_sm;       /* persistent CTAs per SM (0 -> occupancy maximum)         */
     int64_t det_batch;         /* deterministic mode: particles per batch (0 -> 65536)    */
     int32_t refill_min;        /* history mode: a warp refills its idle lanes once at least
-                                  this many are idle (0 -> 1)                              */
+                                  this many are idle (0 -> 8)                              */
     int32_t density_format;    /* 0: lossless u8/u16 material codes when the density map
                                   holds <= 256 / 65536 distinct values, else f64;
                                   1: always the f64 map                                    */

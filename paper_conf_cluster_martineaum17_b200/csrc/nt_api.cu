@@ -8,6 +8,7 @@
 #include <cmath>
 #include <cstdarg>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <string>
 #include <vector>
@@ -70,8 +71,8 @@ struct nt_ctx {
   uint64_t seed = 0;
   DevBuf soa;
   Soa p{};
-  // step scratch: [counter][stats_u][stats_f]
-  DevBuf scratch;
+  // step scratch: [counter][stats_u][stats_f]; per-thread f64 statistic slots
+  DevBuf scratch, slots;
   // deterministic mode
   DevBuf rec_key, rec_val, rec_key2, rec_val2, sort_tmp, backup;
   unsigned long long rec_cap = 0;
@@ -181,7 +182,7 @@ nt_status nt_options_default(nt_options* opt) {
   opt->w_min = 1.0e-3;
   opt->max_events_per_history = 1000000000ll;
   opt->det_batch = 65536;
-  opt->refill_min = 1;
+  opt->refill_min = 8;
   return NT_OK;
 }
 
@@ -241,7 +242,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   }
   for (auto& ev : c->ev) cudaEventCreate(&ev);
   init_phys(c);
-  if (opt.nranks > 1) {
+  if (opt.nranks > 1 || opt.nccl_unique_id) {
     ncclUniqueId id;
     std::memcpy(&id, opt.nccl_unique_id, sizeof id);
     ncclResult_t r = ncclCommInitRank(&c->comm, opt.nranks, id, opt.rank);
@@ -260,7 +261,7 @@ nt_status nt_destroy(nt_ctx* c) {
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
   for (DevBuf* b : {&c->rho_code, &c->nd_tab, &c->enc_keys, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
-                    &c->scratch, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
+                    &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup})
     b->release();
   for (auto& ev : c->ev)
@@ -513,11 +514,16 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.seed = c->seed;
   tp.dt = dt;
   tp.max_events = c->opt.max_events_per_history;
-  tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 1;
+  tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 8;
+  {
+    const char* d = std::getenv("NT_DIAG");   // diagnostics experiments only (wrong results)
+    tp.diag = d ? std::atoi(d) : 0;
+  }
   char* s = c->scratch.as<char>();
   tp.counter = reinterpret_cast<unsigned long long*>(s);
   tp.stats_u = reinterpret_cast<unsigned long long*>(s + 256);
   tp.stats_f = reinterpret_cast<double*>(s + 512);
+  tp.slot_f = c->slots.as<double>();
   return tp;
 }
 
@@ -640,6 +646,8 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   if (c->stage < ST_PARTICLES) return fail(c, NT_ERR_STATE, "nt_inject_particles must come first");
   if (!(dt > 0.0) || !is_fin(dt)) return fail(c, NT_ERR_ARG, "dt must be finite and > 0");
   NT_CUDA(c, c->scratch.ensure(1024));
+  // per-thread statistic slots for the largest persistent grid (8 CTAs of 256 per SM)
+  NT_CUDA(c, c->slots.ensure((size_t)c->sm_count * 8 * kHistoryBlock * SF_COUNT * 8));
   const size_t cells = (size_t)c->nx * (size_t)c->ny;
   uint32_t launches = 0;
   const bool det = c->opt.deterministic != 0;

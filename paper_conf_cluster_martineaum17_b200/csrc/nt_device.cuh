@@ -142,6 +142,38 @@ __device__ __forceinline__ double number_density(const Mesh& M, const double* __
   }
 }
 
+// Split form of number_density for latency hiding: dens_load issues the gather (raw code or
+// raw density), dens_nd consumes it later -- the history kernel issues the load at a facet
+// and consumes it at the start of the next event, so the gather overlaps the loop overhead.
+template <int kFmt> struct DensRaw { using type = uint32_t; };
+template <> struct DensRaw<kDensF64> { using type = double; };
+
+template <int kFmt>
+__device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M, int64_t cell) {
+  if constexpr (kFmt == kDensU8) return (uint32_t)__ldg(M.rho8 + cell);
+  else if constexpr (kFmt == kDensU16) return (uint32_t)__ldg(M.rho16 + cell);
+  else return __ldg(M.rho + cell);
+}
+
+__device__ __forceinline__ void prefetch_l1(const void* p) {
+  asm volatile("prefetch.global.L1 [%0];" ::"l"(p));
+}
+
+template <int kFmt>
+__device__ __forceinline__ void dens_prefetch(const Mesh& M, int64_t cell) {
+  if constexpr (kFmt == kDensU8) prefetch_l1(M.rho8 + cell);
+  else if constexpr (kFmt == kDensU16) prefetch_l1(M.rho16 + cell);
+  else prefetch_l1(M.rho + cell);
+}
+
+template <int kFmt>
+__device__ __forceinline__ double dens_nd(typename DensRaw<kFmt>::type raw,
+                                          const double* __restrict__ tab, double cn) {
+  if constexpr (kFmt == kDensU8) return tab[raw];
+  else if constexpr (kFmt == kDensU16) return __ldg(tab + raw);
+  else return raw * cn;
+}
+
 // ---- microscopic cross sections -----------------------------------------------
 // Bin i = max{i in [0,N-2]: k[i] <= e} for e already in [k0, k_{N-1}] (the energy-bin
 // search), then linear interpolation.  The bucket index narrows the binary search to a

@@ -20,9 +20,12 @@ struct TrackParams {
   double dt;
   int64_t max_events;
   int32_t refill_min;         // refill a warp's idle lanes once at least this many are idle
+  int32_t diag;               // diagnostics only (env NT_DIAG): 1 skip RED, 2 skip density
+                              // gather, 4 skip edge gather -- results are then WRONG
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]
+  double* slot_f;                   // [SF_COUNT][grid * block] per-thread f64 statistic slots
   // deterministic-mode flush records (cell << 40 | (pid - lo) << 24 | seq, value)
   unsigned long long* rec_key;
   double* rec_val;

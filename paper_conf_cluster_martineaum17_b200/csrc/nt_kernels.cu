@@ -82,18 +82,28 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 template <bool kDet, int kMinBlocks, int kFmt>
 __global__ void __launch_bounds__(kHistoryBlock, kMinBlocks)
 history_kernel(const __grid_constant__ TrackParams P) {
-  __shared__ uint32_t s_u[SU_COUNT][kHistoryBlock];
-  __shared__ double s_f[SF_COUNT][kHistoryBlock];
+  // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
+  // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
+  // almost no shared memory and the L1 stays free for the density / edge gathers.
+  constexpr int kWarps = kHistoryBlock / 32;
+  __shared__ uint32_t s_u[kWarps][SU_COUNT];
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
   const int t = threadIdx.x;
+  const int64_t gt = (int64_t)blockIdx.x * kHistoryBlock + t;
+  const int64_t sstride = (int64_t)gridDim.x * kHistoryBlock;
+  double* __restrict__ sf = P.slot_f + gt;          // sf[k * sstride]: statistic k
 #pragma unroll
-  for (int k = 0; k < SU_COUNT; ++k) s_u[k][t] = 0u;
-#pragma unroll
-  for (int k = 0; k < SF_COUNT; ++k) s_f[k][t] = 0.0;
+  for (int k = 0; k < SF_COUNT; ++k) sf[k * sstride] = 0.0;
+  if (t < kWarps * SU_COUNT) (&s_u[0][0])[t] = 0u;
+  __syncthreads();
   if constexpr (kFmt == kDensU8) {
     for (int k = t; k < 256; k += kHistoryBlock) s_nd[k] = k < P.mesh.ncodes ? P.mesh.nd_tab[k] : 0.0;
     __syncthreads();
   }
+  const int wid = t >> 5;
+  auto cnt = [&](int k, uint32_t v) { atomicAdd(&s_u[wid][k], v); };
+  auto fsum = [&](int k, double v) { sf[k * sstride] += v; };
+  double wabs = 0.0;   // weight absorbed by implicit capture, this thread
   const double* __restrict__ ndtab = (kFmt == kDensU8) ? s_nd : P.mesh.nd_tab;
 
   const int lane = t & 31;
@@ -104,13 +114,16 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
   const Phys& ph = P.ph;
   const int refill_min = P.refill_min;
+  const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
 
   bool active = false, exhausted = false;
   int32_t i = 0;                 // local particle index (< 2^31)
   // register-resident history state
   double x = 0, y = 0, ox = 0, oy = 0, iox = 0, ioy = 0, e = 0, w = 0, mfp = 0, dcen = 0;
-  double nd = 0;      // number density of the current cell: Sigma_t = nd * st
+  typename DensRaw<kFmt>::type draw = 0;  // density (code) of the current cell, as loaded
   double exn = 0, eyn = 0;  // edge each axis is heading to (facet distance, snap value)
+  double enext = 0;         // edge loaded at the last facet, for axis eax (2 = none pending)
+  int eax = 2;
   double acc = 0;     // deposit accumulated in the current cell
   double dstep = 0;   // deposits this particle flushed this step
   Mat m{0, 0, 0};
@@ -142,9 +155,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
             cx = P.p.cx[i];
             cy = P.p.cy[i];
             ctr = P.p.ctr[i];
-            nd = number_density<kFmt>(P.mesh, ndtab, (int64_t)cy * nx + cx, ph.cn);
+            draw = dens_load<kFmt>(P.mesh, (int64_t)cy * nx + cx);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
+            eax = 2;
             m = refresh_xs(P.xs, ph, e, nrange);
             dcen = speed(e, ph) * P.dt;
             iox = 1.0 / ox;
@@ -154,7 +168,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
             nf = 0u;
             nc = 0u;
             seq = 0u;
-            s_u[SU_ALIVE][t] += 1u;
+            cnt(SU_ALIVE, 1u);
           }
         }
       }
@@ -163,178 +177,185 @@ history_kernel(const __grid_constant__ TrackParams P) {
       if (exhausted) break;
       continue;
     }
-    if (!active) continue;
 
-    // ---- one event (Listing 1) ----
-    const double sig = nd * m.st;
-    double tx = (exn - x) * iox;
-    tx = tx < 0.0 ? 0.0 : tx;
-    tx = ox != 0.0 ? tx : d_inf();
-    double ty = (eyn - y) * ioy;
-    ty = ty < 0.0 ? 0.0 : ty;
-    ty = oy != 0.0 ? ty : d_inf();
-    const bool ax = tx < ty;
-    const double df = ax ? tx : ty;
-    const double dc = sig > 0.0 ? mfp / sig : d_inf();
-    const double ds = dcen;
-    int outcome = 0;                      // 0 continue, 1 census, 2 dead
+    // ---- events until enough lanes are idle to refill (or none is active) ----
+    for (;;) {
+      if (active) {
+        // ---- one event (Listing 1) ----
+        // consume the gathers issued by the previous facet (density code, next edge)
+        const double nd = dens_nd<kFmt>(draw, ndtab, ph.cn);
+        exn = eax == 0 ? enext : exn;
+        eyn = eax == 1 ? enext : eyn;
+        eax = 2;
+        const double sig = nd * m.st;
+        // clamp at 0 with fmax: differs from "t < 0 ? 0 : t" only in the sign of a zero and
+        // for NaN, neither of which can change any result
+        const double tx = ox != 0.0 ? fmax((exn - x) * iox, 0.0) : d_inf();
+        const double ty = oy != 0.0 ? fmax((eyn - y) * ioy, 0.0) : d_inf();
+        const bool ax = tx < ty;
+        const double df = ax ? tx : ty;
+        const double dc = sig > 0.0 ? mfp / sig : d_inf();
+        const double ds = dcen;
+        int outcome = 0;                      // 0 continue, 1 census, 2 dead
 
-    auto flush = [&]() {
-      const int64_t cell = (int64_t)cy * nx + cx;
-      if constexpr (kDet) {
-        const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
-        if (slot < P.rec_cap) {
-          P.rec_key[slot] = ((unsigned long long)cell << 40) |
-                            ((unsigned long long)((int64_t)i - P.lo) << 24) |
-                            (unsigned long long)(seq & 0xffffffu);
-          P.rec_val[slot] = acc;
+        auto flush = [&]() {
+          const int64_t cell = (int64_t)cy * nx + cx;
+          if constexpr (kDet) {
+            const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
+            if (slot < P.rec_cap) {
+              P.rec_key[slot] = ((unsigned long long)cell << 40) |
+                                ((unsigned long long)((int64_t)i - P.lo) << 24) |
+                                (unsigned long long)(seq & 0xffffffu);
+              P.rec_val[slot] = acc;
+            }
+            if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
+            ++seq;
+          } else {
+            if (!(P.diag & 1)) atomicAdd(P.mesh.tally + cell, acc);  // fire-and-forget fp64 RED at L2
+          }
+          dstep += acc;
+          acc = 0.0;
+        };
+
+        if (nf + nc >= max_ev) {
+          // guard (R27): count, flush, kill
+          cnt(SU_EVENT_CAP, 1u);
+          flush();
+          cnt(SU_KILLED, 1u);
+          fsum(SF_KILLED_E, w * e);
+          fsum(SF_KILLED_W, w);
+          outcome = 2;
+        } else if (dc < df && dc < ds) {
+          // ---- collision (implicit capture + elastic scatter) ----
+          acc += ((w * dc) * sig) * m.H;
+          x = x + dc * ox;
+          y = y + dc * oy;
+          dcen = dcen - dc;
+          const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+          ctr += 1u;
+          nc += 1u;
+          const double w_old = w;
+          w = w * (1.0 - m.pa);
+          wabs += w_old - w;
+          const double mu = 1.0 - 2.0 * u01(r.a);
+          const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
+          const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
+          const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
+          const double q = 1.0 - ct * ct;
+          const double stt = sgn * sqrt(q > 0.0 ? q : 0.0);
+          const double nox = ox * ct - oy * stt;
+          const double noy = ox * stt + oy * ct;
+          ox = nox;
+          oy = noy;
+          const double tcen = dcen / speed(e, ph);
+          e = e2;
+          if (e < ph.e_min || w < ph.w_min) {
+            flush();
+            fsum(SF_KILLED_E, w * e);
+            fsum(SF_KILLED_W, w);
+            cnt(SU_KILLED, 1u);
+            outcome = 2;
+          } else {
+            exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
+            eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
+            dcen = tcen * speed(e, ph);
+            m = refresh_xs(P.xs, ph, e, nrange);
+            iox = 1.0 / ox;
+            ioy = 1.0 / oy;
+            mfp = -log(u01(r.b));
+          }
+        } else if (df < ds) {
+          // ---- facet: one code path for both axes (no X/Y divergence) ----
+          acc += ((w * df) * sig) * m.H;
+          mfp = fmax(mfp - df * sig, 0.0);
+          dcen = dcen - df;
+          const double xm = x + df * ox, ym = y + df * oy;
+          x = ax ? exn : xm;                          // snap the crossed coordinate
+          y = ax ? ym : eyn;
+          flush();                                    // deposit of the cell being left
+          const int32_t c = ax ? cx : cy;
+          const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
+          const int32_t last = (ax ? nx : ny) - 1;
+          const bool refl = pos ? (c == last) : (c == 0);   // reflective boundary
+          const int32_t c2 = refl ? c : (pos ? c + 1 : c - 1);
+          cx = ax ? c2 : cx;
+          cy = ax ? cy : c2;
+          if (refl) {                               // rare: a branch beats 8 selects
+            if (ax) { ox = -ox; iox = -iox; } else { oy = -oy; ioy = -ioy; }
+          }
+          // next edge on the crossed axis and the new cell's density: two independent loads
+          const bool pos2 = refl ? !pos : pos;
+          const double ev = (P.diag & 4) ? (ax ? exn : eyn) + 0.000244140625 * (pos2 ? 1.0 : -1.0) * (refl ? 0.0 : 1.0)
+                                         : __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
+          if (!(P.diag & 2)) draw = dens_load<kFmt>(P.mesh, (int64_t)cy * nx + cx);
+          enext = ev;
+          eax = ax ? 0 : 1;
+          nf += 1u;
+        } else {
+          // ---- census ----
+          acc += ((w * ds) * sig) * m.H;
+          x = x + ds * ox;
+          y = y + ds * oy;
+          const double nm = mfp - ds * sig;
+          mfp = nm > 0.0 ? nm : 0.0;
+          flush();
+          cnt(SU_CENSUS, 1u);
+          fsum(SF_CENSUS_E, w * e);
+          fsum(SF_CENSUS_W, w);
+          outcome = 1;
         }
-        if (seq >= (1u << 24)) s_u[SU_REC_OVERFLOW][t] += 1u;
-        ++seq;
-      } else {
-        atomicAdd(P.mesh.tally + cell, acc);      // fire-and-forget fp64 RED at L2
-      }
-      dstep += acc;
-      acc = 0.0;
-    };
 
-    if ((int64_t)(nf + nc) >= P.max_events) {
-      // guard (R27): count, flush, kill
-      s_u[SU_EVENT_CAP][t] += 1u;
-      flush();
-      s_u[SU_KILLED][t] += 1u;
-      s_f[SF_KILLED_E][t] += w * e;
-      s_f[SF_KILLED_W][t] += w;
-      outcome = 2;
-    } else if (dc < df && dc < ds) {
-      // ---- collision (implicit capture + elastic scatter) ----
-      acc += ((w * dc) * sig) * m.H;
-      x = x + dc * ox;
-      y = y + dc * oy;
-      dcen = dcen - dc;
-      const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
-      ctr += 1u;
-      nc += 1u;
-      const double w_old = w;
-      w = w * (1.0 - m.pa);
-      s_f[SF_ABSORBED_W][t] += w_old - w;
-      const double mu = 1.0 - 2.0 * u01(r.a);
-      const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
-      const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
-      const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
-      const double q = 1.0 - ct * ct;
-      const double stt = sgn * sqrt(q > 0.0 ? q : 0.0);
-      const double nox = ox * ct - oy * stt;
-      const double noy = ox * stt + oy * ct;
-      ox = nox;
-      oy = noy;
-      const double tcen = dcen / speed(e, ph);
-      e = e2;
-      if (e < ph.e_min || w < ph.w_min) {
-        flush();
-        s_f[SF_KILLED_E][t] += w * e;
-        s_f[SF_KILLED_W][t] += w;
-        s_u[SU_KILLED][t] += 1u;
-        outcome = 2;
-      } else {
-        exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
-        eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
-        dcen = tcen * speed(e, ph);
-        m = refresh_xs(P.xs, ph, e, nrange);
-        iox = 1.0 / ox;
-        ioy = 1.0 / oy;
-        mfp = -log(u01(r.b));
+        if (outcome != 0) {
+          if (!(isfinite(x) && isfinite(y) && isfinite(e) && isfinite(w)))
+            cnt(SU_NONFINITE, 1u);
+          P.p.x[i] = x;
+          P.p.y[i] = y;
+          P.p.ox[i] = ox;
+          P.p.oy[i] = oy;
+          P.p.e[i] = e;
+          P.p.w[i] = w;
+          P.p.mfp[i] = mfp;
+          P.p.dep[i] += dstep;
+          P.p.cx[i] = cx;
+          P.p.cy[i] = cy;
+          P.p.ctr[i] = ctr;
+          P.p.nfac[i] += nf;
+          P.p.ncol[i] += nc;
+          if (outcome == 1) {
+            P.p.ncen[i] += 1u;
+          } else {
+            P.p.status[i] = 0u;
+          }
+          cnt(SU_FACETS, nf);
+          cnt(SU_COLLISIONS, nc);
+          fsum(SF_TALLY, dstep);
+          active = false;
+        }
       }
-    } else if (df < ds) {
-      // ---- facet: one code path for both axes (no X/Y divergence) ----
-      acc += ((w * df) * sig) * m.H;
-      const double nm = mfp - df * sig;
-      mfp = nm > 0.0 ? nm : 0.0;
-      dcen = dcen - df;
-      const double xm = x + df * ox, ym = y + df * oy;
-      x = ax ? exn : xm;                          // snap the crossed coordinate
-      y = ax ? ym : eyn;
-      flush();                                    // deposit of the cell being left
-      const int32_t c = ax ? cx : cy;
-      const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
-      const int32_t last = (ax ? nx : ny) - 1;
-      const bool refl = pos ? (c == last) : (c == 0);   // reflective boundary
-      const int32_t c2 = refl ? c : (pos ? c + 1 : c - 1);
-      cx = ax ? c2 : cx;
-      cy = ax ? cy : c2;
-      const bool fx = refl && ax, fy = refl && !ax;
-      ox = fx ? -ox : ox;
-      iox = fx ? -iox : iox;
-      oy = fy ? -oy : oy;
-      ioy = fy ? -ioy : ioy;
-      // next edge on the crossed axis and the new cell's density: two independent loads
-      const bool pos2 = refl ? !pos : pos;
-      const double ev = __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
-      nd = number_density<kFmt>(P.mesh, ndtab, (int64_t)cy * nx + cx, ph.cn);
-      exn = ax ? ev : exn;
-      eyn = ax ? eyn : ev;
-      nf += 1u;
-    } else {
-      // ---- census ----
-      acc += ((w * ds) * sig) * m.H;
-      x = x + ds * ox;
-      y = y + ds * oy;
-      const double nm = mfp - ds * sig;
-      mfp = nm > 0.0 ? nm : 0.0;
-      flush();
-      s_u[SU_CENSUS][t] += 1u;
-      s_f[SF_CENSUS_E][t] += w * e;
-      s_f[SF_CENSUS_W][t] += w;
-      outcome = 1;
-    }
-
-    if (outcome != 0) {
-      if (!(isfinite(x) && isfinite(y) && isfinite(e) && isfinite(w)))
-        s_u[SU_NONFINITE][t] += 1u;
-      P.p.x[i] = x;
-      P.p.y[i] = y;
-      P.p.ox[i] = ox;
-      P.p.oy[i] = oy;
-      P.p.e[i] = e;
-      P.p.w[i] = w;
-      P.p.mfp[i] = mfp;
-      P.p.dep[i] += dstep;
-      P.p.cx[i] = cx;
-      P.p.cy[i] = cy;
-      P.p.ctr[i] = ctr;
-      P.p.nfac[i] += nf;
-      P.p.ncol[i] += nc;
-      if (outcome == 1) {
-        P.p.ncen[i] += 1u;
-      } else {
-        P.p.status[i] = 0u;
-      }
-      s_u[SU_FACETS][t] += nf;
-      s_u[SU_COLLISIONS][t] += nc;
-      s_f[SF_TALLY][t] += dstep;
-      active = false;
+      const unsigned idle_now = __ballot_sync(kFull, !active);
+      if (idle_now == kFull || (!exhausted && __popc(idle_now) >= refill_min)) break;
     }
   }
 
-  // ---- CTA reduction of the per-thread statistics, one atomic per statistic ----
-  s_u[SU_XS_RANGE][t] += nrange;
+  // ---- CTA reduction of the statistics, one atomic per statistic per CTA ----
+  if (nrange) cnt(SU_XS_RANGE, nrange);
+  fsum(SF_ABSORBED_W, wabs);
   __syncthreads();
-  const int warp = t >> 5;
-  constexpr int kWarps = kHistoryBlock / 32;
-  for (int k = warp; k < SU_COUNT + SF_COUNT; k += kWarps) {
+  const int lane2 = t & 31;
+  for (int k = wid; k < SU_COUNT + SF_COUNT; k += kWarps) {
     if (k < SU_COUNT) {
-      unsigned long long v = 0;
-      for (int j = lane; j < kHistoryBlock; j += 32) v += s_u[k][j];
+      unsigned long long v = lane2 < kWarps ? s_u[lane2][k] : 0u;
 #pragma unroll
       for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(kFull, v, o);
-      if (lane == 0 && v != 0) atomicAdd(P.stats_u + k, v);
+      if (lane2 == 0 && v != 0) atomicAdd(P.stats_u + k, v);
     } else {
       const int kf = k - SU_COUNT;
       double v = 0.0;
-      for (int j = lane; j < kHistoryBlock; j += 32) v += s_f[kf][j];
+      for (int j = lane2; j < kHistoryBlock; j += 32)
+        v += P.slot_f[(int64_t)blockIdx.x * kHistoryBlock + j + kf * sstride];
 #pragma unroll
       for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(kFull, v, o);
-      if (lane == 0 && v != 0.0) atomicAdd(P.stats_f + kf, v);
+      if (lane2 == 0 && v != 0.0) atomicAdd(P.stats_f + kf, v);
     }
   }
 }

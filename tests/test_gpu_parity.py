@@ -297,3 +297,21 @@ def test_scale_deterministic_subrange(nt, orc, mode):
     rep = compare_tally(gt, ot)
     compare_stats(gs, os_)
     print(rep)
+
+
+@pytest.mark.parametrize("mode", MODES)
+def test_nccl_allreduce_path_single_rank(nt, orc, mode):
+    """The NCCL tally/stats allreduce path (nranks > 1 in production), on a 1-rank
+    communicator: the reduced tally equals the local tally and the oracle's."""
+    cfg = wl.CONFIGS["tiny_csp"]
+    uid = nt.get_unique_id()
+    t = nt.setup(cfg, mode=mode, deterministic=True, rank=0, nranks=1, unique_id=uid)
+    s = t.run_timestep(cfg.dt)
+    red = t.read_tally(reduced=True)
+    loc = t.read_tally(reduced=False)
+    t.close()
+    ot, _, (os_,) = orc.run(cfg)
+    assert np.array_equal(red, loc)
+    compare_tally(red, ot)
+    compare_stats(s, os_)
+    assert s["reduce_ms"] > 0.0
