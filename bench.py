@@ -172,7 +172,9 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--ctas-per-sm", type=int, default=0)
     ap.add_argument("--refill-min", type=int, default=0)
+    ap.add_argument("--layout", type=int, default=0, help="0 tiled 4x4 (default), 1 row-major")
     ap.add_argument("--json-out", default=None)
+    ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
     return ap.parse_args()
 
 
@@ -233,6 +235,8 @@ def main():
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     torch.cuda.set_device(local)
     cfg = wl.CONFIGS[a.config]
+    if a.mesh:
+        cfg = cfg.with_(nx=a.mesh, ny=a.mesh, name=f"{cfg.name}@{a.mesh}")
     n_per = cfg.n_particles
     n_total = n_per * world
     first_id = rank * n_per
@@ -245,7 +249,7 @@ def main():
     tr = binding.Tracker(device=local, stream=stream.cuda_stream, mode=a.mode, rank=rank,
                          nranks=world, unique_id=uid, A=cfg.A, molar_mass=cfg.molar_mass,
                          e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm,
-                         refill_min=a.refill_min)
+                         refill_min=a.refill_min, layout=a.layout)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -332,6 +336,7 @@ def main():
             "warmup": a.warmup, "ms_per_step": ms / a.steps, "higher_is_better": True,
             "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
             "config": {"workload": cfg.name, "mode": a.mode, "nx": cfg.nx, "ny": cfg.ny,
+                       "layout": "tiled4x4" if a.layout == 0 else "row-major",
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
                        "tables": [len(tables[0]), len(tables[2])],
                        "parallelism": f"dp{world} (particle id shards, tally NCCL allreduce)",

@@ -79,6 +79,11 @@ typedef struct {
     int32_t density_format;    /* 0: lossless u8/u16 material codes when the density map
                                   holds <= 256 / 65536 distinct values, else f64;
                                   1: always the f64 map                                    */
+    int32_t layout;            /* storage of the tally and density maps: 0: 4x4-cell tiles
+                                  (a tile's 16 f64 tally cells = one 128 B line, so a
+                                  particle's consecutive facets stay in few L2 lines);
+                                  1: row-major.  nt_read_tally always returns row-major.  */
+    int32_t reserved;
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

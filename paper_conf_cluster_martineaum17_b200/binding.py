@@ -40,7 +40,8 @@ class Options(C.Structure):
                 ("e_min", C.c_double), ("w_min", C.c_double),
                 ("max_events_per_history", C.c_int64), ("block_size", C.c_int32),
                 ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64),
-                ("refill_min", C.c_int32), ("density_format", C.c_int32)]
+                ("refill_min", C.c_int32), ("density_format", C.c_int32),
+                ("layout", C.c_int32), ("reserved", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -144,7 +145,7 @@ class Tracker:
                  unique_id: bytes | None = None, A: float = 1.0, molar_mass: float = 1e-3,
                  e_min: float = 1.0, w_min: float = 1e-3, max_events: int = 0,
                  ctas_per_sm: int = 0, det_batch: int = 0, refill_min: int = 0,
-                 density_format: int = 0):
+                 density_format: int = 0, layout: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -161,6 +162,7 @@ class Tracker:
         o.det_batch = det_batch
         o.refill_min = refill_min
         o.density_format = density_format
+        o.layout = layout
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:

@@ -62,7 +62,10 @@ struct nt_ctx {
   double W = 0, H = 0;
   DevBuf rho, tally, tally_local, ex, ey;
   DevBuf rho_code, nd_tab, enc_keys;     // lossless density encoding
+  DevBuf rho_st, tally_rm;               // f64 density in storage layout; row-major staging
   int dens_fmt = kDensF64, dens_codes = 0;
+  int tiled = 0, ntx = 0;                // storage layout of tally / density (cell_index)
+  int64_t cells_st = 0;                  // cells in the storage layout (tiles padded)
   // tables
   DevBuf xs;
   Tables tables{};
@@ -260,7 +263,7 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
-  for (DevBuf* b : {&c->rho_code, &c->nd_tab, &c->enc_keys, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
+  for (DevBuf* b : {&c->rho_code, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup})
     b->release();
@@ -289,8 +292,16 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   if (!density) return fail(c, NT_ERR_ARG, "density is NULL");
   const int64_t cells = (int64_t)nx * (int64_t)ny;
   c->stage = ST_CREATED;
+  const int tiled = c->opt.layout == 0 ? 1 : 0;
+  const int ntx = (nx + 3) / 4, nty = (ny + 3) / 4;
+  const int64_t cells_st = tiled ? (int64_t)ntx * nty * 16 : cells;
+  Mesh ml{};
+  ml.nx = nx;
+  ml.ny = ny;
+  ml.tiled = tiled;
+  ml.ntx = ntx;
   NT_CUDA(c, c->rho.ensure((size_t)cells * 8));
-  NT_CUDA(c, c->tally.ensure((size_t)cells * 8));
+  NT_CUDA(c, c->tally.ensure((size_t)cells_st * 8));
   NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
   NT_CUDA(c, c->ey.ensure(((size_t)ny + 1) * 8));
   NT_CUDA(c, c->scratch.ensure(1024));
@@ -321,17 +332,26 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
     else if (nu <= 65536) fmt = kDensU16;
   }
   if (fmt != kDensF64) {
-    NT_CUDA(c, c->rho_code.ensure((size_t)cells * (fmt == kDensU8 ? 1 : 2)));
+    const size_t cb = (size_t)cells_st * (fmt == kDensU8 ? 1 : 2);
+    NT_CUDA(c, c->rho_code.ensure(cb));
+    NT_CUDA(c, cudaMemsetAsync(c->rho_code.p, 0, cb, c->stream));        // tile padding
     NT_CUDA(c, c->nd_tab.ensure((size_t)nu * 8));
-    NT_CUDA(c, launch_encode(c->rho.as<double>(), cells, c->enc_keys.as<unsigned long long>(), nu,
-                             c->ph.cn, fmt, c->rho_code.p, c->nd_tab.as<double>(), c->stream));
+    NT_CUDA(c, launch_encode(c->rho.as<double>(), cells, ml, c->enc_keys.as<unsigned long long>(),
+                             nu, c->ph.cn, fmt, c->rho_code.p, c->nd_tab.as<double>(), c->stream));
+  } else if (tiled) {
+    NT_CUDA(c, c->rho_st.ensure((size_t)cells_st * 8));
+    NT_CUDA(c, cudaMemsetAsync(c->rho_st.p, 0, (size_t)cells_st * 8, c->stream));
+    NT_CUDA(c, launch_relayout(c->rho.as<double>(), c->rho_st.as<double>(), cells, ml, true, c->stream));
   }
-  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, (size_t)cells * 8, c->stream));
+  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, (size_t)cells_st * 8, c->stream));
   launch_edges(c->ex.as<double>(), nx, width, c->ey.as<double>(), ny, height, c->stream);
   NT_CUDA(c, cudaGetLastError());
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   c->dens_fmt = fmt;
   c->dens_codes = nu;
+  c->tiled = tiled;
+  c->ntx = ntx;
+  c->cells_st = cells_st;
   c->nx = nx;
   c->ny = ny;
   c->W = width;
@@ -493,7 +513,9 @@ nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int6
 // ---- timestep ---------------------------------------------------------------------------
 static TrackParams make_params(nt_ctx* c, double dt) {
   TrackParams tp{};
-  tp.mesh.rho = c->rho.as<double>();
+  tp.mesh.rho = (c->tiled && c->dens_fmt == kDensF64) ? c->rho_st.as<double>() : c->rho.as<double>();
+  tp.mesh.tiled = c->tiled;
+  tp.mesh.ntx = c->ntx;
   tp.mesh.rho8 = c->rho_code.as<uint8_t>();
   tp.mesh.rho16 = c->rho_code.as<uint16_t>();
   tp.mesh.nd_tab = c->nd_tab.as<double>();
@@ -580,7 +602,7 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
 
 static nt_status run_det(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
   int cell_bits = 0;
-  while ((1ull << cell_bits) < (unsigned long long)c->nx * (unsigned long long)c->ny) ++cell_bits;
+  while ((1ull << cell_bits) < (unsigned long long)c->cells_st) ++cell_bits;
   if (cell_bits > 24)
     return fail(c, NT_ERR_UNSUPPORTED, "deterministic mode supports at most 2^24 cells");
   if (c->rec_cap == 0) c->rec_cap = 1ull << 20;
@@ -648,7 +670,7 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   NT_CUDA(c, c->scratch.ensure(1024));
   // per-thread statistic slots for the largest persistent grid (8 CTAs of 256 per SM)
   NT_CUDA(c, c->slots.ensure((size_t)c->sm_count * 8 * kHistoryBlock * SF_COUNT * 8));
-  const size_t cells = (size_t)c->nx * (size_t)c->ny;
+  const size_t cells = (size_t)c->cells_st;   // storage layout (tiles padded with zeros)
   uint32_t launches = 0;
   const bool det = c->opt.deterministic != 0;
 
@@ -736,10 +758,20 @@ nt_status nt_read_tally(nt_ctx* c, double* dst, int32_t reduced) {
   cudaSetDevice(c->device);
   if (c->stage < ST_MESH) return fail(c, NT_ERR_STATE, "no mesh");
   if (!dst) return fail(c, NT_ERR_ARG, "dst is NULL");
-  const size_t cells = (size_t)c->nx * (size_t)c->ny;
-  const void* src = (!reduced && c->comm) ? c->tally_local.p : c->tally.p;
+  const int64_t cells = (int64_t)c->nx * (int64_t)c->ny;
+  const double* src = (!reduced && c->comm) ? c->tally_local.as<double>() : c->tally.as<double>();
   if (!src) return fail(c, NT_ERR_STATE, "no local tally yet");
-  NT_CUDA(c, cudaMemcpyAsync(dst, src, cells * 8, cudaMemcpyDefault, c->stream));
+  if (c->tiled) {            // storage layout -> row-major [ny][nx]
+    NT_CUDA(c, c->tally_rm.ensure((size_t)cells * 8));
+    Mesh ml{};
+    ml.nx = c->nx;
+    ml.ny = c->ny;
+    ml.tiled = 1;
+    ml.ntx = c->ntx;
+    NT_CUDA(c, launch_relayout(src, c->tally_rm.as<double>(), cells, ml, false, c->stream));
+    src = c->tally_rm.as<double>();
+  }
+  NT_CUDA(c, cudaMemcpyAsync(dst, src, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   return NT_OK;
 }

@@ -43,7 +43,18 @@ struct Mesh {
   const double* __restrict__ ey;      // [ny+1]
   int32_t nx, ny;
   int32_t fmt, ncodes;
+  int32_t tiled;                      // 1: 4x4-cell tiles (one 128 B tally line per tile)
+  int32_t ntx;                        // tiles per row = ceil(nx / 4)
 };
+
+// Storage index of cell (cx, cy) in the tally and density arrays.  Tiled layout: 4x4-cell
+// tiles in row-major tile order, row-major inside a tile, so the 16 f64 tally cells of a
+// tile fill one 128 B line and a particle's consecutive facets (x or y) mostly stay in it.
+__device__ __forceinline__ int64_t cell_index(const Mesh& M, int32_t cx, int32_t cy) {
+  if (M.tiled)
+    return ((int64_t)((cy >> 2) * M.ntx + (cx >> 2)) << 4) | (int64_t)(((cy & 3) << 2) | (cx & 3));
+  return (int64_t)cy * M.nx + cx;
+}
 
 // One microscopic cross-section table with its bucket index: bucket b covers the IEEE bit
 // patterns [base + (b << shift), base + ((b+1) << shift)) of positive energies (monotone in

@@ -74,7 +74,7 @@ template <bool kDet>
 __device__ __forceinline__ void ev_flush(const TrackParams& P, const EvCols& C, int32_t i,
                                          int32_t cx, int32_t cy, double& acc, double& dstep,
                                          Acc& a) {
-  const int64_t cell = (int64_t)cy * P.mesh.nx + cx;
+  const int64_t cell = cell_index(P.mesh, cx, cy);
   if constexpr (kDet) {
     const uint32_t seq = C.seq[i];
     const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
@@ -216,7 +216,7 @@ ev_init_kernel(const TrackParams* __restrict__ Pp, EvCols C, unsigned long long*
       uint32_t nrange = 0;
       const Mat m = refresh_xs(P.xs, P.ph, e, nrange);
       a.u[SU_XS_RANGE] += nrange;
-      const double nd = ev_nd<kFmt>(P.mesh, (int64_t)cy * P.mesh.nx + cx, P.ph.cn);
+      const double nd = ev_nd<kFmt>(P.mesh, cell_index(P.mesh, cx, cy), P.ph.cn);
       const double exn = __ldg(P.mesh.ex + cx + (ox > 0.0 ? 1 : 0));
       const double eyn = __ldg(P.mesh.ey + cy + (oy > 0.0 ? 1 : 0));
       const double dcen = speed(e, P.ph) * P.dt;
@@ -437,7 +437,7 @@ ev_step_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, const E
         ioy = fy ? -ioy : ioy;
         const bool pos2 = refl ? !pos : pos;
         const double ev = __ldg((ax ? P.mesh.ex : P.mesh.ey) + (pos2 ? c2 + 1 : c2));
-        nd = ev_nd<kFmt>(P.mesh, (int64_t)cy * nx + cx, ph.cn);
+        nd = ev_nd<kFmt>(P.mesh, cell_index(P.mesh, cx, cy), ph.cn);
         exn = ax ? ev : exn;
         eyn = ax ? eyn : ev;
         C.nf[i] += 1u;

@@ -76,6 +76,10 @@ cudaError_t launch_density_check(const double* rho, int64_t n, unsigned long lon
 cudaError_t density_distinct(const double* rho, int64_t n, unsigned long long* k0,
                              unsigned long long* k1, void* temp, size_t& temp_bytes,
                              int* d_count, cudaStream_t s);
-cudaError_t launch_encode(const double* rho, int64_t n, const unsigned long long* uniq, int nu,
-                          double cn, int fmt, void* code, double* nd_tab, cudaStream_t s);
+cudaError_t launch_encode(const double* rho, int64_t n, const Mesh& M,
+                          const unsigned long long* uniq, int nu, double cn, int fmt, void* code,
+                          double* nd_tab, cudaStream_t s);
+// Row-major [ny][nx] <-> the mesh's storage layout (cell_index).
+cudaError_t launch_relayout(const double* src, double* dst, int64_t n, const Mesh& M,
+                            bool to_storage, cudaStream_t s);
 }  // namespace nt

@@ -155,7 +155,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
             cx = P.p.cx[i];
             cy = P.p.cy[i];
             ctr = P.p.ctr[i];
-            draw = dens_load<kFmt>(P.mesh, (int64_t)cy * nx + cx);
+            draw = dens_load<kFmt>(P.mesh, cell_index(P.mesh, cx, cy));
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             eax = 2;
@@ -199,7 +199,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
 
         auto flush = [&]() {
-          const int64_t cell = (int64_t)cy * nx + cx;
+          const int64_t cell = cell_index(P.mesh, cx, cy);
           if constexpr (kDet) {
             const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
             if (slot < P.rec_cap) {
@@ -287,7 +287,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const bool pos2 = refl ? !pos : pos;
           const double ev = (P.diag & 4) ? (ax ? exn : eyn) + 0.000244140625 * (pos2 ? 1.0 : -1.0) * (refl ? 0.0 : 1.0)
                                          : __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
-          if (!(P.diag & 2)) draw = dens_load<kFmt>(P.mesh, (int64_t)cy * nx + cx);
+          if (!(P.diag & 2)) draw = dens_load<kFmt>(P.mesh, cell_index(P.mesh, cx, cy));
           enext = ev;
           eax = ax ? 0 : 1;
           nf += 1u;

@@ -27,9 +27,10 @@ __global__ void bits_kernel(const double* __restrict__ rho, int64_t n,
     out[i] = (unsigned long long)__double_as_longlong(rho[i]);
 }
 
-// code[i] = index of rho[i]'s bit pattern among the sorted distinct patterns uniq[0..nu)
+// code[cell_index(cx, cy)] = index of rho[cy][cx]'s bit pattern among the sorted distinct
+// patterns uniq[0..nu)  (rho row-major as given; codes in the storage layout)
 template <class T>
-__global__ void encode_kernel(const double* __restrict__ rho, int64_t n,
+__global__ void encode_kernel(const double* __restrict__ rho, int64_t n, Mesh M,
                               const unsigned long long* __restrict__ uniq, int nu,
                               T* __restrict__ code) {
   for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
@@ -40,7 +41,19 @@ __global__ void encode_kernel(const double* __restrict__ rho, int64_t n,
       const int mid = (lo + hi) >> 1;
       if (uniq[mid] <= b) lo = mid; else hi = mid;
     }
-    code[i] = (T)lo;
+    const int32_t cy = (int32_t)(i / M.nx), cx = (int32_t)(i - (int64_t)cy * M.nx);
+    code[cell_index(M, cx, cy)] = (T)lo;
+  }
+}
+
+// Row-major [ny][nx] <-> storage layout (to_storage: gather from rm into st; else back).
+__global__ void relayout_kernel(const double* __restrict__ src, double* __restrict__ dst,
+                                int64_t n, Mesh M, int to_storage) {
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+       i += (int64_t)gridDim.x * blockDim.x) {
+    const int32_t cy = (int32_t)(i / M.nx), cx = (int32_t)(i - (int64_t)cy * M.nx);
+    const int64_t s = cell_index(M, cx, cy);
+    if (to_storage) dst[s] = src[i]; else dst[i] = src[s];
   }
 }
 
@@ -79,13 +92,20 @@ cudaError_t density_distinct(const double* rho, int64_t n, unsigned long long* k
   return cub::DeviceSelect::Unique(temp, temp_bytes, k1, k0, d_count, n, s);
 }
 
-cudaError_t launch_encode(const double* rho, int64_t n, const unsigned long long* uniq, int nu,
-                          double cn, int fmt, void* code, double* nd_tab, cudaStream_t s) {
+cudaError_t launch_encode(const double* rho, int64_t n, const Mesh& M,
+                          const unsigned long long* uniq, int nu, double cn, int fmt, void* code,
+                          double* nd_tab, cudaStream_t s) {
   if (fmt == kDensU8)
-    encode_kernel<uint8_t><<<grid_for(n), 256, 0, s>>>(rho, n, uniq, nu, (uint8_t*)code);
+    encode_kernel<uint8_t><<<grid_for(n), 256, 0, s>>>(rho, n, M, uniq, nu, (uint8_t*)code);
   else
-    encode_kernel<uint16_t><<<grid_for(n), 256, 0, s>>>(rho, n, uniq, nu, (uint16_t*)code);
+    encode_kernel<uint16_t><<<grid_for(n), 256, 0, s>>>(rho, n, M, uniq, nu, (uint16_t*)code);
   nd_table_kernel<<<(nu + 255) / 256, 256, 0, s>>>(uniq, nu, cn, nd_tab);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_relayout(const double* src, double* dst, int64_t n, const Mesh& M,
+                            bool to_storage, cudaStream_t s) {
+  relayout_kernel<<<grid_for(n), 256, 0, s>>>(src, dst, n, M, to_storage ? 1 : 0);
   return cudaGetLastError();
 }
 

@@ -121,11 +121,13 @@ def test_parity_deterministic(nt, orc, cfgname, mode):
 
 
 @pytest.mark.parametrize("mode", MODES)
+@pytest.mark.parametrize("layout", [0, 1])
 @pytest.mark.parametrize("density_format", [0, 1])
 @pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_split", "tiny_mid", "small_scatter", "tiny_levels"])
-def test_parity_production_atomic(nt, orc, cfgname, mode, density_format):
+def test_parity_production_atomic(nt, orc, cfgname, mode, density_format, layout):
     cfg = wl.CONFIGS[cfgname]
-    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, density_format=density_format)
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, density_format=density_format,
+                             layout=layout)
     ot, op, (os_,) = orc.run(cfg)
     compare_particles(gp, op)                  # per-particle results do not depend on the tally
     compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
