@@ -537,10 +537,7 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.dt = dt;
   tp.max_events = c->opt.max_events_per_history;
   tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 8;
-  {
-    const char* d = std::getenv("NT_DIAG");   // diagnostics experiments only (wrong results)
-    tp.diag = d ? std::atoi(d) : 0;
-  }
+
   char* s = c->scratch.as<char>();
   tp.counter = reinterpret_cast<unsigned long long*>(s);
   tp.stats_u = reinterpret_cast<unsigned long long*>(s + 256);
@@ -549,16 +546,11 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   return tp;
 }
 
-// Register budget / CTAs per SM of the production history kernel: ctas_per_sm option
-// (3: <= 80 registers, no spills; 4: <= 64 registers, spills; 0 -> 3), persistent grid =
-// SMs x resident CTAs.
-static int history_min_blocks(nt_ctx* c) {
-  return c->opt.ctas_per_sm >= 4 ? 4 : 3;
-}
-
+// Persistent grid of the history kernel: SMs x resident CTAs (ctas_per_sm caps it).
 static int history_grid(nt_ctx* c, bool det) {
-  int per_sm = history_max_ctas_per_sm(det, det ? 3 : history_min_blocks(c), c->dens_fmt);
+  int per_sm = history_max_ctas_per_sm(det, c->dens_fmt, c->tiled != 0);
   if (per_sm < 1) per_sm = 1;
+  if (c->opt.ctas_per_sm > 0 && c->opt.ctas_per_sm < per_sm) per_sm = c->opt.ctas_per_sm;
   return c->sm_count * per_sm;
 }
 
@@ -594,7 +586,7 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
     if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
     return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
   }
-  launch_history(bp, det, history_grid(c, det), det ? 3 : history_min_blocks(c), c->stream);
+  launch_history(bp, det, history_grid(c, det), c->stream);
   ++launches;
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;

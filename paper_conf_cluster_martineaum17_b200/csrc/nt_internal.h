@@ -20,8 +20,6 @@ struct TrackParams {
   double dt;
   int64_t max_events;
   int32_t refill_min;         // refill a warp's idle lanes once at least this many are idle
-  int32_t diag;               // diagnostics only (env NT_DIAG): 1 skip RED, 2 skip density
-                              // gather, 4 skip edge gather -- results are then WRONG
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]
@@ -49,10 +47,10 @@ void launch_edges(double* ex, int32_t nx, double W, double* ey, int32_t ny, doub
                   cudaStream_t s);
 void launch_inject(const InjectParams& ip, cudaStream_t s);
 // History (Over Particles) tracking: grid = persistent CTAs.
-// min_blocks selects the register budget: 4 -> <= 64 regs (1024 threads/SM), 3 -> <= 80;
-// the density format (tp.mesh.fmt) selects the instantiation.
-void launch_history(const TrackParams& tp, bool det, int grid, int min_blocks, cudaStream_t s);
-int history_max_ctas_per_sm(bool det, int min_blocks, int fmt);
+// The density format (tp.mesh.fmt) and the storage layout (tp.mesh.tiled) select the
+// instantiation; 256-thread CTAs with <= 80 registers (3 resident per SM).
+void launch_history(const TrackParams& tp, bool det, int grid, cudaStream_t s);
+int history_max_ctas_per_sm(bool det, int fmt, bool tiled);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);
 void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s);

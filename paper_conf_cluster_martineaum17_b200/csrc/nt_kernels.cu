@@ -79,8 +79,8 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet, int kMinBlocks, int kFmt>
-__global__ void __launch_bounds__(kHistoryBlock, kMinBlocks)
+template <bool kDet, int kFmt, bool kTiled>
+__global__ void __launch_bounds__(kHistoryBlock, 3)
 history_kernel(const __grid_constant__ TrackParams P) {
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
   // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
@@ -114,6 +114,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
   const Phys& ph = P.ph;
   const int refill_min = P.refill_min;
+  const int32_t ntx = P.mesh.ntx;
+  // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, see nt_device.cuh cell_index
+  auto cidx_of = [&](int32_t cx_, int32_t cy_) -> int64_t {
+    if constexpr (kTiled)
+      return ((int64_t)((cy_ >> 2) * ntx + (cx_ >> 2)) << 4) | (int64_t)(((cy_ & 3) << 2) | (cx_ & 3));
+    else
+      return (int64_t)cy_ * nx + cx_;
+  };
   const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
 
   bool active = false, exhausted = false;
@@ -128,6 +136,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   double dstep = 0;   // deposits this particle flushed this step
   Mat m{0, 0, 0};
   int32_t cx = 0, cy = 0;
+  int64_t cidx = 0;          // storage index of (cx, cy)
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
 
   for (;;) {
@@ -155,7 +164,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
             cx = P.p.cx[i];
             cy = P.p.cy[i];
             ctr = P.p.ctr[i];
-            draw = dens_load<kFmt>(P.mesh, cell_index(P.mesh, cx, cy));
+            cidx = cidx_of(cx, cy);
+            draw = dens_load<kFmt>(P.mesh, cidx);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             eax = 2;
@@ -194,12 +204,19 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const double ty = oy != 0.0 ? fmax((eyn - y) * ioy, 0.0) : d_inf();
         const bool ax = tx < ty;
         const double df = ax ? tx : ty;
-        const double dc = sig > 0.0 ? mfp / sig : d_inf();
         const double ds = dcen;
+        // dc = n_mfp / Sigma_t only matters if a collision is possible: when
+        // n_mfp > (min(df, ds) * Sigma_t) * (1 + 2^-50) the rounded quotient provably exceeds
+        // min(df, ds), so the event is not a collision and dc is never used.
+        // (The relative-error argument needs a normal product: tiny ones take the division.)
+        const double dmin = df < ds ? df : ds;
+        const double dsig = dmin * sig;
+        const bool maybe_coll = !(mfp > dsig * 1.0000000000000009) || dsig < 1e-290;
+        const double dc = (maybe_coll && sig > 0.0) ? mfp / sig : d_inf();
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
 
         auto flush = [&]() {
-          const int64_t cell = cell_index(P.mesh, cx, cy);
+          const int64_t cell = cidx;                 // storage index of the current cell
           if constexpr (kDet) {
             const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
             if (slot < P.rec_cap) {
@@ -211,7 +228,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
             if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
             ++seq;
           } else {
-            if (!(P.diag & 1)) atomicAdd(P.mesh.tally + cell, acc);  // fire-and-forget fp64 RED at L2
+            atomicAdd(P.mesh.tally + cell, acc);      // fire-and-forget fp64 RED at L2
           }
           dstep += acc;
           acc = 0.0;
@@ -285,9 +302,9 @@ history_kernel(const __grid_constant__ TrackParams P) {
           }
           // next edge on the crossed axis and the new cell's density: two independent loads
           const bool pos2 = refl ? !pos : pos;
-          const double ev = (P.diag & 4) ? (ax ? exn : eyn) + 0.000244140625 * (pos2 ? 1.0 : -1.0) * (refl ? 0.0 : 1.0)
-                                         : __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
-          if (!(P.diag & 2)) draw = dens_load<kFmt>(P.mesh, cell_index(P.mesh, cx, cy));
+          const double ev = __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
+          cidx = cidx_of(cx, cy);
+          draw = dens_load<kFmt>(P.mesh, cidx);     // new cell's density
           enext = ev;
           eax = ax ? 0 : 1;
           nf += 1u;
@@ -360,28 +377,27 @@ history_kernel(const __grid_constant__ TrackParams P) {
   }
 }
 
-template <bool kDet, int kMinBlocks>
+template <bool kDet, bool kTiled>
 static void* history_fn(int fmt) {
-  if (fmt == kDensU8) return (void*)history_kernel<kDet, kMinBlocks, kDensU8>;
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kMinBlocks, kDensU16>;
-  return (void*)history_kernel<kDet, kMinBlocks, kDensF64>;
+  if (fmt == kDensU8) return (void*)history_kernel<kDet, kDensU8, kTiled>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled>;
 }
 
-static void* history_select(bool det, int min_blocks, int fmt) {
-  if (det) return history_fn<true, 3>(fmt);
-  if (min_blocks >= 4) return history_fn<false, 4>(fmt);
-  return history_fn<false, 3>(fmt);
+static void* history_select(bool det, int fmt, bool tiled) {
+  if (det) return tiled ? history_fn<true, true>(fmt) : history_fn<true, false>(fmt);
+  return tiled ? history_fn<false, true>(fmt) : history_fn<false, false>(fmt);
 }
 
-void launch_history(const TrackParams& tp, bool det, int grid, int min_blocks, cudaStream_t s) {
-  void* fn = history_select(det, min_blocks, tp.mesh.fmt);
+void launch_history(const TrackParams& tp, bool det, int grid, cudaStream_t s) {
+  void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
 
-int history_max_ctas_per_sm(bool det, int min_blocks, int fmt) {
+int history_max_ctas_per_sm(bool det, int fmt, bool tiled) {
   int n = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, min_blocks, fmt),
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled),
                                                 kHistoryBlock, 0);
   return n;
 }
