@@ -212,7 +212,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const double dmin = df < ds ? df : ds;
         const double dsig = dmin * sig;
         const bool maybe_coll = !(mfp > dsig * 1.0000000000000009) || dsig < 1e-290;
-        const double dc = (maybe_coll && sig > 0.0) ? mfp / sig : d_inf();
+        double dc = d_inf();
+        if (__builtin_expect(maybe_coll && sig > 0.0, 0)) dc = mfp / sig;   // branch, not a select
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
 
         auto flush = [&]() {
