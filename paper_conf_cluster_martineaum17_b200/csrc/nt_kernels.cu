@@ -173,6 +173,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
             dcen = speed(e, ph) * P.dt;
             iox = 1.0 / ox;
             ioy = 1.0 / oy;
+            if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
+            if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
             acc = 0.0;
             dstep = 0.0;
             nf = 0u;
@@ -198,10 +200,12 @@ history_kernel(const __grid_constant__ TrackParams P) {
         eyn = eax == 1 ? enext : eyn;
         eax = 2;
         const double sig = nd * m.st;
-        // clamp at 0 with fmax: differs from "t < 0 ? 0 : t" only in the sign of a zero and
-        // for NaN, neither of which can change any result
-        const double tx = ox != 0.0 ? fmax((exn - x) * iox, 0.0) : d_inf();
-        const double ty = oy != 0.0 ? fmax((eyn - y) * ioy, 0.0) : d_inf();
+        // An axis with direction cosine 0 carries exn = iox = +inf (set where the direction
+        // changes), so (exn - x) * iox = +inf without a select -- the "ω = 0 -> ∞" of §3.
+        double tx = (exn - x) * iox;
+        tx = tx < 0.0 ? 0.0 : tx;
+        double ty = (eyn - y) * ioy;
+        ty = ty < 0.0 ? 0.0 : ty;
         const bool ax = tx < ty;
         const double df = ax ? tx : ty;
         const double ds = dcen;
@@ -280,12 +284,15 @@ history_kernel(const __grid_constant__ TrackParams P) {
             m = refresh_xs(P.xs, ph, e, nrange);
             iox = 1.0 / ox;
             ioy = 1.0 / oy;
+            if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
+            if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
             mfp = -log(u01(r.b));
           }
         } else if (df < ds) {
           // ---- facet: one code path for both axes (no X/Y divergence) ----
           acc += ((w * df) * sig) * m.H;
-          mfp = fmax(mfp - df * sig, 0.0);
+          const double nm = mfp - df * sig;
+          mfp = nm > 0.0 ? nm : 0.0;
           dcen = dcen - df;
           const double xm = x + df * ox, ym = y + df * oy;
           x = ax ? exn : xm;                          // snap the crossed coordinate
