@@ -153,6 +153,62 @@ __device__ __forceinline__ double number_density(const Mesh& M, const double* __
   }
 }
 
+// ---- L2 residency hints ----------------------------------------------------------------
+// The tally (128 MB at 4000^2) and the density map compete for the 126 MB L2 with the
+// particle store, which is read and written once per step: tally REDs and density gathers
+// carry an evict_last policy, particle-store traffic evict_first.
+__device__ __forceinline__ uint64_t l2_evict_last() {
+  uint64_t p;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+  return p;
+}
+__device__ __forceinline__ uint64_t l2_evict_first() {
+  uint64_t p;
+  asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
+  return p;
+}
+__device__ __forceinline__ void red_add_hint(double* a, double v, uint64_t pol) {
+  asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol)
+               : "memory");
+}
+__device__ __forceinline__ uint32_t ldg_u8_hint(const uint8_t* p, uint64_t pol) {
+  unsigned short v;
+  asm volatile("ld.global.nc.L2::cache_hint.u8 %0, [%1], %2;" : "=h"(v) : "l"(p), "l"(pol));
+  return v;
+}
+template <class T>
+__device__ __forceinline__ T ld_stream(const T* p, uint64_t pol);
+template <>
+__device__ __forceinline__ double ld_stream<double>(const double* p, uint64_t pol) {
+  double v;
+  asm volatile("ld.global.L1::no_allocate.L2::cache_hint.f64 %0, [%1], %2;"
+               : "=d"(v) : "l"(p), "l"(pol));
+  return v;
+}
+template <>
+__device__ __forceinline__ int32_t ld_stream<int32_t>(const int32_t* p, uint64_t pol) {
+  int32_t v;
+  asm volatile("ld.global.L1::no_allocate.L2::cache_hint.s32 %0, [%1], %2;"
+               : "=r"(v) : "l"(p), "l"(pol));
+  return v;
+}
+template <>
+__device__ __forceinline__ uint32_t ld_stream<uint32_t>(const uint32_t* p, uint64_t pol) {
+  uint32_t v;
+  asm volatile("ld.global.L1::no_allocate.L2::cache_hint.u32 %0, [%1], %2;"
+               : "=r"(v) : "l"(p), "l"(pol));
+  return v;
+}
+__device__ __forceinline__ void st_stream(double* p, double v, uint64_t pol) {
+  asm volatile("st.global.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(p), "d"(v), "l"(pol) : "memory");
+}
+__device__ __forceinline__ void st_stream(int32_t* p, int32_t v, uint64_t pol) {
+  asm volatile("st.global.L2::cache_hint.s32 [%0], %1, %2;" ::"l"(p), "r"(v), "l"(pol) : "memory");
+}
+__device__ __forceinline__ void st_stream(uint32_t* p, uint32_t v, uint64_t pol) {
+  asm volatile("st.global.L2::cache_hint.u32 [%0], %1, %2;" ::"l"(p), "r"(v), "l"(pol) : "memory");
+}
+
 // Split form of number_density for latency hiding: dens_load issues the gather (raw code or
 // raw density), dens_nd consumes it later -- the history kernel issues the load at a facet
 // and consumes it at the start of the next event, so the gather overlaps the loop overhead.
@@ -160,8 +216,9 @@ template <int kFmt> struct DensRaw { using type = uint32_t; };
 template <> struct DensRaw<kDensF64> { using type = double; };
 
 template <int kFmt>
-__device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M, int64_t cell) {
-  if constexpr (kFmt == kDensU8) return (uint32_t)__ldg(M.rho8 + cell);
+__device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M, int64_t cell,
+                                                                  uint64_t pol) {
+  if constexpr (kFmt == kDensU8) return ldg_u8_hint(M.rho8 + cell, pol);
   else if constexpr (kFmt == kDensU16) return (uint32_t)__ldg(M.rho16 + cell);
   else return __ldg(M.rho + cell);
 }

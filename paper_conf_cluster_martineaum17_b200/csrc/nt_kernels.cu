@@ -123,6 +123,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
       return (int64_t)cy_ * nx + cx_;
   };
   const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
+  const uint64_t pol_keep = l2_evict_last();     // tally REDs, density gathers
+  const uint64_t pol_stream = l2_evict_first();  // particle store (read / written once)
 
   bool active = false, exhausted = false;
   int32_t i = 0;                 // local particle index (< 2^31)
@@ -154,18 +156,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
           i = (int32_t)(P.lo + (int64_t)my);
           if (P.p.status[i] == 1u) {
             active = true;
-            x = P.p.x[i];
-            y = P.p.y[i];
-            ox = P.p.ox[i];
-            oy = P.p.oy[i];
-            e = P.p.e[i];
-            w = P.p.w[i];
-            mfp = P.p.mfp[i];
-            cx = P.p.cx[i];
-            cy = P.p.cy[i];
-            ctr = P.p.ctr[i];
+            x = ld_stream(P.p.x + i, pol_stream);
+            y = ld_stream(P.p.y + i, pol_stream);
+            ox = ld_stream(P.p.ox + i, pol_stream);
+            oy = ld_stream(P.p.oy + i, pol_stream);
+            e = ld_stream(P.p.e + i, pol_stream);
+            w = ld_stream(P.p.w + i, pol_stream);
+            mfp = ld_stream(P.p.mfp + i, pol_stream);
+            cx = ld_stream(P.p.cx + i, pol_stream);
+            cy = ld_stream(P.p.cy + i, pol_stream);
+            ctr = ld_stream(P.p.ctr + i, pol_stream);
             cidx = cidx_of(cx, cy);
-            draw = dens_load<kFmt>(P.mesh, cidx);
+            draw = dens_load<kFmt>(P.mesh, cidx, pol_keep);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             eax = 2;
@@ -233,7 +235,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
             if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
             ++seq;
           } else {
-            atomicAdd(P.mesh.tally + cell, acc);      // fire-and-forget fp64 RED at L2
+            red_add_hint(P.mesh.tally + cell, acc, pol_keep);   // fire-and-forget fp64 RED at L2
           }
           dstep += acc;
           acc = 0.0;
@@ -312,7 +314,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const bool pos2 = refl ? !pos : pos;
           const double ev = __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
           cidx = cidx_of(cx, cy);
-          draw = dens_load<kFmt>(P.mesh, cidx);     // new cell's density
+          draw = dens_load<kFmt>(P.mesh, cidx, pol_keep);   // new cell's density
           enext = ev;
           eax = ax ? 0 : 1;
           nf += 1u;
@@ -333,19 +335,19 @@ history_kernel(const __grid_constant__ TrackParams P) {
         if (outcome != 0) {
           if (!(isfinite(x) && isfinite(y) && isfinite(e) && isfinite(w)))
             cnt(SU_NONFINITE, 1u);
-          P.p.x[i] = x;
-          P.p.y[i] = y;
-          P.p.ox[i] = ox;
-          P.p.oy[i] = oy;
-          P.p.e[i] = e;
-          P.p.w[i] = w;
-          P.p.mfp[i] = mfp;
-          P.p.dep[i] += dstep;
-          P.p.cx[i] = cx;
-          P.p.cy[i] = cy;
-          P.p.ctr[i] = ctr;
-          P.p.nfac[i] += nf;
-          P.p.ncol[i] += nc;
+          st_stream(P.p.x + i, x, pol_stream);
+          st_stream(P.p.y + i, y, pol_stream);
+          st_stream(P.p.ox + i, ox, pol_stream);
+          st_stream(P.p.oy + i, oy, pol_stream);
+          st_stream(P.p.e + i, e, pol_stream);
+          st_stream(P.p.w + i, w, pol_stream);
+          st_stream(P.p.mfp + i, mfp, pol_stream);
+          st_stream(P.p.dep + i, ld_stream(P.p.dep + i, pol_stream) + dstep, pol_stream);
+          st_stream(P.p.cx + i, cx, pol_stream);
+          st_stream(P.p.cy + i, cy, pol_stream);
+          st_stream(P.p.ctr + i, ctr, pol_stream);
+          st_stream(P.p.nfac + i, ld_stream(P.p.nfac + i, pol_stream) + nf, pol_stream);
+          st_stream(P.p.ncol + i, ld_stream(P.p.ncol + i, pol_stream) + nc, pol_stream);
           if (outcome == 1) {
             P.p.ncen[i] += 1u;
           } else {
