@@ -77,8 +77,12 @@ typedef struct {
     int32_t refill_min;        /* history mode: a warp refills its idle lanes once at least
                                   this many are idle (0 -> 8)                              */
     int32_t density_format;    /* 0: lossless u8/u16 material codes when the density map
-                                  holds <= 256 / 65536 distinct values, else f64;
-                                  1: always the f64 map                                    */
+                                  holds <= 256 / 65536 distinct values, else f64; with u8
+                                  codes (<= 254 values) also a block map (the code of each
+                                  uniform 2^k x 2^k-cell block, <= 16 KB) that the history
+                                  kernel keeps in shared memory;
+                                  1: always the f64 map;
+                                  2: as 0 without the block map (ablation)                 */
     int32_t layout;            /* storage of the tally and density maps: 0: 4x4-cell tiles
                                   (a tile's 16 f64 tally cells = one 128 B line, so a
                                   particle's consecutive facets stay in few L2 lines);

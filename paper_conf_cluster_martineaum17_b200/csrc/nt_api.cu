@@ -62,6 +62,8 @@ struct nt_ctx {
   double W = 0, H = 0;
   DevBuf rho, tally, tally_local, ex, ey;
   DevBuf rho_code, nd_tab, enc_keys;     // lossless density encoding
+  DevBuf blk;                            // block map of the u8 codes (Mesh::blk)
+  int blk_shift = 0, blk_nbx = 0, blk_n = 0;   // blk_n = 0: no block map
   DevBuf rho_st, tally_rm;               // f64 density in storage layout; row-major staging
   int dens_fmt = kDensF64, dens_codes = 0;
   int tiled = 0, ntx = 0;                // storage layout of tally / density (cell_index)
@@ -221,7 +223,8 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.refill_min > 32) opt.refill_min = 32;
   if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
-      opt.rank < 0 || opt.rank >= opt.nranks)
+      opt.rank < 0 || opt.rank >= opt.nranks || opt.density_format < 0 ||
+      opt.density_format > 2 || opt.layout < 0 || opt.layout > 1)
     return NT_ERR_ARG;
   if (opt.nranks > 1 && !opt.nccl_unique_id) return NT_ERR_ARG;
 
@@ -263,7 +266,7 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
-  for (DevBuf* b : {&c->rho_code, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
+  for (DevBuf* b : {&c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup})
     b->release();
@@ -311,7 +314,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   NT_CUDA(c, launch_density_check(c->rho.as<double>(), cells, bad, c->stream));
   // distinct density values (for the lossless encoding)
   int fmt = kDensF64, nu = 0;
-  if (c->opt.density_format == 0) {
+  if (c->opt.density_format == 0 || c->opt.density_format == 2) {
     size_t tmp = 0;
     NT_CUDA(c, c->enc_keys.ensure((size_t)cells * 16));
     unsigned long long* k0 = c->enc_keys.as<unsigned long long>();
@@ -326,7 +329,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   if (hb[0] != 0)
     return fail(c, NT_ERR_ARG, "%llu density values are not finite and >= 0", hb[0]);
-  if (c->opt.density_format == 0) {
+  if (c->opt.density_format == 0 || c->opt.density_format == 2) {
     nu = (int)(hb[1] & 0xffffffffu);
     if (nu <= 256) fmt = kDensU8;
     else if (nu <= 65536) fmt = kDensU16;
@@ -338,7 +341,28 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
     NT_CUDA(c, c->nd_tab.ensure((size_t)nu * 8));
     NT_CUDA(c, launch_encode(c->rho.as<double>(), cells, ml, c->enc_keys.as<unsigned long long>(),
                              nu, c->ph.cn, fmt, c->rho_code.p, c->nd_tab.as<double>(), c->stream));
-  } else if (tiled) {
+  }
+  // block map (density_format 0, u8 codes with a spare code for "mixed"): the smallest
+  // power-of-two block side >= 4 whose map fits kBlkMax bytes of shared memory
+  int blk_shift = 0, blk_nbx = 0, blk_n = 0;
+  if (fmt == kDensU8 && nu < (int)kBlkMixed && c->opt.density_format == 0) {
+    for (int s = 2; s < 31; ++s) {
+      const int64_t bx = ((int64_t)nx + (1 << s) - 1) >> s, by = ((int64_t)ny + (1 << s) - 1) >> s;
+      if (bx * by <= kBlkMax) {
+        blk_shift = s;
+        blk_nbx = (int)bx;
+        blk_n = (int)(bx * by);
+        break;
+      }
+    }
+    Mesh mb = ml;
+    mb.bshift = blk_shift;
+    mb.nbx = blk_nbx;
+    mb.nblk = blk_n;
+    NT_CUDA(c, c->blk.ensure(align256((size_t)blk_n)));
+    NT_CUDA(c, launch_block_map(c->rho_code.as<uint8_t>(), mb, c->blk.as<uint8_t>(), c->stream));
+  }
+  if (fmt == kDensF64 && tiled) {
     NT_CUDA(c, c->rho_st.ensure((size_t)cells_st * 8));
     NT_CUDA(c, cudaMemsetAsync(c->rho_st.p, 0, (size_t)cells_st * 8, c->stream));
     NT_CUDA(c, launch_relayout(c->rho.as<double>(), c->rho_st.as<double>(), cells, ml, true, c->stream));
@@ -349,6 +373,9 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   c->dens_fmt = fmt;
   c->dens_codes = nu;
+  c->blk_shift = blk_shift;
+  c->blk_nbx = blk_nbx;
+  c->blk_n = blk_n;
   c->tiled = tiled;
   c->ntx = ntx;
   c->cells_st = cells_st;
@@ -521,6 +548,10 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.mesh.nd_tab = c->nd_tab.as<double>();
   tp.mesh.fmt = c->dens_fmt;
   tp.mesh.ncodes = c->dens_codes;
+  tp.mesh.blk = c->blk_n > 0 ? c->blk.as<uint8_t>() : nullptr;
+  tp.mesh.bshift = c->blk_shift;
+  tp.mesh.nbx = c->blk_nbx;
+  tp.mesh.nblk = c->blk_n;
   tp.mesh.tally = c->tally.as<double>();
   tp.mesh.ex = c->ex.as<double>();
   tp.mesh.ey = c->ey.as<double>();
@@ -548,7 +579,8 @@ static TrackParams make_params(nt_ctx* c, double dt) {
 
 // Persistent grid of the history kernel: SMs x resident CTAs (ctas_per_sm caps it).
 static int history_grid(nt_ctx* c, bool det) {
-  int per_sm = history_max_ctas_per_sm(det, c->dens_fmt, c->tiled != 0);
+  int per_sm = history_max_ctas_per_sm(det, c->dens_fmt, c->tiled != 0, c->blk_n > 0,
+                                       c->opt.ctas_per_sm);
   if (per_sm < 1) per_sm = 1;
   if (c->opt.ctas_per_sm > 0 && c->opt.ctas_per_sm < per_sm) per_sm = c->opt.ctas_per_sm;
   return c->sm_count * per_sm;
@@ -586,7 +618,7 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
     if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
     return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
   }
-  launch_history(bp, det, history_grid(c, det), c->stream);
+  launch_history(bp, det, history_grid(c, det), c->opt.ctas_per_sm, c->stream);
   ++launches;
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;

@@ -45,7 +45,16 @@ struct Mesh {
   int32_t fmt, ncodes;
   int32_t tiled;                      // 1: 4x4-cell tiles (one 128 B tally line per tile)
   int32_t ntx;                        // tiles per row = ceil(nx / 4)
+  // Block map (kDensU8 only, lossless): blocks of 2^bshift x 2^bshift cells, row-major
+  // [nby][nbx]; entry = the block's material code when every cell of the block has that
+  // code, kBlkMixed otherwise.  The history kernel keeps it in shared memory, so a facet
+  // into a uniform block needs no global gather.  blk == nullptr: no block map.
+  const uint8_t* __restrict__ blk;
+  int32_t bshift, nbx, nblk, pad2;
 };
+
+constexpr uint32_t kBlkMixed = 255u;   // block-map entry: block holds more than one code
+constexpr int kBlkMax = 16384;         // max block-map entries (bytes of shared memory)
 
 // Storage index of cell (cx, cy) in the tally and density arrays.  Tiled layout: 4x4-cell
 // tiles in row-major tile order, row-major inside a tile, so the 16 f64 tally cells of a
@@ -221,6 +230,16 @@ __device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M,
   if constexpr (kFmt == kDensU8) return ldg_u8_hint(M.rho8 + cell, pol);
   else if constexpr (kFmt == kDensU16) return (uint32_t)__ldg(M.rho16 + cell);
   else return __ldg(M.rho + cell);
+}
+
+// u8 code of cell (cx, cy) via the shared-memory block map: the block's code when the block
+// is uniform, else the cell's own code from the global map (storage index cidx).
+__device__ __forceinline__ uint32_t dens_load_blk(const Mesh& M, const uint8_t* s_blk,
+                                                  int32_t cx, int32_t cy, int64_t cidx,
+                                                  uint64_t pol) {
+  uint32_t code = s_blk[(cy >> M.bshift) * M.nbx + (cx >> M.bshift)];
+  if (code == kBlkMixed) code = ldg_u8_hint(M.rho8 + cidx, pol);
+  return code;
 }
 
 __device__ __forceinline__ void prefetch_l1(const void* p) {

@@ -48,9 +48,10 @@ void launch_edges(double* ex, int32_t nx, double W, double* ey, int32_t ny, doub
 void launch_inject(const InjectParams& ip, cudaStream_t s);
 // History (Over Particles) tracking: grid = persistent CTAs.
 // The density format (tp.mesh.fmt) and the storage layout (tp.mesh.tiled) select the
-// instantiation; 256-thread CTAs with <= 80 registers (3 resident per SM).
-void launch_history(const TrackParams& tp, bool det, int grid, cudaStream_t s);
-int history_max_ctas_per_sm(bool det, int fmt, bool tiled);
+// instantiation; 256-thread CTAs with <= 80 registers (3 resident per SM), or -- minb = 4,
+// production u8 + block map only -- <= 64 registers (4 per SM).
+void launch_history(const TrackParams& tp, bool det, int grid, int minb, cudaStream_t s);
+int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);
 void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s);
@@ -78,6 +79,9 @@ cudaError_t launch_encode(const double* rho, int64_t n, const Mesh& M,
                           const unsigned long long* uniq, int nu, double cn, int fmt, void* code,
                           double* nd_tab, cudaStream_t s);
 // Row-major [ny][nx] <-> the mesh's storage layout (cell_index).
+// Block map (Mesh::blk) of the u8 code map: blk[by * nbx + bx] = the block's code if uniform,
+// else kBlkMixed.  M.bshift / M.nbx / M.nblk describe the blocks.
+cudaError_t launch_block_map(const uint8_t* code, const Mesh& M, uint8_t* blk, cudaStream_t s);
 cudaError_t launch_relayout(const double* src, double* dst, int64_t n, const Mesh& M,
                             bool to_storage, cudaStream_t s);
 }  // namespace nt

@@ -79,15 +79,17 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet, int kFmt, bool kTiled>
-__global__ void __launch_bounds__(kHistoryBlock, 3)
+template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB>
+__global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
+  static_assert(!kBlk || kFmt == kDensU8, "the block map indexes u8 material codes");
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
   // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
   // almost no shared memory and the L1 stays free for the density / edge gathers.
   constexpr int kWarps = kHistoryBlock / 32;
   __shared__ uint32_t s_u[kWarps][SU_COUNT];
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
+  __shared__ uint8_t s_blk[kBlk ? kBlkMax : 1];
   const int t = threadIdx.x;
   const int64_t gt = (int64_t)blockIdx.x * kHistoryBlock + t;
   const int64_t sstride = (int64_t)gridDim.x * kHistoryBlock;
@@ -98,6 +100,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
   __syncthreads();
   if constexpr (kFmt == kDensU8) {
     for (int k = t; k < 256; k += kHistoryBlock) s_nd[k] = k < P.mesh.ncodes ? P.mesh.nd_tab[k] : 0.0;
+    if constexpr (kBlk) {
+      const uint4* src = reinterpret_cast<const uint4*>(P.mesh.blk);
+      for (int k = t; k < (P.mesh.nblk + 15) / 16; k += kHistoryBlock)
+        reinterpret_cast<uint4*>(s_blk)[k] = __ldg(src + k);
+    }
     __syncthreads();
   }
   const int wid = t >> 5;
@@ -125,6 +132,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
   const uint64_t pol_keep = l2_evict_last();     // tally REDs, density gathers
   const uint64_t pol_stream = l2_evict_first();  // particle store (read / written once)
+  // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather
+  auto dload = [&](int32_t cx_, int32_t cy_, int64_t ci_) {
+    if constexpr (kBlk) return dens_load_blk(P.mesh, s_blk, cx_, cy_, ci_, pol_keep);
+    else return dens_load<kFmt>(P.mesh, ci_, pol_keep);
+  };
 
   bool active = false, exhausted = false;
   int32_t i = 0;                 // local particle index (< 2^31)
@@ -167,7 +179,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
             cy = ld_stream(P.p.cy + i, pol_stream);
             ctr = ld_stream(P.p.ctr + i, pol_stream);
             cidx = cidx_of(cx, cy);
-            draw = dens_load<kFmt>(P.mesh, cidx, pol_keep);
+            draw = dload(cx, cy, cidx);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             eax = 2;
@@ -314,7 +326,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const bool pos2 = refl ? !pos : pos;
           const double ev = __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
           cidx = cidx_of(cx, cy);
-          draw = dens_load<kFmt>(P.mesh, cidx, pol_keep);   // new cell's density
+          draw = dload(cx, cy, cidx);                 // new cell's density
           enext = ev;
           eax = ax ? 0 : 1;
           nf += 1u;
@@ -387,27 +399,34 @@ history_kernel(const __grid_constant__ TrackParams P) {
   }
 }
 
+// Instantiations: deterministic/production x density format x layout x block map; the
+// production u8 + block-map kernels also come with a 64-register cap (4 CTAs per SM,
+// selected by ctas_per_sm = 4; the default is 80 registers, 3 CTAs per SM).
 template <bool kDet, bool kTiled>
-static void* history_fn(int fmt) {
-  if (fmt == kDensU8) return (void*)history_kernel<kDet, kDensU8, kTiled>;
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled>;
-  return (void*)history_kernel<kDet, kDensF64, kTiled>;
+static void* history_fn(int fmt, bool blk, int minb) {
+  if (fmt == kDensU8) {
+    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 3>;
+    if (!kDet && minb >= 4) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 4>;
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 3>;
+  }
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 3>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 3>;
 }
 
-static void* history_select(bool det, int fmt, bool tiled) {
-  if (det) return tiled ? history_fn<true, true>(fmt) : history_fn<true, false>(fmt);
-  return tiled ? history_fn<false, true>(fmt) : history_fn<false, false>(fmt);
+static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb) {
+  if (det) return tiled ? history_fn<true, true>(fmt, blk, minb) : history_fn<true, false>(fmt, blk, minb);
+  return tiled ? history_fn<false, true>(fmt, blk, minb) : history_fn<false, false>(fmt, blk, minb);
 }
 
-void launch_history(const TrackParams& tp, bool det, int grid, cudaStream_t s) {
-  void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0);
+void launch_history(const TrackParams& tp, bool det, int grid, int minb, cudaStream_t s) {
+  void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
 
-int history_max_ctas_per_sm(bool det, int fmt, bool tiled) {
+int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb) {
   int n = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled),
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb),
                                                 kHistoryBlock, 0);
   return n;
 }

@@ -57,6 +57,27 @@ __global__ void relayout_kernel(const double* __restrict__ src, double* __restri
   }
 }
 
+// One thread per block: the block's code if all its cells (inside the mesh) share it.
+__global__ void block_map_kernel(const uint8_t* __restrict__ code, Mesh M,
+                                 uint8_t* __restrict__ blk) {
+  const int32_t b = blockIdx.x * blockDim.x + threadIdx.x;
+  if (b >= M.nblk) return;
+  const int32_t by = b / M.nbx, bx = b - by * M.nbx;
+  const int32_t x0 = bx << M.bshift, y0 = by << M.bshift, side = 1 << M.bshift;
+  const int32_t x1 = min(x0 + side, M.nx), y1 = min(y0 + side, M.ny);
+  const uint32_t c0 = code[cell_index(M, x0, y0)];
+  uint32_t out = c0;
+  for (int32_t cy = y0; cy < y1 && out != kBlkMixed; ++cy)
+    for (int32_t cx = x0; cx < x1; ++cx)
+      if (code[cell_index(M, cx, cy)] != c0) { out = kBlkMixed; break; }
+  blk[b] = (uint8_t)out;
+}
+
+cudaError_t launch_block_map(const uint8_t* code, const Mesh& M, uint8_t* blk, cudaStream_t s) {
+  block_map_kernel<<<(M.nblk + 127) / 128, 128, 0, s>>>(code, M, blk);
+  return cudaGetLastError();
+}
+
 // nd_tab[k] = rho_k * cn: the first product of DESIGN.md §3 MAT, rounded once, as in place.
 __global__ void nd_table_kernel(const unsigned long long* __restrict__ uniq, int nu, double cn,
                                 double* __restrict__ tab) {

@@ -105,6 +105,10 @@ CONFIGS: dict[str, Config] = {
     "small_random": Config("small_random", 300, 300, "random", (0.3, 0.3, 0.4, 0.4), 3000, 17, rho=2.0),
     "tiny_stream": Config("tiny_stream", 64, 64, "uniform_lo", (0.45, 0.45, 0.1, 0.1), 2000, 8),
     "tiny_split": Config("tiny_split", 64, 64, "split", (0.0, 0.0, 1.0, 1.0), 2000, 9),
+    # a few materials in random rectangles on ragged meshes: u8 codes whose block map holds
+    # both uniform and mixed blocks (block sides 4 and 8)
+    "tiny_mosaic": Config("tiny_mosaic", 70, 50, "mosaic", (0.1, 0.1, 0.8, 0.8), 2000, 18, _SINGLE, rho=2.0),
+    "small_mosaic": Config("small_mosaic", 601, 590, "mosaic", (0.2, 0.2, 0.6, 0.6), 3000, 19, rho=0.5),
     "small_csp": Config("small_csp", 256, 256, "csp", (0.0, 0.0, 0.1, 0.1), 4096, 10),
     "small_scatter": Config("small_scatter", 256, 256, "uniform_hi", (0.45, 0.45, 0.1, 0.1), 8192, 12),
 }
@@ -129,6 +133,15 @@ def density(cfg: Config) -> np.ndarray:
     if cfg.density == "random":      # continuous random densities: no lossless code fits
         rng = np.random.default_rng(cfg.seed)
         return rng.uniform(0.0, cfg.rho, (ny, nx))
+    if cfg.density == "mosaic":      # 12 random rectangles of 5 materials over rho_lo
+        rng = np.random.default_rng(cfg.seed)
+        levels = np.array([0.0, RHO_LO, 0.05 * cfg.rho, cfg.rho, 20.0 * cfg.rho])
+        rho = np.full((ny, nx), RHO_LO)
+        for _ in range(12):
+            x0, y0 = rng.integers(0, nx), rng.integers(0, ny)
+            w, h = rng.integers(1, max(2, nx // 3)), rng.integers(1, max(2, ny // 3))
+            rho[y0:y0 + h, x0:x0 + w] = levels[rng.integers(0, len(levels))]
+        return rho
     if cfg.density == "csp":
         inx = (xc >= 0.25 * cfg.width) & (xc <= 0.75 * cfg.width)
         iny = (yc >= 0.25 * cfg.height) & (yc <= 0.75 * cfg.height)
