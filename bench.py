@@ -175,6 +175,7 @@ def parse():
     ap.add_argument("--layout", type=int, default=0, help="0 tiled 4x4 (default), 1 row-major")
     ap.add_argument("--density-format", type=int, default=0,
                     help="0 u8/u16 codes + block map (default), 1 f64 map, 2 codes without block map")
+    ap.add_argument("--tally-mode", type=int, default=0, help="0 one RED per flush, 1 warp-aggregated")
     ap.add_argument("--json-out", default=None)
     ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
     return ap.parse_args()
@@ -251,7 +252,8 @@ def main():
     tr = binding.Tracker(device=local, stream=stream.cuda_stream, mode=a.mode, rank=rank,
                          nranks=world, unique_id=uid, A=cfg.A, molar_mass=cfg.molar_mass,
                          e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm,
-                         refill_min=a.refill_min, layout=a.layout, density_format=a.density_format)
+                         refill_min=a.refill_min, layout=a.layout, density_format=a.density_format,
+                         tally_mode=a.tally_mode)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -340,6 +342,7 @@ def main():
             "config": {"workload": cfg.name, "mode": a.mode, "nx": cfg.nx, "ny": cfg.ny,
                        "layout": "tiled4x4" if a.layout == 0 else "row-major",
                        "density_format": ["codes+block map", "f64", "codes"][a.density_format],
+                       "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED"][a.tally_mode],
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
                        "tables": [len(tables[0]), len(tables[2])],
                        "parallelism": f"dp{world} (particle id shards, tally NCCL allreduce)",

@@ -87,7 +87,11 @@ typedef struct {
                                   (a tile's 16 f64 tally cells = one 128 B line, so a
                                   particle's consecutive facets stay in few L2 lines);
                                   1: row-major.  nt_read_tally always returns row-major.  */
-    int32_t reserved;
+    int32_t tally_mode;        /* production tally flushes: 0: one fp64
+                                  atomic add per flush; 1: warp-aggregated -- lanes flushing
+                                  into the same cell at the same time are summed with warp
+                                  shuffles and one lane issues the atomic (history mode,
+                                  u8 block-map meshes; others fall back to 0)              */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

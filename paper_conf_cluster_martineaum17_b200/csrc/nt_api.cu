@@ -224,7 +224,8 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
       opt.rank < 0 || opt.rank >= opt.nranks || opt.density_format < 0 ||
-      opt.density_format > 2 || opt.layout < 0 || opt.layout > 1)
+      opt.density_format > 2 || opt.layout < 0 || opt.layout > 1 || opt.tally_mode < 0 ||
+      opt.tally_mode > 1)
     return NT_ERR_ARG;
   if (opt.nranks > 1 && !opt.nccl_unique_id) return NT_ERR_ARG;
 
@@ -298,6 +299,8 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   const int tiled = c->opt.layout == 0 ? 1 : 0;
   const int ntx = (nx + 3) / 4, nty = (ny + 3) / 4;
   const int64_t cells_st = tiled ? (int64_t)ntx * nty * 16 : cells;
+  if (cells_st >= (1ll << 32))
+    return fail(c, NT_ERR_ARG, "the tiled mesh storage must hold < 2^32 cells");
   Mesh ml{};
   ml.nx = nx;
   ml.ny = ny;
@@ -618,7 +621,7 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
     if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
     return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
   }
-  launch_history(bp, det, history_grid(c, det), c->opt.ctas_per_sm, c->stream);
+  launch_history(bp, det, history_grid(c, det), c->opt.ctas_per_sm, c->opt.tally_mode, c->stream);
   ++launches;
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;
@@ -692,8 +695,8 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   if (c->stage < ST_PARTICLES) return fail(c, NT_ERR_STATE, "nt_inject_particles must come first");
   if (!(dt > 0.0) || !is_fin(dt)) return fail(c, NT_ERR_ARG, "dt must be finite and > 0");
   NT_CUDA(c, c->scratch.ensure(1024));
-  // per-thread statistic slots for the largest persistent grid (8 CTAs of 256 per SM)
-  NT_CUDA(c, c->slots.ensure((size_t)c->sm_count * 8 * kHistoryBlock * SF_COUNT * 8));
+  // per-thread statistic slots for the largest persistent grid (16 CTAs per SM)
+  NT_CUDA(c, c->slots.ensure((size_t)c->sm_count * 16 * kHistoryBlock * SF_COUNT * 8));
   const size_t cells = (size_t)c->cells_st;   // storage layout (tiles padded with zeros)
   uint32_t launches = 0;
   const bool det = c->opt.deterministic != 0;

@@ -162,6 +162,13 @@ __device__ __forceinline__ double number_density(const Mesh& M, const double* __
   }
 }
 
+// max(v, 0) on the sign bit: +0 for negative v and -0 (R28: differs from
+// v > 0 ? v : 0 only for a NaN with the sign bit clear, which stays NaN).
+__device__ __forceinline__ double clamp0(double v) {
+  const long long b = __double_as_longlong(v);
+  return __longlong_as_double(b & ~(b >> 63));
+}
+
 // ---- L2 residency hints ----------------------------------------------------------------
 // The tally (128 MB at 4000^2) and the density map compete for the 126 MB L2 with the
 // particle store, which is read and written once per step: tally REDs and density gathers
@@ -180,6 +187,30 @@ __device__ __forceinline__ void red_add_hint(double* a, double v, uint64_t pol) 
   asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol)
                : "memory");
 }
+// Warp-aggregated flush (tally_mode 1): the lanes executing this call that flush into the
+// same cell are grouped with __match_any_sync; the group's lowest lane adds the group's
+// values (its own first, then the others in lane order) and issues the one RED.  Lanes
+// without a peer (the usual case away from hot spots) take the plain RED after one vote.
+__device__ __forceinline__ void red_add_warp(double* tally, uint32_t cell, double v, uint64_t pol) {
+  const unsigned act = __activemask();
+  const unsigned peers = __match_any_sync(act, cell);
+  const unsigned gmax = __reduce_max_sync(act, (unsigned)__popc(peers));
+  if (gmax > 1u) {
+    const int lane = threadIdx.x & 31;
+    const unsigned g = (unsigned)__popc(peers);
+    const bool leader = (__ffs(peers) - 1) == lane;
+    double sum = v;
+    for (unsigned k = 1; k < gmax; ++k) {
+      const int src = k < g ? (int)__fns(peers, 0, (int)k + 1) : lane;
+      const double o = __shfl_sync(act, v, src);
+      if (leader && k < g) sum += o;
+    }
+    if (leader) red_add_hint(tally + cell, sum, pol);
+  } else {
+    red_add_hint(tally + cell, v, pol);
+  }
+}
+
 __device__ __forceinline__ uint32_t ldg_u8_hint(const uint8_t* p, uint64_t pol) {
   unsigned short v;
   asm volatile("ld.global.nc.L2::cache_hint.u8 %0, [%1], %2;" : "=h"(v) : "l"(p), "l"(pol));
@@ -225,7 +256,7 @@ template <int kFmt> struct DensRaw { using type = uint32_t; };
 template <> struct DensRaw<kDensF64> { using type = double; };
 
 template <int kFmt>
-__device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M, int64_t cell,
+__device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M, uint32_t cell,
                                                                   uint64_t pol) {
   if constexpr (kFmt == kDensU8) return ldg_u8_hint(M.rho8 + cell, pol);
   else if constexpr (kFmt == kDensU16) return (uint32_t)__ldg(M.rho16 + cell);
@@ -235,7 +266,7 @@ __device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M,
 // u8 code of cell (cx, cy) via the shared-memory block map: the block's code when the block
 // is uniform, else the cell's own code from the global map (storage index cidx).
 __device__ __forceinline__ uint32_t dens_load_blk(const Mesh& M, const uint8_t* s_blk,
-                                                  int32_t cx, int32_t cy, int64_t cidx,
+                                                  int32_t cx, int32_t cy, uint32_t cidx,
                                                   uint64_t pol) {
   uint32_t code = s_blk[(cy >> M.bshift) * M.nbx + (cx >> M.bshift)];
   if (code == kBlkMixed) code = ldg_u8_hint(M.rho8 + cidx, pol);

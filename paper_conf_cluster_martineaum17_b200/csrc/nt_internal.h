@@ -48,9 +48,11 @@ void launch_edges(double* ex, int32_t nx, double W, double* ey, int32_t ny, doub
 void launch_inject(const InjectParams& ip, cudaStream_t s);
 // History (Over Particles) tracking: grid = persistent CTAs.
 // The density format (tp.mesh.fmt) and the storage layout (tp.mesh.tiled) select the
-// instantiation; 256-thread CTAs with <= 80 registers (3 resident per SM), or -- minb = 4,
-// production u8 + block map only -- <= 64 registers (4 per SM).
-void launch_history(const TrackParams& tp, bool det, int grid, int minb, cudaStream_t s);
+// instantiation; 128-thread CTAs with <= 80 registers (6 resident per SM), or -- minb = 7,
+// production u8 + block map only -- <= 72 registers (7 per SM).
+// tally_mode 1 (production u8 + block map only): warp-aggregated tally flushes.
+void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
+                    cudaStream_t s);
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);
@@ -62,7 +64,7 @@ cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long*
                        unsigned long long* kout, const double* vin, double* vout,
                        unsigned long long n, int end_bit, cudaStream_t s);
 
-constexpr int kHistoryBlock = 256;
+constexpr int kHistoryBlock = 128;
 
 }  // namespace nt
 

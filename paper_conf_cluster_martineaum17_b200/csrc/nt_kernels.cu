@@ -79,10 +79,11 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB>
+template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
   static_assert(!kBlk || kFmt == kDensU8, "the block map indexes u8 material codes");
+  static_assert(!(kAgg && kDet), "aggregation reorders the sum: production tally only");
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
   // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
   // almost no shared memory and the L1 stays free for the density / edge gathers.
@@ -123,17 +124,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const int refill_min = P.refill_min;
   const int32_t ntx = P.mesh.ntx;
   // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, see nt_device.cuh cell_index
-  auto cidx_of = [&](int32_t cx_, int32_t cy_) -> int64_t {
+  // (32-bit: nt_init_mesh guarantees the storage fits 2^32 cells)
+  auto cidx_of = [&](int32_t cx_, int32_t cy_) -> uint32_t {
     if constexpr (kTiled)
-      return ((int64_t)((cy_ >> 2) * ntx + (cx_ >> 2)) << 4) | (int64_t)(((cy_ & 3) << 2) | (cx_ & 3));
+      return ((uint32_t)((cy_ >> 2) * ntx + (cx_ >> 2)) << 4) | (uint32_t)(((cy_ & 3) << 2) | (cx_ & 3));
     else
-      return (int64_t)cy_ * nx + cx_;
+      return (uint32_t)cy_ * (uint32_t)nx + (uint32_t)cx_;
   };
   const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
   const uint64_t pol_keep = l2_evict_last();     // tally REDs, density gathers
   const uint64_t pol_stream = l2_evict_first();  // particle store (read / written once)
   // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather
-  auto dload = [&](int32_t cx_, int32_t cy_, int64_t ci_) {
+  auto dload = [&](int32_t cx_, int32_t cy_, uint32_t ci_) {
     if constexpr (kBlk) return dens_load_blk(P.mesh, s_blk, cx_, cy_, ci_, pol_keep);
     else return dens_load<kFmt>(P.mesh, ci_, pol_keep);
   };
@@ -144,15 +146,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
   double x = 0, y = 0, ox = 0, oy = 0, iox = 0, ioy = 0, e = 0, w = 0, mfp = 0, dcen = 0;
   typename DensRaw<kFmt>::type draw = 0;  // density (code) of the current cell, as loaded
   double exn = 0, eyn = 0;  // edge each axis is heading to (facet distance, snap value)
-  double enext = 0;         // edge loaded at the last facet, for axis eax (2 = none pending)
-  int eax = 2;
   double acc = 0;     // deposit accumulated in the current cell
   double dstep = 0;   // deposits this particle flushed this step
   Mat m{0, 0, 0};
   int32_t cx = 0, cy = 0;
-  int64_t cidx = 0;          // storage index of (cx, cy)
+  uint32_t cidx = 0;         // storage index of (cx, cy)
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
 
+  int thr = refill_min;   // break the event loop once this many lanes are idle (32: all)
   for (;;) {
     // ---- refill idle lanes with new particles: one atomic per warp ----
     const unsigned idle = __ballot_sync(kFull, !active);
@@ -161,7 +162,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
       unsigned long long base = 0;
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
       base = __shfl_sync(kFull, base, leader);
-      if (base + (unsigned long long)__popc(idle) >= span) exhausted = true;
+      if (base + (unsigned long long)__popc(idle) >= span) {
+        exhausted = true;
+        thr = 32;
+      }
       if (!active) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
         if (my < span) {
@@ -182,7 +186,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
             draw = dload(cx, cy, cidx);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
-            eax = 2;
             m = refresh_xs(P.xs, ph, e, nrange);
             dcen = speed(e, ph) * P.dt;
             iox = 1.0 / ox;
@@ -209,10 +212,9 @@ history_kernel(const __grid_constant__ TrackParams P) {
       if (active) {
         // ---- one event (Listing 1) ----
         // consume the gathers issued by the previous facet (density code, next edge)
-        const double nd = dens_nd<kFmt>(draw, ndtab, ph.cn);
-        exn = eax == 0 ? enext : exn;
-        eyn = eax == 1 ? enext : eyn;
-        eax = 2;
+        double nd;
+        if constexpr (kFmt == kDensU8) nd = s_nd[draw];
+        else nd = dens_nd<kFmt>(draw, ndtab, ph.cn);
         const double sig = nd * m.st;
         // An axis with direction cosine 0 carries exn = iox = +inf (set where the direction
         // changes), so (exn - x) * iox = +inf without a select -- the "ω = 0 -> ∞" of §3.
@@ -231,11 +233,15 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const double dsig = dmin * sig;
         const bool maybe_coll = !(mfp > dsig * 1.0000000000000009) || dsig < 1e-290;
         double dc = d_inf();
-        if (__builtin_expect(maybe_coll && sig > 0.0, 0)) dc = mfp / sig;   // branch, not a select
+        bool coll = false;
+        if (__builtin_expect(maybe_coll && sig > 0.0, 0)) {  // branch, not a select
+          dc = mfp / sig;
+          coll = dc < df && dc < ds;
+        }
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
 
         auto flush = [&]() {
-          const int64_t cell = cidx;                 // storage index of the current cell
+          const uint32_t cell = cidx;                // storage index of the current cell
           if constexpr (kDet) {
             const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
             if (slot < P.rec_cap) {
@@ -246,6 +252,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
             }
             if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
             ++seq;
+          } else if constexpr (kAgg) {
+            red_add_warp(P.mesh.tally, cell, acc, pol_keep);
           } else {
             red_add_hint(P.mesh.tally + cell, acc, pol_keep);   // fire-and-forget fp64 RED at L2
           }
@@ -261,7 +269,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_KILLED_E, w * e);
           fsum(SF_KILLED_W, w);
           outcome = 2;
-        } else if (dc < df && dc < ds) {
+        } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
           acc += ((w * dc) * sig) * m.H;
           x = x + dc * ox;
@@ -305,8 +313,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
         } else if (df < ds) {
           // ---- facet: one code path for both axes (no X/Y divergence) ----
           acc += ((w * df) * sig) * m.H;
-          const double nm = mfp - df * sig;
-          mfp = nm > 0.0 ? nm : 0.0;
+          mfp = clamp0(mfp - df * sig);
           dcen = dcen - df;
           const double xm = x + df * ox, ym = y + df * oy;
           x = ax ? exn : xm;                          // snap the crossed coordinate
@@ -322,13 +329,13 @@ history_kernel(const __grid_constant__ TrackParams P) {
           if (refl) {                               // rare: a branch beats 8 selects
             if (ax) { ox = -ox; iox = -iox; } else { oy = -oy; ioy = -ioy; }
           }
-          // next edge on the crossed axis and the new cell's density: two independent loads
+          // next edge on the crossed axis and the new cell's density: two independent loads,
+          // consumed at the next event
           const bool pos2 = refl ? !pos : pos;
-          const double ev = __ldg((ax ? ex : ey) + (pos2 ? c2 + 1 : c2));
+          const int32_t ke = pos2 ? c2 + 1 : c2;
+          if (ax) exn = __ldg(ex + ke); else eyn = __ldg(ey + ke);
           cidx = cidx_of(cx, cy);
           draw = dload(cx, cy, cidx);                 // new cell's density
-          enext = ev;
-          eax = ax ? 0 : 1;
           nf += 1u;
         } else {
           // ---- census ----
@@ -371,8 +378,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           active = false;
         }
       }
-      const unsigned idle_now = __ballot_sync(kFull, !active);
-      if (idle_now == kFull || (!exhausted && __popc(idle_now) >= refill_min)) break;
+      if (__popc(__ballot_sync(kFull, !active)) >= thr) break;
     }
   }
 
@@ -400,33 +406,39 @@ history_kernel(const __grid_constant__ TrackParams P) {
 }
 
 // Instantiations: deterministic/production x density format x layout x block map; the
-// production u8 + block-map kernels also come with a 64-register cap (4 CTAs per SM,
-// selected by ctas_per_sm = 4; the default is 80 registers, 3 CTAs per SM).
+// production u8 + block-map kernels also come with a 72-register cap (7 CTAs per SM,
+// selected by ctas_per_sm = 7; the default is 80 registers, 6 CTAs per SM) and with
+// warp-aggregated flushes (tally_mode 1).
 template <bool kDet, bool kTiled>
-static void* history_fn(int fmt, bool blk, int minb) {
+static void* history_fn(int fmt, bool blk, int minb, int agg) {
   if (fmt == kDensU8) {
-    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 3>;
-    if (!kDet && minb >= 4) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 4>;
-    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 3>;
+    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false>;
+    if constexpr (!kDet) {
+      if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false>;
+      if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true>;
+    }
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false>;
   }
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 3>;
-  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 3>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false>;
 }
 
-static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb) {
-  if (det) return tiled ? history_fn<true, true>(fmt, blk, minb) : history_fn<true, false>(fmt, blk, minb);
-  return tiled ? history_fn<false, true>(fmt, blk, minb) : history_fn<false, false>(fmt, blk, minb);
+static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg) {
+  if (det) return tiled ? history_fn<true, true>(fmt, blk, minb, agg) : history_fn<true, false>(fmt, blk, minb, agg);
+  return tiled ? history_fn<false, true>(fmt, blk, minb, agg) : history_fn<false, false>(fmt, blk, minb, agg);
 }
 
-void launch_history(const TrackParams& tp, bool det, int grid, int minb, cudaStream_t s) {
-  void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb);
+void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
+                    cudaStream_t s) {
+  void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
+                            tally_mode);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
 
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb) {
   int n = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb),
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, 0),
                                                 kHistoryBlock, 0);
   return n;
 }

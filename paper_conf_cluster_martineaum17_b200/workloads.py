@@ -84,6 +84,9 @@ CONFIGS: dict[str, Config] = {
     "stream": Config("stream", 4000, 4000, "uniform_lo", (0.45, 0.45, 0.1, 0.1), 1_000_000, 21),
     "stream_8m": Config("stream_8m", 4000, 4000, "uniform_lo", (0.45, 0.45, 0.1, 0.1), 1 << 23, 21),
     "scatter": Config("scatter", 4000, 4000, "uniform_hi", (0.45, 0.45, 0.1, 0.1), 10_000_000, 31),
+    # scatter's atomic-contention sweep: source side 0.5 / 0.01 m
+    "scatter_src050": Config("scatter_src050", 4000, 4000, "uniform_hi", (0.25, 0.25, 0.5, 0.5), 10_000_000, 32),
+    "scatter_src001": Config("scatter_src001", 4000, 4000, "uniform_hi", (0.495, 0.495, 0.01, 0.01), 10_000_000, 33),
     "split": Config("split", 4000, 4000, "split", (0.0, 0.0, 1.0, 1.0), 1 << 23, 41),
     # test-only problems
     "tiny_vacuum": Config("tiny_vacuum", 64, 64, "zero", (0.4, 0.4, 0.2, 0.2), 1000, 3, _SINGLE),
@@ -109,6 +112,8 @@ CONFIGS: dict[str, Config] = {
     # both uniform and mixed blocks (block sides 4 and 8)
     "tiny_mosaic": Config("tiny_mosaic", 70, 50, "mosaic", (0.1, 0.1, 0.8, 0.8), 2000, 18, _SINGLE, rho=2.0),
     "small_mosaic": Config("small_mosaic", 601, 590, "mosaic", (0.2, 0.2, 0.6, 0.6), 3000, 19, rho=0.5),
+    # every particle born in one cell of a dense medium: maximal tally contention
+    "tiny_hotspot": Config("tiny_hotspot", 64, 64, "uniform_hi", (0.5, 0.5, 0.01, 0.01), 10_000, 20, _SINGLE),
     "small_csp": Config("small_csp", 256, 256, "csp", (0.0, 0.0, 0.1, 0.1), 4096, 10),
     "small_scatter": Config("small_scatter", 256, 256, "uniform_hi", (0.45, 0.45, 0.1, 0.1), 8192, 12),
 }

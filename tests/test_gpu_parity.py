@@ -104,7 +104,7 @@ def test_inject_matches_oracle(nt, orc, cfgname):
 # ---------------------------------------------------------------------------------------------
 TINY = ["tiny_csp", "tiny_stream", "tiny_split", "tiny_vacuum", "tiny_vacuum_lo", "tiny_scatter_1g",
         "tiny_wkill", "tiny_A12", "tiny_mid", "tiny_thin", "tiny_absorber", "small_csp", "small_scatter",
-        "tiny_levels", "small_random", "tiny_mosaic", "small_mosaic"]
+        "tiny_levels", "small_random", "tiny_mosaic", "small_mosaic", "tiny_hotspot"]
 
 
 @pytest.mark.parametrize("mode", MODES)
@@ -131,6 +131,18 @@ def test_parity_production_atomic(nt, orc, cfgname, mode, density_format, layout
                              layout=layout)
     ot, op, (os_,) = orc.run(cfg)
     compare_particles(gp, op)                  # per-particle results do not depend on the tally
+    compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+    compare_stats(gs, os_, rtol=1e-9)
+
+
+@pytest.mark.parametrize("mode", MODES)
+@pytest.mark.parametrize("cfgname", ["tiny_hotspot", "tiny_scatter_1g", "tiny_mosaic", "tiny_csp"])
+def test_parity_warp_aggregated_tally(nt, orc, cfgname, mode):
+    """tally_mode 1: same-cell flushes of a warp summed with shuffles, one atomic per cell."""
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, tally_mode=1)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)
     compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
     compare_stats(gs, os_, rtol=1e-9)
 
