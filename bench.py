@@ -176,6 +176,8 @@ def parse():
     ap.add_argument("--density-format", type=int, default=0,
                     help="0 u8/u16 codes + block map (default), 1 f64 map, 2 codes without block map")
     ap.add_argument("--tally-mode", type=int, default=0, help="0 one RED per flush, 1 warp-aggregated")
+    ap.add_argument("--defer-below", type=int, default=0,
+                    help="collision deferral threshold (0 default 8, 1 off, 33 park every collision)")
     ap.add_argument("--json-out", default=None)
     ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
     return ap.parse_args()
@@ -253,7 +255,7 @@ def main():
                          nranks=world, unique_id=uid, A=cfg.A, molar_mass=cfg.molar_mass,
                          e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm,
                          refill_min=a.refill_min, layout=a.layout, density_format=a.density_format,
-                         tally_mode=a.tally_mode)
+                         tally_mode=a.tally_mode, defer_below=a.defer_below)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -343,6 +345,7 @@ def main():
                        "layout": "tiled4x4" if a.layout == 0 else "row-major",
                        "density_format": ["codes+block map", "f64", "codes"][a.density_format],
                        "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED"][a.tally_mode],
+                       "defer_below": a.defer_below or 8,
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
                        "tables": [len(tables[0]), len(tables[2])],
                        "parallelism": f"dp{world} (particle id shards, tally NCCL allreduce)",

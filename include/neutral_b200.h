@@ -33,7 +33,7 @@
 extern "C" {
 #endif
 
-#define NT_ABI_VERSION 1
+#define NT_ABI_VERSION 2
 
 typedef struct nt_ctx nt_ctx;
 
@@ -92,6 +92,14 @@ typedef struct {
                                   into the same cell at the same time are summed with warp
                                   shuffles and one lane issues the atomic (history mode,
                                   u8 block-map meshes; others fall back to 0)              */
+    int32_t defer_below;       /* history mode, collision deferral: a lane whose next event
+                                  is a collision while fewer than this many lanes of its
+                                  warp collide is parked (state to the particle store) and
+                                  resumed by a second launch of the tracking kernel, where
+                                  such particles -- mostly inside dense matter -- collide
+                                  together.  Results are unchanged.  0 -> 8; 1 disables;
+                                  at most 33 (33: park every collision)                    */
+    int32_t pad0;
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

@@ -41,7 +41,8 @@ class Options(C.Structure):
                 ("max_events_per_history", C.c_int64), ("block_size", C.c_int32),
                 ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64),
                 ("refill_min", C.c_int32), ("density_format", C.c_int32),
-                ("layout", C.c_int32), ("tally_mode", C.c_int32)]
+                ("layout", C.c_int32), ("tally_mode", C.c_int32),
+                ("defer_below", C.c_int32), ("pad0", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -145,7 +146,8 @@ class Tracker:
                  unique_id: bytes | None = None, A: float = 1.0, molar_mass: float = 1e-3,
                  e_min: float = 1.0, w_min: float = 1e-3, max_events: int = 0,
                  ctas_per_sm: int = 0, det_batch: int = 0, refill_min: int = 0,
-                 density_format: int = 0, layout: int = 0, tally_mode: int = 0):
+                 density_format: int = 0, layout: int = 0, tally_mode: int = 0,
+                 defer_below: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -164,6 +166,7 @@ class Tracker:
         o.density_format = density_format
         o.layout = layout
         o.tally_mode = tally_mode
+        o.defer_below = defer_below
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:

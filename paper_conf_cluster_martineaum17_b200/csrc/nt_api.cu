@@ -76,6 +76,7 @@ struct nt_ctx {
   uint64_t seed = 0;
   DevBuf soa;
   Soa p{};
+  int32_t* defer_q = nullptr;            // collision-deferral queue (in soa)
   // step scratch: [counter][stats_u][stats_f]; per-thread f64 statistic slots
   DevBuf scratch, slots;
   // deterministic mode
@@ -188,6 +189,7 @@ nt_status nt_options_default(nt_options* opt) {
   opt->max_events_per_history = 1000000000ll;
   opt->det_batch = 65536;
   opt->refill_min = 8;
+  opt->defer_below = 8;
   return NT_OK;
 }
 
@@ -221,6 +223,8 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.det_batch > 65536) opt.det_batch = 65536;
   if (opt.refill_min <= 0) opt.refill_min = def.refill_min;
   if (opt.refill_min > 32) opt.refill_min = 32;
+  if (opt.defer_below == 0) opt.defer_below = def.defer_below;
+  if (opt.defer_below < 0 || opt.defer_below > 33) return NT_ERR_ARG;
   if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
       opt.rank < 0 || opt.rank >= opt.nranks || opt.density_format < 0 ||
@@ -485,17 +489,18 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
 static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   const size_t N = (size_t)(n > 0 ? n : 1);
   const size_t b8 = align256(N * 8), b4 = align256(N * 4), b1 = align256(N);
-  cudaError_t e = c->soa.ensure(8 * b8 + 6 * b4 + b1);
+  // 8 + 3 f64 columns, 6 + 3 u32 columns, the deferral queue, status
+  cudaError_t e = c->soa.ensure(11 * b8 + 10 * b4 + b1);
   if (e != cudaSuccess) return e;
   char* q = c->soa.as<char>();
-  double** d8[8] = {&c->p.x, &c->p.y, &c->p.ox, &c->p.oy, &c->p.e, &c->p.w, &c->p.mfp, &c->p.dep};
+  double** d8[11] = {&c->p.x, &c->p.y, &c->p.ox, &c->p.oy, &c->p.e, &c->p.w, &c->p.mfp, &c->p.dep,
+                     &c->p.dcen, &c->p.acc, &c->p.dstep};
   for (auto d : d8) { *d = reinterpret_cast<double*>(q); q += b8; }
+  uint32_t** d4[7] = {&c->p.ctr, &c->p.nfac, &c->p.ncol, &c->p.ncen, &c->p.nf_s, &c->p.nc_s, &c->p.seq_s};
   c->p.cx = reinterpret_cast<int32_t*>(q); q += b4;
   c->p.cy = reinterpret_cast<int32_t*>(q); q += b4;
-  c->p.ctr = reinterpret_cast<uint32_t*>(q); q += b4;
-  c->p.nfac = reinterpret_cast<uint32_t*>(q); q += b4;
-  c->p.ncol = reinterpret_cast<uint32_t*>(q); q += b4;
-  c->p.ncen = reinterpret_cast<uint32_t*>(q); q += b4;
+  for (auto d : d4) { *d = reinterpret_cast<uint32_t*>(q); q += b4; }
+  c->defer_q = reinterpret_cast<int32_t*>(q); q += b4;
   c->p.status = reinterpret_cast<uint8_t*>(q);
   return cudaSuccess;
 }
@@ -621,8 +626,21 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
     if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
     return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
   }
-  launch_history(bp, det, history_grid(c, det), c->opt.ctas_per_sm, c->opt.tally_mode, c->stream);
-  ++launches;
+  // phase 1: particles [lo, hi), parking lonely collisions; phase 2: the parked particles
+  char* s = c->scratch.as<char>();
+  NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 16, c->stream));     // queue length, phase-2 counter
+  TrackParams p1 = bp;
+  p1.phase = 1;
+  p1.defer_below = c->opt.defer_below;
+  p1.defer_q = c->defer_q;
+  p1.defer_count = reinterpret_cast<unsigned long long*>(s + 16);
+  const int grid = history_grid(c, det);
+  launch_history(p1, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->stream);
+  TrackParams p2 = p1;
+  p2.phase = 2;
+  p2.counter = reinterpret_cast<unsigned long long*>(s + 24);
+  launch_history(p2, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->stream);
+  launches += 2;
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;
 }
@@ -733,8 +751,6 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   float reduce_ms = 0.f;
   if (c->comm) {
     // small stats allreduce through the same communicator
-    double* d = reinterpret_cast<double*>(c->scratch.as<char>() + 768 - 8 * 0);
-    (void)d;
     DevBuf tmp;
     NT_CUDA(c, tmp.ensure(sizeof hs));
     NT_CUDA(c, cudaMemcpyAsync(tmp.p, hs, sizeof hs, cudaMemcpyHostToDevice, c->stream));
@@ -746,7 +762,6 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
     ncclResult_t async_err;
     ncclCommGetAsyncError(c->comm, &async_err);
     if (async_err != ncclSuccess) return fail(c, NT_ERR_NCCL, "NCCL async error: %s", ncclGetErrorString(async_err));
-    launches += 0;
   }
   float track_ms = 0.f, step_ms = 0.f;
   cudaEventElapsedTime(&track_ms, c->ev[1], c->ev[2]);

@@ -24,7 +24,10 @@ struct Soa {
   double *x, *y, *ox, *oy, *e, *w, *mfp, *dep;
   int32_t *cx, *cy;
   uint32_t *ctr, *nfac, *ncol, *ncen;
-  uint8_t *status;
+  uint8_t *status;             // 1 alive (at census), 0 dead, 2 parked mid-step (deferral)
+  // mid-step state of a particle parked by the history kernel's collision deferral
+  double *dcen, *acc, *dstep;  // census distance left, pending deposit, deposits flushed
+  uint32_t *nf_s, *nc_s, *seq_s;   // facets, collisions, flush records so far this step
 };
 
 // Density storage (lossless): the f64 map, or -- when the map holds <= 256 (65536) distinct

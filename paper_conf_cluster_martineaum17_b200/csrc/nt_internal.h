@@ -20,6 +20,10 @@ struct TrackParams {
   double dt;
   int64_t max_events;
   int32_t refill_min;         // refill a warp's idle lanes once at least this many are idle
+  int32_t phase;              // history kernel: 1 track [lo, hi) (may park), 2 resume parked
+  int32_t defer_below;        // phase 1 parks a colliding lane while fewer lanes collide
+  int32_t* defer_q;           // parked local indices
+  unsigned long long* defer_count;
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]

@@ -153,6 +153,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
   uint32_t cidx = 0;         // storage index of (cx, cy)
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
 
+  // Collision deferral: phase 1 tracks particles [lo, hi) and parks a lane
+  // whose next event is a collision while fewer than defer_below lanes of its warp collide
+  // (its state goes to the particle store, its index to the deferred queue, the lane takes
+  // a new particle); phase 2 resumes the queued particles -- mostly in dense matter, so
+  // their collisions run warp-converged.  Per-particle results are unchanged.
+  const bool resume = P.phase == 2;
+  const unsigned long long span2 = resume ? *P.defer_count : span;
+  const int defer_below = resume ? 0 : P.defer_below;
   int thr = refill_min;   // break the event loop once this many lanes are idle (32: all)
   for (;;) {
     // ---- refill idle lanes with new particles: one atomic per warp ----
@@ -162,15 +170,15 @@ history_kernel(const __grid_constant__ TrackParams P) {
       unsigned long long base = 0;
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
       base = __shfl_sync(kFull, base, leader);
-      if (base + (unsigned long long)__popc(idle) >= span) {
+      if (base + (unsigned long long)__popc(idle) >= span2) {
         exhausted = true;
         thr = 32;
       }
       if (!active) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
-        if (my < span) {
-          i = (int32_t)(P.lo + (int64_t)my);
-          if (P.p.status[i] == 1u) {
+        if (my < span2) {
+          i = resume ? P.defer_q[my] : (int32_t)(P.lo + (int64_t)my);
+          if (P.p.status[i] == (resume ? 2u : 1u)) {
             active = true;
             x = ld_stream(P.p.x + i, pol_stream);
             y = ld_stream(P.p.y + i, pol_stream);
@@ -186,18 +194,29 @@ history_kernel(const __grid_constant__ TrackParams P) {
             draw = dload(cx, cy, cidx);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
-            m = refresh_xs(P.xs, ph, e, nrange);
-            dcen = speed(e, ph) * P.dt;
             iox = 1.0 / ox;
             ioy = 1.0 / oy;
             if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
             if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
-            acc = 0.0;
-            dstep = 0.0;
-            nf = 0u;
-            nc = 0u;
-            seq = 0u;
-            cnt(SU_ALIVE, 1u);
+            if (!resume) {
+              m = refresh_xs(P.xs, ph, e, nrange);
+              dcen = speed(e, ph) * P.dt;
+              acc = 0.0;
+              dstep = 0.0;
+              nf = 0u;
+              nc = 0u;
+              seq = 0u;
+              cnt(SU_ALIVE, 1u);
+            } else {                 // the parked state (phase 1 counted the XS clamps)
+              uint32_t nr_dummy = 0;
+              m = refresh_xs(P.xs, ph, e, nr_dummy);
+              dcen = P.p.dcen[i];
+              acc = P.p.acc[i];
+              dstep = P.p.dstep[i];
+              nf = P.p.nf_s[i];
+              nc = P.p.nc_s[i];
+              seq = P.p.seq_s[i];
+            }
           }
         }
       }
@@ -269,6 +288,32 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_KILLED_E, w * e);
           fsum(SF_KILLED_W, w);
           outcome = 2;
+        } else if (coll && __popc(__activemask()) < defer_below) {
+          // ---- park for phase 2: the state before this event, index into the queue ----
+          P.p.x[i] = x;
+          P.p.y[i] = y;
+          P.p.ox[i] = ox;
+          P.p.oy[i] = oy;
+          P.p.e[i] = e;
+          P.p.w[i] = w;
+          P.p.mfp[i] = mfp;
+          P.p.cx[i] = cx;
+          P.p.cy[i] = cy;
+          P.p.ctr[i] = ctr;
+          P.p.dcen[i] = dcen;
+          P.p.acc[i] = acc;
+          P.p.dstep[i] = dstep;
+          P.p.nf_s[i] = nf;
+          P.p.nc_s[i] = nc;
+          P.p.seq_s[i] = seq;
+          P.p.status[i] = 2u;
+          const unsigned am = __activemask();
+          const int ld = __ffs(am) - 1;
+          unsigned long long q = 0;
+          if (lane == ld) q = atomicAdd(P.defer_count, (unsigned long long)__popc(am));
+          q = __shfl_sync(am, q, ld) + (unsigned long long)__popc(am & lt_mask);
+          P.defer_q[q] = i;
+          active = false;
         } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
           acc += ((w * dc) * sig) * m.H;
@@ -369,6 +414,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           st_stream(P.p.ncol + i, ld_stream(P.p.ncol + i, pol_stream) + nc, pol_stream);
           if (outcome == 1) {
             P.p.ncen[i] += 1u;
+            if (resume) P.p.status[i] = 1u;           // was parked (2)
           } else {
             P.p.status[i] = 0u;
           }

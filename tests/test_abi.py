@@ -40,7 +40,7 @@ def test_exports_every_declared_symbol(L):
 
 def test_identity_calls(L):
     from paper_conf_cluster_martineaum17_b200 import binding
-    assert L.nt_abi_version() == 1
+    assert L.nt_abi_version() == 2
     assert b"sm_100a" in L.nt_build_info()
     assert b"-fmad=false" in L.nt_build_info()
     for k, v in binding.STATUS.items():
@@ -49,6 +49,7 @@ def test_identity_calls(L):
     assert L.nt_options_default(C.byref(o)) == 0
     assert o.nranks == 1 and o.A == 1.0 and o.e_min == 1.0 and o.w_min == 1e-3
     assert o.max_events_per_history == 10**9 and o.det_batch == 65536 and o.refill_min == 8
+    assert o.defer_below == 8
 
 
 def test_struct_layouts_match_header():

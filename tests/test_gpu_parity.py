@@ -147,6 +147,20 @@ def test_parity_warp_aggregated_tally(nt, orc, cfgname, mode):
     compare_stats(gs, os_, rtol=1e-9)
 
 
+@pytest.mark.parametrize("defer_below", [1, 4, 33])
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_split", "tiny_mid", "small_csp", "tiny_mosaic"])
+def test_parity_collision_deferral(nt, orc, cfgname, defer_below):
+    """History mode with collision deferral off (1), at 4, and parking every collision (33):
+    per-particle results and the deterministic tally are unchanged."""
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=True, defer_below=defer_below)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)
+    compare_tally(gt, ot)
+    compare_stats(gs, os_)
+    assert np.all(gp["status"] <= 1)
+
+
 @pytest.mark.parametrize("mode", MODES)
 def test_parity_two_steps_and_shard(nt, orc, mode):
     cfg = wl.CONFIGS["tiny_split"]
