@@ -355,6 +355,11 @@ def main():
             "event_mix": {"facets": s0["n_facets"], "collisions": s0["n_collisions"],
                           "census": s0["n_census"], "killed": s0["n_killed"]},
             "status": sorted(status),
+            # per-event grind time (the paper's 3 ns/facet on stream, 18 ns/collision on
+            # scatter, were measured on a Xeon): tracking time / events this rank
+            "grind_ns": {"per_event": track_ms * 1e6 * world / max(1.0, events / a.steps),
+                         "per_facet_if_all_facets": track_ms * 1e6 * world / max(1, s0["n_facets"]),
+                         "per_collision_if_all_collisions": track_ms * 1e6 * world / max(1, s0["n_collisions"])},
             "roofline": {"bound": "hbm", "kernel": f"history_kernel<false>" if a.mode == "history" else "event kernels",
                          "achieved": achieved, "peak": peaks["hbm_gbs"], "unit": "GB/s",
                          "frac": achieved / peaks["hbm_gbs"], "traffic": traffic,

@@ -13,6 +13,7 @@
 // last compaction block sets the loop condition with cudaGraphSetConditional).
 // Arithmetic: DESIGN.md §3, identical to the history kernel, so per-particle results
 // match it (and the oracle) bit for bit.
+#include <cstdlib>
 #include <cstring>
 #include <cub/device/device_radix_sort.cuh>
 
@@ -252,7 +253,7 @@ constexpr int kCompactItems = 8;
 
 __global__ void __launch_bounds__(kEvBlock)
 ev_compact_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, EvCtl* ctl,
-                  cudaGraphConditionalHandle h) {
+                  cudaGraphConditionalHandle h, int in_graph) {
   __shared__ unsigned s_wsum[3][kEvBlock / 32];
   __shared__ unsigned s_base[3];
   __shared__ bool s_last;
@@ -322,7 +323,7 @@ ev_compact_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, EvCt
     }
     vc->done = 0u;
     vc->iter = vc->iter + 1u;
-    cudaGraphSetConditional(h, tot > 0u ? 1u : 0u);
+    if (in_graph) cudaGraphSetConditional(h, tot > 0u ? 1u : 0u);
   }
 }
 
@@ -606,7 +607,8 @@ static cudaError_t build_graph(EventState* s, bool det, int fmt, int sm_count) {
   unsigned long long* su = s->slot_u;
   double* sf = s->slot_f;
 
-  void* cmp_args[] = {&tp, &cols, &qs, &ctl, &h};
+  int in_graph = 1;
+  void* cmp_args[] = {&tp, &cols, &qs, &ctl, &h, &in_graph};
   cudaKernelNodeParams kc;
   std::memset(&kc, 0, sizeof kc);
   kc.func = (void*)ev_compact_kernel;
@@ -627,6 +629,39 @@ static cudaError_t build_graph(EventState* s, bool det, int fmt, int sm_count) {
   e = cudaGraphAddKernelNode(&n_step, body, &n_cmp, 1, &kp);
   if (e != cudaSuccess) return e;
   return cudaGraphInstantiate(&s->exec, s->graph, 0);
+}
+
+static cudaError_t host_loop(EventState* s, bool det, int fmt, int sm_count, cudaStream_t st,
+                             uint32_t& launches) {
+  int per_sm_c = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm_c, ev_compact_kernel, kEvBlock, 0);
+  if (per_sm_c < 1) per_sm_c = 1;
+  const int grid_c = sm_count * (per_sm_c < 4 ? per_sm_c : 4);
+  const TrackParams* tp = s->d_tp;
+  EvCols cols = s->cols;
+  EvQueues qs = s->qs;
+  EvCtl* ctl = s->ctl;
+  const EvCtl* cctl = s->ctl;
+  unsigned long long* su = s->slot_u;
+  double* sf = s->slot_f;
+  cudaGraphConditionalHandle h = 0;
+  int in_graph = 0;
+  void* cmp_args[] = {&tp, &cols, &qs, &ctl, &h, &in_graph};
+  void* step_args[] = {&tp, &cols, &qs, &cctl, &su, &sf};
+  for (;;) {
+    for (int k = 0; k < 64; ++k) {
+      cudaError_t e = cudaLaunchKernel((void*)ev_compact_kernel, dim3(grid_c), dim3(kEvBlock), cmp_args, 0, st);
+      if (e == cudaSuccess)
+        e = cudaLaunchKernel(ev_fn(det, fmt, true), dim3(s->grid), dim3(kEvBlock), step_args, 0, st);
+      if (e != cudaSuccess) return e;
+      launches += 2;
+    }
+    EvCtl hc;
+    cudaError_t e = cudaMemcpyAsync(&hc, s->ctl, sizeof hc, cudaMemcpyDeviceToHost, st);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(st);
+    if (e != cudaSuccess) return e;
+    if (hc.cur[0] + hc.cur[1] + hc.cur[2] == 0u) return cudaSuccess;
+  }
 }
 
 // One particle range [tp.lo, tp.hi): zero the stat slots, ev_init, the graph loop, and the
@@ -664,8 +699,14 @@ nt_status event_run_range(EventState* s, const TrackParams& tp, bool det, int sm
     e = cudaLaunchKernel(ev_fn(det, tp.mesh.fmt, false), dim3((unsigned)blocks), dim3(kEvBlock),
                          args, 0, st);
     ++launches;
-    if (e == cudaSuccess) e = cudaGraphLaunch(s->exec, st);
-    launches += 2;     // >= one [ev_compact, ev_step] iteration; the rest run inside the graph
+    if (std::getenv("NT_EVENT_HOST_LOOP") == nullptr) {
+      if (e == cudaSuccess) e = cudaGraphLaunch(s->exec, st);
+      launches += 2;   // >= one [ev_compact, ev_step] iteration; the rest run inside the graph
+    } else {
+      // profiling aid (ncu cannot see kernels inside a conditional graph): the same two
+      // kernels launched from the host, 64 iterations between checks of the queue lengths
+      e = host_loop(s, det, tp.mesh.fmt, sm_count, st, launches);
+    }
     if (e != cudaSuccess) { err = cudaGetErrorString(e); return NT_ERR_CUDA; }
   }
   ev_stats_kernel<<<SU_COUNT + SF_COUNT, 256, 0, st>>>(s->slot_u, s->slot_f, tp.stats_u,

@@ -1,8 +1,25 @@
-set -x
-mkdir -p gpurun_out/r01
+# usage: bash scripts/gpu_round.sh TAG -- the round's evidence: GPU tests, default bench (csp, with
+# cpu_baseline + e2e), the other configs, launch list, ncu --set full of csp/stream history.
+TAG=${1:-round}
+OUT=gpurun_out/$TAG
+mkdir -p $OUT
 python -c "import __graft_entry__ as g; g.build()"
-python bench.py --json-out gpurun_out/r01/bench_csp.json 2>&1 | tail -3
-for c in stream scatter split; do python bench.py --config $c --no-cpu-baseline --no-e2e --steps 5 --json-out gpurun_out/r01/bench_$c.json 2>&1 | tail -2; done
-ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-file gpurun_out/r01/launches_csp.csv python bench.py --steps 2 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/r01/ncu_launch_bench.log 2>&1
-ncu --set full --clock-control none --import-source on -k regex:history -s 1 -c 1 -o gpurun_out/r01/prof_csp_history python bench.py --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/r01/ncu_full.log 2>&1
-ls -la gpurun_out/r01
+timeout 1200 python -m pytest tests -m gpu -x -q -p no:cacheprovider > $OUT/pytest_gpu.log 2>&1
+tail -1 $OUT/pytest_gpu.log | sed "s/^/PYTEST: /"
+python bench.py --json-out $OUT/bench_csp.json > $OUT/bench_csp.log 2>&1
+for c in stream scatter split stream_8m; do
+  python bench.py --config $c --no-cpu-baseline --no-e2e --steps 5 --json-out $OUT/bench_$c.json > $OUT/bench_$c.log 2>&1
+done
+for c in csp stream scatter split; do
+  python bench.py --config $c --mode event --no-cpu-baseline --no-e2e --steps 3 --json-out $OUT/bench_${c}_event.json > $OUT/bench_${c}_event.log 2>&1
+done
+for f in $OUT/bench_*.json; do python -c "
+import json; d=json.load(open('$f')); r=d['roofline']
+print('$f'.split('/')[-1], f\"value={d['value']:.3e} ms={d['ms_per_step']:.2f} frac={r['frac']:.3f} clocks={d['clocks']['sm_mhz']}\")"; done
+ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-file $OUT/launches_csp.csv \
+    python bench.py --steps 2 --warmup 1 --no-cpu-baseline --no-e2e > $OUT/ncu_launch_bench.log 2>&1
+for c in csp stream; do
+  ncu --set full --clock-control none --import-source on -k regex:history -s 2 -c 2 \
+      -o $OUT/prof_${c} python bench.py --config $c --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > $OUT/ncu_$c.log 2>&1
+done
+ls $OUT
