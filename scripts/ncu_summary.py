@@ -46,7 +46,7 @@ def main():
     raw = list(csv.reader(io.StringIO(ncu(["-i", a.rep, "--page", "raw", "--csv"]))))
     hdr, units, rows = raw[0], raw[1], raw[2:]
     lines = [f"# ncu summary: {Path(a.rep).name}", ""]
-    traffic = None
+    traffic = 0.0      # summed over the captured launches (history phases 1 + 2 of one step)
     for r in rows:
         d = dict(zip(hdr, r))
         u = dict(zip(hdr, units))
@@ -77,9 +77,12 @@ def main():
             un = u.get(k, "")
             mult = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "Tbyte": 1e12}.get(un, 1)
             return f * mult
-        traffic = num("dram__bytes_read.sum", 1) + num("dram__bytes_write.sum", 1)
+        tr = num("dram__bytes_read.sum", 1) + num("dram__bytes_write.sum", 1)
+        traffic += tr
         lines.append("")
-        lines.append(f"DRAM traffic per launch (read + write): {traffic:.4g} B")
+        lines.append(f"DRAM traffic of this launch (read + write): {tr:.4g} B")
+        lines.append("")
+    lines.append(f"DRAM traffic of all captured launches: {traffic:.4g} B")
     # source page: top stall-sampled SASS lines
     try:
         src = list(csv.reader(io.StringIO(ncu(["-i", a.rep, "--page", "source", "--csv",
