@@ -178,6 +178,10 @@ def parse():
     ap.add_argument("--tally-mode", type=int, default=0, help="0 one RED per flush, 1 warp-aggregated")
     ap.add_argument("--defer-below", type=int, default=0,
                     help="collision deferral threshold (0 default 8, 1 off, 33 park every collision)")
+    ap.add_argument("--xs-search", type=int, default=0,
+                    help="0 bucketed binary search, 1 plain binary search, 2 cached-bin linear walk")
+    ap.add_argument("--table-size", type=int, default=0,
+                    help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
     ap.add_argument("--json-out", default=None)
     ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
     return ap.parse_args()
@@ -242,6 +246,9 @@ def main():
     cfg = wl.CONFIGS[a.config]
     if a.mesh:
         cfg = cfg.with_(nx=a.mesh, ny=a.mesh, name=f"{cfg.name}@{a.mesh}")
+    if a.table_size:
+        cfg = cfg.with_(tables=wl.Tables(n_scatter=a.table_size, n_capture=max(2, 3 * a.table_size // 4)),
+                        name=f"{cfg.name}@xs{a.table_size}")
     n_per = cfg.n_particles
     n_total = n_per * world
     first_id = rank * n_per
@@ -255,7 +262,8 @@ def main():
                          nranks=world, unique_id=uid, A=cfg.A, molar_mass=cfg.molar_mass,
                          e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm,
                          refill_min=a.refill_min, layout=a.layout, density_format=a.density_format,
-                         tally_mode=a.tally_mode, defer_below=a.defer_below)
+                         tally_mode=a.tally_mode, defer_below=a.defer_below,
+                         xs_search=a.xs_search)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -346,6 +354,7 @@ def main():
                        "density_format": ["codes+block map", "f64", "codes"][a.density_format],
                        "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED"][a.tally_mode],
                        "defer_below": a.defer_below or 8,
+                       "xs_search": ["bucketed binary", "binary", "cached-bin walk"][a.xs_search],
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
                        "tables": [len(tables[0]), len(tables[2])],
                        "parallelism": f"dp{world} (particle id shards, tally NCCL allreduce)",

@@ -99,7 +99,12 @@ typedef struct {
                                   such particles -- mostly inside dense matter -- collide
                                   together.  Results are unchanged.  0 -> 8; 1 disables;
                                   at most 33 (33: park every collision)                    */
-    int32_t pad0;
+    int32_t xs_search;         /* cross-section bin search: 0 a bucket
+                                  index over the keys' bit patterns narrows a binary search;
+                                  1 plain binary search over the table; 2 the paper's
+                                  cached-index search -- a linear walk from the particle's
+                                  previous bin (history mode, u8 block-map meshes; others
+                                  use 0).  All three return the same bin.                 */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

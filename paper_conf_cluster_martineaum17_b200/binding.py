@@ -42,7 +42,7 @@ class Options(C.Structure):
                 ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64),
                 ("refill_min", C.c_int32), ("density_format", C.c_int32),
                 ("layout", C.c_int32), ("tally_mode", C.c_int32),
-                ("defer_below", C.c_int32), ("pad0", C.c_int32)]
+                ("defer_below", C.c_int32), ("xs_search", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -147,7 +147,7 @@ class Tracker:
                  e_min: float = 1.0, w_min: float = 1e-3, max_events: int = 0,
                  ctas_per_sm: int = 0, det_batch: int = 0, refill_min: int = 0,
                  density_format: int = 0, layout: int = 0, tally_mode: int = 0,
-                 defer_below: int = 0):
+                 defer_below: int = 0, xs_search: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -167,6 +167,7 @@ class Tracker:
         o.layout = layout
         o.tally_mode = tally_mode
         o.defer_below = defer_below
+        o.xs_search = xs_search
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:

@@ -225,6 +225,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.refill_min > 32) opt.refill_min = 32;
   if (opt.defer_below == 0) opt.defer_below = def.defer_below;
   if (opt.defer_below < 0 || opt.defer_below > 33) return NT_ERR_ARG;
+  if (opt.xs_search < 0 || opt.xs_search > 2) return NT_ERR_ARG;
   if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
       opt.rank < 0 || opt.rank >= opt.nranks || opt.density_format < 0 ||
@@ -566,6 +567,10 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.mesh.nx = c->nx;
   tp.mesh.ny = c->ny;
   tp.xs = c->tables;
+  if (c->opt.xs_search == 1) {          // plain binary search over the whole table
+    tp.xs.s.nb = 0;
+    tp.xs.c.nb = 0;
+  }
   tp.ph = c->ph;
   tp.p = c->p;
   tp.n = c->n_local;
@@ -635,11 +640,11 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
   p1.defer_q = c->defer_q;
   p1.defer_count = reinterpret_cast<unsigned long long*>(s + 16);
   const int grid = history_grid(c, det);
-  launch_history(p1, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->stream);
+  launch_history(p1, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
   TrackParams p2 = p1;
   p2.phase = 2;
   p2.counter = reinterpret_cast<unsigned long long*>(s + 24);
-  launch_history(p2, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->stream);
+  launch_history(p2, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
   launches += 2;
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;

@@ -60,11 +60,13 @@ constexpr uint32_t kBlkMixed = 255u;   // block-map entry: block holds more than
 constexpr int kBlkMax = 16384;         // max block-map entries (bytes of shared memory)
 
 // Storage index of cell (cx, cy) in the tally and density arrays.  Tiled layout: 4x4-cell
-// tiles in row-major tile order, row-major inside a tile, so the 16 f64 tally cells of a
-// tile fill one 128 B line and a particle's consecutive facets (x or y) mostly stay in it.
+// tiles in row-major tile order, column-major inside a tile -- index
+// (cy/4)*(16*ntx) + 4*cx + cy%4 -- so the 16 f64 tally cells of a tile fill one 128 B line
+// and a particle's consecutive facets (x or y) mostly stay in it; the index costs one shift
+// and two integer multiply-adds.
 __device__ __forceinline__ int64_t cell_index(const Mesh& M, int32_t cx, int32_t cy) {
   if (M.tiled)
-    return ((int64_t)((cy >> 2) * M.ntx + (cx >> 2)) << 4) | (int64_t)(((cy & 3) << 2) | (cx & 3));
+    return (int64_t)(cy >> 2) * (16 * (int64_t)M.ntx) + ((int64_t)cx << 2) + (int64_t)(cy & 3);
   return (int64_t)cy * M.nx + cx;
 }
 
@@ -344,6 +346,59 @@ __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, doubl
   const double ea = clamp_count(e, T.c.k, T.c.n, nrange);
   const double ss = xs_lookup(T.s, es);
   const double sa = xs_lookup(T.c, ea);
+  const double t = ss + sa;
+  Mat m;
+  m.st = t * kBarn;
+  m.pa = t > 0.0 ? sa / t : 0.0;
+  const double rs = t > 0.0 ? ss / t : 0.0;
+  m.H = e - rs * (e * ph.f);
+  return m;
+}
+
+// ---- the paper's cached-index search: the bin of the last lookup is kept and
+// the new bin is found by a linear walk from it (energies only fall in elastic scatter
+// off a target at rest, so the walk goes down).  Same bin as xs_lookup by definition.
+__device__ __forceinline__ double clamp_only(double e, const Table& T) {
+  const double lo = __ldg(T.k), hi = __ldg(T.k + T.n - 1);
+  return e < lo ? lo : (e > hi ? hi : e);
+}
+
+// Bin of e (already in [k0, k_{N-1}]) by the bucketed binary search of xs_lookup.
+__device__ __forceinline__ int32_t xs_bin(const Table& T, double e) {
+  const double* __restrict__ k = T.k;
+  const int32_t n = T.n;
+  if (e >= __ldg(k + n - 1)) return n - 2;
+  int32_t lo = 0, hi = n - 1;
+  if (T.nb > 0) {
+    const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
+    lo = (int32_t)__ldg(T.idx + b);
+    hi = (int32_t)__ldg(T.idx + b + 1) + 1;
+  }
+  while (hi - lo > 1) {
+    const int32_t mid = (lo + hi) >> 1;
+    if (__ldg(k + mid) <= e) lo = mid; else hi = mid;
+  }
+  return lo;
+}
+
+__device__ __forceinline__ double xs_walk(const Table& T, double e, int32_t& bin) {
+  const double* __restrict__ k = T.k;
+  int32_t i = bin;
+  while (i > 0 && __ldg(k + i) > e) --i;
+  while (i < T.n - 2 && __ldg(k + i + 1) <= e) ++i;
+  bin = i;
+  const double k0 = __ldg(k + i), k1 = __ldg(k + i + 1);
+  const double v0 = __ldg(T.v + i), v1 = __ldg(T.v + i + 1);
+  const double t = (e - k0) / (k1 - k0);
+  return v0 + t * (v1 - v0);
+}
+
+__device__ __forceinline__ Mat refresh_xs_walk(const Tables& T, const Phys& ph, double e,
+                                               uint32_t& nrange, int32_t& bin_s, int32_t& bin_a) {
+  const double es = clamp_count(e, T.s.k, T.s.n, nrange);
+  const double ea = clamp_count(e, T.c.k, T.c.n, nrange);
+  const double ss = xs_walk(T.s, es, bin_s);
+  const double sa = xs_walk(T.c, ea, bin_a);
   const double t = ss + sa;
   Mat m;
   m.st = t * kBarn;

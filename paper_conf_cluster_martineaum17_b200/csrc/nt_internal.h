@@ -55,8 +55,10 @@ void launch_inject(const InjectParams& ip, cudaStream_t s);
 // instantiation; 128-thread CTAs with <= 80 registers (6 resident per SM), or -- minb = 7,
 // production u8 + block map only -- <= 72 registers (7 per SM).
 // tally_mode 1 (production u8 + block map only): warp-aggregated tally flushes.
+// xs_search 2 (u8 + block map only): the cached-bin linear walk; 1 is a data change (the
+// caller passes tables without bucket index, nb = 0).
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
-                    cudaStream_t s);
+                    int xs_search, cudaStream_t s);
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);

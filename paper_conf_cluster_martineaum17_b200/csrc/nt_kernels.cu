@@ -79,7 +79,7 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg>
+template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg, bool kXsWalk>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
   static_assert(!kBlk || kFmt == kDensU8, "the block map indexes u8 material codes");
@@ -122,12 +122,12 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
   const Phys& ph = P.ph;
   const int refill_min = P.refill_min;
-  const int32_t ntx = P.mesh.ntx;
-  // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, see nt_device.cuh cell_index
+  const uint32_t strip = 16u * (uint32_t)P.mesh.ntx;    // tiled: cells per row of tiles
+  // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, as nt_device.cuh cell_index
   // (32-bit: nt_init_mesh guarantees the storage fits 2^32 cells)
   auto cidx_of = [&](int32_t cx_, int32_t cy_) -> uint32_t {
     if constexpr (kTiled)
-      return ((uint32_t)((cy_ >> 2) * ntx + (cx_ >> 2)) << 4) | (uint32_t)(((cy_ & 3) << 2) | (cx_ & 3));
+      return (uint32_t)(cy_ >> 2) * strip + ((uint32_t)cx_ << 2) + (uint32_t)(cy_ & 3);
     else
       return (uint32_t)cy_ * (uint32_t)nx + (uint32_t)cx_;
   };
@@ -152,6 +152,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   int32_t cx = 0, cy = 0;
   uint32_t cidx = 0;         // storage index of (cx, cy)
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
+  int32_t bin_s = 0, bin_a = 0;   // kXsWalk: the bins of the last lookup
 
   // Collision deferral: phase 1 tracks particles [lo, hi) and parks a lane
   // whose next event is a collision while fewer than defer_below lanes of its warp collide
@@ -198,6 +199,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
             ioy = 1.0 / oy;
             if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
             if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
+            if constexpr (kXsWalk) {
+              bin_s = xs_bin(P.xs.s, clamp_only(e, P.xs.s));
+              bin_a = xs_bin(P.xs.c, clamp_only(e, P.xs.c));
+            }
             if (!resume) {
               m = refresh_xs(P.xs, ph, e, nrange);
               dcen = speed(e, ph) * P.dt;
@@ -348,7 +353,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             dcen = tcen * speed(e, ph);
-            m = refresh_xs(P.xs, ph, e, nrange);
+            if constexpr (kXsWalk) m = refresh_xs_walk(P.xs, ph, e, nrange, bin_s, bin_a);
+            else m = refresh_xs(P.xs, ph, e, nrange);
             iox = 1.0 / ox;
             ioy = 1.0 / oy;
             if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
@@ -452,39 +458,42 @@ history_kernel(const __grid_constant__ TrackParams P) {
 }
 
 // Instantiations: deterministic/production x density format x layout x block map; the
-// production u8 + block-map kernels also come with a 72-register cap (7 CTAs per SM,
-// selected by ctas_per_sm = 7; the default is 80 registers, 6 CTAs per SM) and with
-// warp-aggregated flushes (tally_mode 1).
+// u8 + block-map kernels also come with the cached-bin linear XS walk (xs_search 2), and the
+// production ones with a 72-register cap (7 CTAs per SM, ctas_per_sm = 7; the default is 80
+// registers, 6 CTAs per SM) and with warp-aggregated flushes (tally_mode 1).
 template <bool kDet, bool kTiled>
-static void* history_fn(int fmt, bool blk, int minb, int agg) {
+static void* history_fn(int fmt, bool blk, int minb, int agg, int xs) {
   if (fmt == kDensU8) {
-    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false>;
+    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false, false>;
+    if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, true>;
     if constexpr (!kDet) {
-      if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false>;
-      if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true>;
+      if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false, false>;
+      if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false>;
     }
-    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false>;
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, false>;
   }
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false>;
-  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false>;
 }
 
-static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg) {
-  if (det) return tiled ? history_fn<true, true>(fmt, blk, minb, agg) : history_fn<true, false>(fmt, blk, minb, agg);
-  return tiled ? history_fn<false, true>(fmt, blk, minb, agg) : history_fn<false, false>(fmt, blk, minb, agg);
+static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs) {
+  if (det) return tiled ? history_fn<true, true>(fmt, blk, minb, agg, xs)
+                        : history_fn<true, false>(fmt, blk, minb, agg, xs);
+  return tiled ? history_fn<false, true>(fmt, blk, minb, agg, xs)
+               : history_fn<false, false>(fmt, blk, minb, agg, xs);
 }
 
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
-                    cudaStream_t s) {
+                    int xs_search, cudaStream_t s) {
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode);
+                            tally_mode, xs_search);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
 
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb) {
   int n = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, 0),
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, 0, 0),
                                                 kHistoryBlock, 0);
   return n;
 }

@@ -161,6 +161,19 @@ def test_parity_collision_deferral(nt, orc, cfgname, defer_below):
     assert np.all(gp["status"] <= 1)
 
 
+@pytest.mark.parametrize("xs_search", [1, 2])
+@pytest.mark.parametrize("cfgname", ["small_scatter", "small_csp", "tiny_split", "small_mosaic", "tiny_A12"])
+def test_parity_xs_search_strategies(nt, orc, cfgname, xs_search):
+    """Plain binary search (1) and the paper's cached-index linear walk (2) give
+    the same bins as the default bucketed search, hence the oracle's results."""
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=True, xs_search=xs_search)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)
+    compare_tally(gt, ot)
+    compare_stats(gs, os_)
+
+
 @pytest.mark.parametrize("mode", MODES)
 def test_parity_two_steps_and_shard(nt, orc, mode):
     cfg = wl.CONFIGS["tiny_split"]
