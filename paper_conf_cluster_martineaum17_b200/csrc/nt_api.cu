@@ -76,7 +76,8 @@ struct nt_ctx {
   uint64_t seed = 0;
   DevBuf soa;
   Soa p{};
-  int32_t* defer_q = nullptr;            // collision-deferral queue (in soa)
+  int32_t* defer_q = nullptr;            // regime-parking queues (in soa)
+  int32_t* defer_q2 = nullptr;
   // step scratch: [counter][stats_u][stats_f]; per-thread f64 statistic slots
   DevBuf scratch, slots;
   // deterministic mode
@@ -490,8 +491,8 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
 static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   const size_t N = (size_t)(n > 0 ? n : 1);
   const size_t b8 = align256(N * 8), b4 = align256(N * 4), b1 = align256(N);
-  // 8 + 3 f64 columns, 6 + 3 u32 columns, the deferral queue, status
-  cudaError_t e = c->soa.ensure(11 * b8 + 10 * b4 + b1);
+  // 8 + 3 f64 columns, 6 + 3 u32 columns, the two parking queues, status
+  cudaError_t e = c->soa.ensure(11 * b8 + 11 * b4 + b1);
   if (e != cudaSuccess) return e;
   char* q = c->soa.as<char>();
   double** d8[11] = {&c->p.x, &c->p.y, &c->p.ox, &c->p.oy, &c->p.e, &c->p.w, &c->p.mfp, &c->p.dep,
@@ -502,6 +503,7 @@ static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   c->p.cy = reinterpret_cast<int32_t*>(q); q += b4;
   for (auto d : d4) { *d = reinterpret_cast<uint32_t*>(q); q += b4; }
   c->defer_q = reinterpret_cast<int32_t*>(q); q += b4;
+  c->defer_q2 = reinterpret_cast<int32_t*>(q); q += b4;
   c->p.status = reinterpret_cast<uint8_t*>(q);
   return cudaSuccess;
 }
@@ -631,21 +633,37 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
     if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
     return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
   }
-  // phase 1: particles [lo, hi), parking lonely collisions; phase 2: the parked particles
+  // Regime parking: phase 1 tracks [lo, hi) and parks lonely collisions; phase 2 resumes
+  // them.  (With more phases, even phases park lonely facets and odd ones lonely collisions,
+  // two queues alternating, the last phase parks nothing; measured with 4 phases: split
+  // 132 -> 130 ms but csp 31 -> 35 ms, as each phase adds its own tail of long streaming
+  // histories -- DESIGN.md §6.)  scratch [16, 32): queue lengths, [32, 56): work counters of
+  // phases 2-4.
+  constexpr int kPhases = 2;
   char* s = c->scratch.as<char>();
-  NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 16, c->stream));     // queue length, phase-2 counter
-  TrackParams p1 = bp;
-  p1.phase = 1;
-  p1.defer_below = c->opt.defer_below;
-  p1.defer_q = c->defer_q;
-  p1.defer_count = reinterpret_cast<unsigned long long*>(s + 16);
+  unsigned long long* qlen[2] = {reinterpret_cast<unsigned long long*>(s + 16),
+                                 reinterpret_cast<unsigned long long*>(s + 24)};
+  int32_t* q[2] = {c->defer_q, c->defer_q2};
+  NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 48, c->stream));
   const int grid = history_grid(c, det);
-  launch_history(p1, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
-  TrackParams p2 = p1;
-  p2.phase = 2;
-  p2.counter = reinterpret_cast<unsigned long long*>(s + 24);
-  launch_history(p2, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
-  launches += 2;
+  for (int ph = 1; ph <= kPhases; ++ph) {
+    TrackParams p = bp;
+    p.phase = ph;
+    const int out = (ph - 1) & 1, in = out ^ 1;
+    if (ph > 1) {
+      p.resume_q = q[in];
+      p.resume_count = qlen[in];
+      p.counter = reinterpret_cast<unsigned long long*>(s + 32 + 8 * (ph - 2));
+    }
+    p.park_q = q[out];
+    p.park_count = qlen[out];
+    if (ph > 2) NT_CUDA(c, cudaMemsetAsync(qlen[out], 0, 8, c->stream));
+    const bool last = ph == kPhases;
+    p.park_coll_below = (!last && (ph & 1)) ? c->opt.defer_below : 0;
+    p.park_fac_below = (!last && !(ph & 1)) ? c->opt.defer_below : 0;
+    launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
+    ++launches;
+  }
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;
 }

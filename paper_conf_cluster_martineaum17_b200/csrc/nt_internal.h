@@ -20,10 +20,14 @@ struct TrackParams {
   double dt;
   int64_t max_events;
   int32_t refill_min;         // refill a warp's idle lanes once at least this many are idle
-  int32_t phase;              // history kernel: 1 track [lo, hi) (may park), 2 resume parked
-  int32_t defer_below;        // phase 1 parks a colliding lane while fewer lanes collide
-  int32_t* defer_q;           // parked local indices
-  unsigned long long* defer_count;
+  // history kernel regime parking
+  int32_t phase;              // 1: track [lo, hi); >= 2: resume resume_q[0, *resume_count)
+  int32_t park_coll_below;    // park a colliding lane while fewer lanes of its warp collide
+  int32_t park_fac_below;     // park a facet lane while fewer lanes of its warp cross facets
+  const int32_t* resume_q;
+  const unsigned long long* resume_count;
+  int32_t* park_q;            // out-queue of parked local indices
+  unsigned long long* park_count;
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]

@@ -154,14 +154,17 @@ history_kernel(const __grid_constant__ TrackParams P) {
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
   int32_t bin_s = 0, bin_a = 0;   // kXsWalk: the bins of the last lookup
 
-  // Collision deferral: phase 1 tracks particles [lo, hi) and parks a lane
-  // whose next event is a collision while fewer than defer_below lanes of its warp collide
-  // (its state goes to the particle store, its index to the deferred queue, the lane takes
-  // a new particle); phase 2 resumes the queued particles -- mostly in dense matter, so
-  // their collisions run warp-converged.  Per-particle results are unchanged.
-  const bool resume = P.phase == 2;
-  const unsigned long long span2 = resume ? *P.defer_count : span;
-  const int defer_below = resume ? 0 : P.defer_below;
+  // Regime parking: phase 1 tracks particles [lo, hi); later phases resume
+  // the particles the previous phase parked.  A phase parks a lane whose next event is a
+  // collision (park_coll_below) or a facet (park_fac_below) while fewer lanes of its warp
+  // have an event of that kind: its state goes to the particle store, its index to the
+  // out-queue, and the lane takes a new particle.  So phase 1 sends the particles that
+  // reach dense matter to phase 2, where they collide warp-converged, and phase 2 sends the
+  // few that scatter back into vacuum on to phase 3.  Per-particle results are unchanged.
+  const bool resume = P.phase >= 2;
+  const unsigned long long span2 = resume ? *P.resume_count : span;
+  const int park_coll_below = P.park_coll_below;
+  const int park_fac_below = P.park_fac_below;
   int thr = refill_min;   // break the event loop once this many lanes are idle (32: all)
   for (;;) {
     // ---- refill idle lanes with new particles: one atomic per warp ----
@@ -178,7 +181,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       if (!active) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
         if (my < span2) {
-          i = resume ? P.defer_q[my] : (int32_t)(P.lo + (int64_t)my);
+          i = resume ? P.resume_q[my] : (int32_t)(P.lo + (int64_t)my);
           if (P.p.status[i] == (resume ? 2u : 1u)) {
             active = true;
             x = ld_stream(P.p.x + i, pol_stream);
@@ -263,6 +266,34 @@ history_kernel(const __grid_constant__ TrackParams P) {
           coll = dc < df && dc < ds;
         }
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
+        // park this lane: the state before this event to the particle store, the index to
+        // the out-queue (one atomicAdd per group of converged lanes), take a new particle
+        auto park = [&]() {
+          P.p.x[i] = x;
+          P.p.y[i] = y;
+          P.p.ox[i] = ox;
+          P.p.oy[i] = oy;
+          P.p.e[i] = e;
+          P.p.w[i] = w;
+          P.p.mfp[i] = mfp;
+          P.p.cx[i] = cx;
+          P.p.cy[i] = cy;
+          P.p.ctr[i] = ctr;
+          P.p.dcen[i] = dcen;
+          P.p.acc[i] = acc;
+          P.p.dstep[i] = dstep;
+          P.p.nf_s[i] = nf;
+          P.p.nc_s[i] = nc;
+          P.p.seq_s[i] = seq;
+          P.p.status[i] = 2u;
+          const unsigned am = __activemask();
+          const int ld = __ffs(am) - 1;
+          unsigned long long q = 0;
+          if (lane == ld) q = atomicAdd(P.park_count, (unsigned long long)__popc(am));
+          q = __shfl_sync(am, q, ld) + (unsigned long long)__popc(am & lt_mask);
+          P.park_q[q] = i;
+          active = false;
+        };
 
         auto flush = [&]() {
           const uint32_t cell = cidx;                // storage index of the current cell
@@ -293,32 +324,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_KILLED_E, w * e);
           fsum(SF_KILLED_W, w);
           outcome = 2;
-        } else if (coll && __popc(__activemask()) < defer_below) {
-          // ---- park for phase 2: the state before this event, index into the queue ----
-          P.p.x[i] = x;
-          P.p.y[i] = y;
-          P.p.ox[i] = ox;
-          P.p.oy[i] = oy;
-          P.p.e[i] = e;
-          P.p.w[i] = w;
-          P.p.mfp[i] = mfp;
-          P.p.cx[i] = cx;
-          P.p.cy[i] = cy;
-          P.p.ctr[i] = ctr;
-          P.p.dcen[i] = dcen;
-          P.p.acc[i] = acc;
-          P.p.dstep[i] = dstep;
-          P.p.nf_s[i] = nf;
-          P.p.nc_s[i] = nc;
-          P.p.seq_s[i] = seq;
-          P.p.status[i] = 2u;
-          const unsigned am = __activemask();
-          const int ld = __ffs(am) - 1;
-          unsigned long long q = 0;
-          if (lane == ld) q = atomicAdd(P.defer_count, (unsigned long long)__popc(am));
-          q = __shfl_sync(am, q, ld) + (unsigned long long)__popc(am & lt_mask);
-          P.defer_q[q] = i;
-          active = false;
+        } else if (coll && __popc(__activemask()) < park_coll_below) {
+          park();
+        } else if (!coll && df < ds && park_fac_below > 0 && __popc(__activemask()) < park_fac_below) {
+          park();
         } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
           acc += ((w * dc) * sig) * m.H;
