@@ -45,7 +45,9 @@ class _Problem(C.Structure):
                 ("n_scatter", C.c_int64), ("capture_keys", C.c_void_p),
                 ("capture_vals", C.c_void_p), ("n_capture", C.c_int64),
                 ("A", C.c_double), ("molar_mass", C.c_double), ("e_min", C.c_double),
-                ("w_min", C.c_double), ("max_events", C.c_int64)]
+                ("w_min", C.c_double), ("max_events", C.c_int64), ("boundary", C.c_int32),
+                ("analog", C.c_int32), ("roulette", C.c_int32), ("pad", C.c_int32),
+                ("roulette_weight", C.c_double)]
 
 
 _PFIELDS = [("x", np.float64), ("y", np.float64), ("ox", np.float64), ("oy", np.float64),
@@ -65,7 +67,10 @@ class _Stats(C.Structure):
                 ("census_energy", C.c_double), ("census_weight", C.c_double),
                 ("killed_energy", C.c_double), ("killed_weight", C.c_double),
                 ("absorbed_weight", C.c_double), ("n_xs_range", C.c_uint64),
-                ("n_nonfinite", C.c_uint64), ("n_event_cap", C.c_uint64)]
+                ("n_nonfinite", C.c_uint64), ("n_event_cap", C.c_uint64),
+                ("n_escaped", C.c_uint64), ("n_absorbed", C.c_uint64),
+                ("escaped_energy", C.c_double), ("escaped_weight", C.c_double),
+                ("absorbed_energy", C.c_double), ("roulette_gain", C.c_double)]
 
 
 _lib_handle = None
@@ -144,7 +149,10 @@ class Problem:
         sk, sv, ck, cv = self.tables
         self.c = _Problem(cfg.nx, cfg.ny, cfg.width, cfg.height, _ptr(self.density),
                           _ptr(sk), _ptr(sv), len(sk), _ptr(ck), _ptr(cv), len(ck),
-                          cfg.A, cfg.molar_mass, cfg.e_min, cfg.w_min, max_events)
+                          cfg.A, cfg.molar_mass, cfg.e_min, cfg.w_min, max_events,
+                          getattr(cfg, "boundary", 0), getattr(cfg, "analog", 0),
+                          getattr(cfg, "roulette", 0), 0,
+                          getattr(cfg, "roulette_weight", 0.0) or 2.0 * cfg.w_min)
 
 
 class Particles:

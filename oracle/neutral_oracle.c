@@ -237,9 +237,28 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
             c += 1;
             pt->ncol[i]++;
             st->n_collisions++;
-            double w_old = w;                      /* implicit capture */
-            w = w * (1.0 - m.pa);
-            st->absorbed_weight += w_old - w;
+            double mfp_u = or_u01(r[1]);           /* the draw for the new n_mfp  */
+            if (!pb->analog) {
+                double w_old = w;                  /* implicit capture */
+                w = w * (1.0 - m.pa);
+                st->absorbed_weight += w_old - w;
+            } else {
+                /* reading R31 (S8 reading A): absorb with probability p_a ("two main
+                 * branches"); the scatter branch draws its n_mfp from the next
+                 * counter because word b decided the branch. */
+                if (or_u01(r[1]) < m.pa) {
+                    or_flush(tally, nx, cx, cy, &acc, &dep, st);
+                    st->n_absorbed++;
+                    st->absorbed_weight += w;
+                    st->absorbed_energy += w * e;
+                    pt->status[i] = 0;
+                    break;
+                }
+                uint64_t r2[2];
+                or_threefry2x64_20(c, 0, pid, seed, r2);
+                c += 1;
+                mfp_u = or_u01(r2[0]);
+            }
             double mu = 1.0 - 2.0 * or_u01(r[0]);  /* CM cosine, isotropic        */
             double e2 = e * (((A * A + (2.0 * A) * mu) + 1.0) / ((A + 1.0) * (A + 1.0)));
             double ct = 0.5 * ((A + 1.0) * sqrt(e2 / e) - (A - 1.0) * sqrt(e / e2));
@@ -252,7 +271,20 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
             oy = noy;
             double tcen = dcen / v;
             e = e2;
-            if (e < pb->e_min || w < pb->w_min) {  /* termination     */
+            int kill = e < pb->e_min || w < pb->w_min;   /* termination    */
+            if (kill && pb->roulette && !(e < pb->e_min)) {
+                /* reading R32: Russian roulette instead of the hard weight cut: survive
+                 * with probability w / w_s at weight w_s (one counter) */
+                uint64_t r3[2];
+                or_threefry2x64_20(c, 0, pid, seed, r3);
+                c += 1;
+                if (or_u01(r3[0]) < w / pb->roulette_weight) {
+                    st->roulette_gain += pb->roulette_weight - w;
+                    w = pb->roulette_weight;
+                    kill = 0;
+                }
+            }
+            if (kill) {
                 or_flush(tally, nx, cx, cy, &acc, &dep, st);
                 st->killed_energy += w * e;
                 st->killed_weight += w;
@@ -266,9 +298,10 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
             sig = nd * m.st;
             iox = 1.0 / ox;
             ioy = 1.0 / oy;
-            mfp = -log(or_u01(r[1]));
+            mfp = -log(mfp_u);
         } else if (df < ds) {
             /* ---- facet ---------------------------- */
+            int escaped = 0;
             acc += ((w * df) * sig) * m.H;
             double nm = mfp - df * sig;
             mfp = nm > 0.0 ? nm : 0.0;
@@ -277,7 +310,9 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
                 y = y + df * oy;
                 x = ox > 0.0 ? or_edge(cx + 1, W, nx) : or_edge(cx, W, nx);
                 or_flush(tally, nx, cx, cy, &acc, &dep, st);
-                if (ox > 0.0) {
+                int at_boundary = ox > 0.0 ? cx == nx - 1 : cx == 0;
+                if (at_boundary && pb->boundary) { escaped = 1; }
+                else if (ox > 0.0) {
                     if (cx == nx - 1) { ox = -ox; iox = -iox; } else { cx += 1; }
                 } else {
                     if (cx == 0) { ox = -ox; iox = -iox; } else { cx -= 1; }
@@ -286,7 +321,9 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
                 x = x + df * ox;
                 y = oy > 0.0 ? or_edge(cy + 1, Hh, ny) : or_edge(cy, Hh, ny);
                 or_flush(tally, nx, cx, cy, &acc, &dep, st);
-                if (oy > 0.0) {
+                int at_boundary = oy > 0.0 ? cy == ny - 1 : cy == 0;
+                if (at_boundary && pb->boundary) { escaped = 1; }
+                else if (oy > 0.0) {
                     if (cy == ny - 1) { oy = -oy; ioy = -ioy; } else { cy += 1; }
                 } else {
                     if (cy == 0) { oy = -oy; ioy = -ioy; } else { cy -= 1; }
@@ -294,6 +331,13 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
             }
             pt->nfac[i]++;
             st->n_facets++;
+            if (escaped) {                 /* reading R30: vacuum boundary, escape */
+                st->n_escaped++;
+                st->escaped_energy += w * e;
+                st->escaped_weight += w;
+                pt->status[i] = 0;
+                break;
+            }
             nd = pb->density[(int64_t)cy * nx + cx] * cn;   /* load new density */
             sig = nd * m.st;
         } else {

@@ -43,6 +43,12 @@ typedef struct {
     double e_min;                  /* eV, energy cutoff */
     double w_min;                  /* weight cutoff */
     int64_t max_events;            /* per history per step; guard */
+    /* variants (readings R30-R32 in DESIGN.md §4) */
+    int32_t boundary;              /* 0 reflective, 1 vacuum: escape     */
+    int32_t analog;                /* 0 implicit capture (R8), 1 sampled absorption  */
+    int32_t roulette;              /* 0 hard w_min kill (R7), 1 Russian roulette     */
+    int32_t pad;
+    double roulette_weight;        /* survivor weight of the roulette                */
 } or_problem;
 
 /* Particle store, structure of arrays, indexed by LOCAL index 0..n-1;
@@ -62,6 +68,8 @@ typedef struct {
     double tally_total, census_energy, census_weight, killed_energy,
            killed_weight, absorbed_weight;
     uint64_t n_xs_range, n_nonfinite, n_event_cap;
+    uint64_t n_escaped, n_absorbed;
+    double escaped_energy, escaped_weight, absorbed_energy, roulette_gain;
 } or_stats;
 
 void     or_threefry2x64_20(uint64_t c0, uint64_t c1, uint64_t k0, uint64_t k1,

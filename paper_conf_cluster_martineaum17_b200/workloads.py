@@ -70,6 +70,11 @@ class Config:
     e_min: float = E_MIN
     w_min: float = W_MIN
     rho: float = RHO_HI          # density of the "uniform" map
+    # physics variants (R30-R32)
+    boundary: int = 0            # 0 reflective, 1 vacuum (escape)
+    analog: int = 0              # 0 implicit capture, 1 sampled absorption
+    roulette: int = 0            # 0 hard w_min kill, 1 Russian roulette
+    roulette_weight: float = 0.0  # survivor weight (0 -> 2 w_min)
 
     def with_(self, **kw) -> "Config":
         return dataclasses.replace(self, **kw)
@@ -114,6 +119,20 @@ CONFIGS: dict[str, Config] = {
     "small_mosaic": Config("small_mosaic", 601, 590, "mosaic", (0.2, 0.2, 0.6, 0.6), 3000, 19, rho=0.5),
     # every particle born in one cell of a dense medium: maximal tally contention
     "tiny_hotspot": Config("tiny_hotspot", 64, 64, "uniform_hi", (0.5, 0.5, 0.01, 0.01), 10_000, 20, _SINGLE),
+    # physics variants
+    "tiny_vacuum_bc": Config("tiny_vacuum_bc", 64, 64, "zero", (0.4, 0.4, 0.2, 0.2), 1000, 21, _SINGLE,
+                             boundary=1),
+    "tiny_mid_bc": Config("tiny_mid_bc", 64, 64, "uniform", (0.0, 0.4, 0.2, 0.2), 10_000, 22, _SINGLE,
+                          rho=0.1, boundary=1),
+    "tiny_analog": Config("tiny_analog", 64, 64, "uniform_hi", (0.4, 0.4, 0.2, 0.2), 10_000, 23, _SINGLE,
+                          analog=1),
+    "tiny_analog_mid": Config("tiny_analog_mid", 64, 64, "uniform", (0.0, 0.4, 0.2, 0.2), 10_000, 24, _SINGLE,
+                              rho=0.1, analog=1, boundary=1),
+    "tiny_roulette": Config("tiny_roulette", 64, 64, "uniform_hi", (0.4, 0.4, 0.2, 0.2), 4000, 25,
+                            Tables(kind="1g", n_scatter=2, n_capture=2, sigma_a_1g=20000.0),
+                            w_min=0.05, roulette=1, roulette_weight=0.2),
+    "small_csp_variants": Config("small_csp_variants", 256, 256, "csp", (0.0, 0.0, 0.1, 0.1), 4096, 26,
+                                 boundary=1, analog=1),
     "small_csp": Config("small_csp", 256, 256, "csp", (0.0, 0.0, 0.1, 0.1), 4096, 10),
     "small_scatter": Config("small_scatter", 256, 256, "uniform_hi", (0.45, 0.45, 0.1, 0.1), 8192, 12),
 }
