@@ -33,7 +33,7 @@
 extern "C" {
 #endif
 
-#define NT_ABI_VERSION 2
+#define NT_ABI_VERSION 3
 
 typedef struct nt_ctx nt_ctx;
 
@@ -105,6 +105,20 @@ typedef struct {
                                   cached-index search -- a linear walk from the particle's
                                   previous bin (history mode, u8 block-map meshes; others
                                   use 0).  All three return the same bin.                 */
+    /* physics variants (DESIGN.md §4 R30-R32; the defaults are the paper's problem)      */
+    int32_t boundary;          /* 0 reflective on all four sides; 1 vacuum: a
+                                  facet on the mesh boundary ends the history (escape)     */
+    int32_t analog_absorption; /* 0 implicit capture, w <- w (1 - p_a) at every collision
+                                  (north star, R8); 1 the paper's two branches
+                                  sampled: absorbed with probability p_a, else scattered
+                                  with w unchanged (the scatter draws its n_mfp from the
+                                  next RNG counter)                                        */
+    int32_t roulette;          /* 0 a weight below w_min ends the history;
+                                  1 Russian roulette: survive with probability
+                                  w / roulette_weight at weight roulette_weight (one RNG
+                                  counter)                                                 */
+    int32_t pad1;
+    double roulette_weight;    /* survivor weight (0 -> 2 w_min)                           */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,
@@ -120,6 +134,13 @@ typedef struct {
     float reduce_ms;           /* device time of the cross-GPU tally reduction            */
     float step_ms;             /* device time of the whole timestep                       */
     uint32_t n_launches;       /* kernels this library launched for the step              */
+    uint64_t n_escaped;        /* histories ended at a vacuum boundary                    */
+    uint64_t n_absorbed;       /* histories ended by a sampled absorption                 */
+    double escaped_energy, escaped_weight;   /* sum of w*E, w over escaped particles       */
+    double absorbed_energy;    /* sum of w*E of the absorbed particles (the track-length
+                                  deposits already carry it in expectation)                */
+    double roulette_gain;      /* weight added by roulette survivors: census + killed +
+                                  absorbed + escaped weight = initial weight + gain        */
 } nt_step_stats;
 
 /* Structure-of-arrays particle view used by nt_read_particles / nt_write_particles.

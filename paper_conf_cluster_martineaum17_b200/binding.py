@@ -42,7 +42,9 @@ class Options(C.Structure):
                 ("ctas_per_sm", C.c_int32), ("det_batch", C.c_int64),
                 ("refill_min", C.c_int32), ("density_format", C.c_int32),
                 ("layout", C.c_int32), ("tally_mode", C.c_int32),
-                ("defer_below", C.c_int32), ("xs_search", C.c_int32)]
+                ("defer_below", C.c_int32), ("xs_search", C.c_int32),
+                ("boundary", C.c_int32), ("analog_absorption", C.c_int32),
+                ("roulette", C.c_int32), ("pad1", C.c_int32), ("roulette_weight", C.c_double)]
 
 
 class StepStats(C.Structure):
@@ -53,7 +55,10 @@ class StepStats(C.Structure):
                 ("killed_weight", C.c_double), ("absorbed_weight", C.c_double),
                 ("n_xs_range", C.c_uint64), ("n_nonfinite", C.c_uint64),
                 ("n_event_cap", C.c_uint64), ("track_ms", C.c_float), ("reduce_ms", C.c_float),
-                ("step_ms", C.c_float), ("n_launches", C.c_uint32)]
+                ("step_ms", C.c_float), ("n_launches", C.c_uint32),
+                ("n_escaped", C.c_uint64), ("n_absorbed", C.c_uint64),
+                ("escaped_energy", C.c_double), ("escaped_weight", C.c_double),
+                ("absorbed_energy", C.c_double), ("roulette_gain", C.c_double)]
 
 
 PARTICLE_FIELDS = [("x", np.float64), ("y", np.float64), ("ox", np.float64), ("oy", np.float64),
@@ -147,7 +152,8 @@ class Tracker:
                  e_min: float = 1.0, w_min: float = 1e-3, max_events: int = 0,
                  ctas_per_sm: int = 0, det_batch: int = 0, refill_min: int = 0,
                  density_format: int = 0, layout: int = 0, tally_mode: int = 0,
-                 defer_below: int = 0, xs_search: int = 0):
+                 defer_below: int = 0, xs_search: int = 0, boundary: int = 0,
+                 analog: int = 0, roulette: int = 0, roulette_weight: float = 0.0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -168,6 +174,10 @@ class Tracker:
         o.tally_mode = tally_mode
         o.defer_below = defer_below
         o.xs_search = xs_search
+        o.boundary = boundary
+        o.analog_absorption = analog
+        o.roulette = roulette
+        o.roulette_weight = roulette_weight
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:
@@ -268,7 +278,10 @@ def setup(cfg, *, density=None, tables=None, first_id: int = 0, n_local: int | N
           **opts) -> Tracker:
     """Create a Tracker for a workloads.Config: mesh, tables and injected particles."""
     from . import workloads as wl
-    t = Tracker(A=cfg.A, molar_mass=cfg.molar_mass, e_min=cfg.e_min, w_min=cfg.w_min, **opts)
+    phys = dict(boundary=cfg.boundary, analog=cfg.analog, roulette=cfg.roulette,
+                roulette_weight=cfg.roulette_weight)
+    phys.update({k: opts.pop(k) for k in list(opts) if k in phys})
+    t = Tracker(A=cfg.A, molar_mass=cfg.molar_mass, e_min=cfg.e_min, w_min=cfg.w_min, **phys, **opts)
     t.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, wl.density(cfg) if density is None else density)
     t.load_cross_sections(*(wl.tables(cfg) if tables is None else tables))
     if n_local is None:

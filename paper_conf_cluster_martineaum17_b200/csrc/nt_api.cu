@@ -76,8 +76,7 @@ struct nt_ctx {
   uint64_t seed = 0;
   DevBuf soa;
   Soa p{};
-  int32_t* defer_q = nullptr;            // regime-parking queues (in soa)
-  int32_t* defer_q2 = nullptr;
+  int32_t* defer_q = nullptr;            // regime-parking queue (in soa)
   // step scratch: [counter][stats_u][stats_f]; per-thread f64 statistic slots
   DevBuf scratch, slots;
   // deterministic mode
@@ -149,6 +148,10 @@ void init_phys(nt_ctx* c) {
   p.kv = (2.0 * kEv) / kNeutronMass;
   p.e_min = c->opt.e_min;
   p.w_min = c->opt.w_min;
+  p.w_roul = c->opt.roulette_weight;
+  p.vacuum = c->opt.boundary;
+  p.analog = c->opt.analog_absorption;
+  p.roulette = c->opt.roulette;
 }
 
 }  // namespace
@@ -227,6 +230,11 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.defer_below == 0) opt.defer_below = def.defer_below;
   if (opt.defer_below < 0 || opt.defer_below > 33) return NT_ERR_ARG;
   if (opt.xs_search < 0 || opt.xs_search > 2) return NT_ERR_ARG;
+  if (opt.boundary < 0 || opt.boundary > 1 || opt.analog_absorption < 0 ||
+      opt.analog_absorption > 1 || opt.roulette < 0 || opt.roulette > 1)
+    return NT_ERR_ARG;
+  if (opt.roulette_weight == 0.0) opt.roulette_weight = 2.0 * opt.w_min;
+  if (opt.roulette && !(opt.roulette_weight > opt.w_min) ) return NT_ERR_ARG;
   if (!(opt.A > 0.0) || !is_fin(opt.A) || !(opt.molar_mass > 0.0) || !is_fin(opt.molar_mass) ||
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
       opt.rank < 0 || opt.rank >= opt.nranks || opt.density_format < 0 ||
@@ -491,8 +499,8 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
 static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   const size_t N = (size_t)(n > 0 ? n : 1);
   const size_t b8 = align256(N * 8), b4 = align256(N * 4), b1 = align256(N);
-  // 8 + 3 f64 columns, 6 + 3 u32 columns, the two parking queues, status
-  cudaError_t e = c->soa.ensure(11 * b8 + 11 * b4 + b1);
+  // 8 + 3 f64 columns, 6 + 3 u32 columns, the parking queue, status
+  cudaError_t e = c->soa.ensure(11 * b8 + 10 * b4 + b1);
   if (e != cudaSuccess) return e;
   char* q = c->soa.as<char>();
   double** d8[11] = {&c->p.x, &c->p.y, &c->p.ox, &c->p.oy, &c->p.e, &c->p.w, &c->p.mfp, &c->p.dep,
@@ -503,7 +511,6 @@ static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   c->p.cy = reinterpret_cast<int32_t*>(q); q += b4;
   for (auto d : d4) { *d = reinterpret_cast<uint32_t*>(q); q += b4; }
   c->defer_q = reinterpret_cast<int32_t*>(q); q += b4;
-  c->defer_q2 = reinterpret_cast<int32_t*>(q); q += b4;
   c->p.status = reinterpret_cast<uint8_t*>(q);
   return cudaSuccess;
 }
@@ -634,33 +641,25 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
     return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
   }
   // Regime parking: phase 1 tracks [lo, hi) and parks lonely collisions; phase 2 resumes
-  // them.  (With more phases, even phases park lonely facets and odd ones lonely collisions,
-  // two queues alternating, the last phase parks nothing; measured with 4 phases: split
-  // 132 -> 130 ms but csp 31 -> 35 ms, as each phase adds its own tail of long streaming
-  // histories -- DESIGN.md §6.)  scratch [16, 32): queue lengths, [32, 56): work counters of
-  // phases 2-4.
-  constexpr int kPhases = 2;
+  // them.  (Measured alternative: 4 phases, even ones parking lonely facets -- split
+  // 132 -> 130 ms but csp 31 -> 35 ms, each phase adding its own tail of long streaming
+  // histories.)  scratch [16, 24): queue length, [32, 40): phase-2 counter.
   char* s = c->scratch.as<char>();
-  unsigned long long* qlen[2] = {reinterpret_cast<unsigned long long*>(s + 16),
-                                 reinterpret_cast<unsigned long long*>(s + 24)};
-  int32_t* q[2] = {c->defer_q, c->defer_q2};
-  NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 48, c->stream));
+  unsigned long long* qlen = reinterpret_cast<unsigned long long*>(s + 16);
+  NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 24, c->stream));
   const int grid = history_grid(c, det);
-  for (int ph = 1; ph <= kPhases; ++ph) {
+  for (int ph = 1; ph <= 2; ++ph) {
     TrackParams p = bp;
     p.phase = ph;
-    const int out = (ph - 1) & 1, in = out ^ 1;
-    if (ph > 1) {
-      p.resume_q = q[in];
-      p.resume_count = qlen[in];
-      p.counter = reinterpret_cast<unsigned long long*>(s + 32 + 8 * (ph - 2));
+    if (ph == 2) {
+      p.resume_q = c->defer_q;
+      p.resume_count = qlen;
+      p.counter = reinterpret_cast<unsigned long long*>(s + 32);
+    } else {
+      p.park_q = c->defer_q;
+      p.park_count = qlen;
+      p.park_coll_below = c->opt.defer_below;
     }
-    p.park_q = q[out];
-    p.park_count = qlen[out];
-    if (ph > 2) NT_CUDA(c, cudaMemsetAsync(qlen[out], 0, 8, c->stream));
-    const bool last = ph == kPhases;
-    p.park_coll_below = (!last && (ph & 1)) ? c->opt.defer_below : 0;
-    p.park_fac_below = (!last && !(ph & 1)) ? c->opt.defer_below : 0;
     launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
     ++launches;
   }
@@ -804,6 +803,12 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   s.killed_energy = hs[SU_COUNT + SF_KILLED_E];
   s.killed_weight = hs[SU_COUNT + SF_KILLED_W];
   s.absorbed_weight = hs[SU_COUNT + SF_ABSORBED_W];
+  s.n_escaped = (uint64_t)hs[SU_ESCAPED];
+  s.n_absorbed = (uint64_t)hs[SU_ABSORBED];
+  s.escaped_energy = hs[SU_COUNT + SF_ESCAPED_E];
+  s.escaped_weight = hs[SU_COUNT + SF_ESCAPED_W];
+  s.absorbed_energy = hs[SU_COUNT + SF_ABSORBED_E];
+  s.roulette_gain = hs[SU_COUNT + SF_ROULETTE];
   s.track_ms = track_ms;
   s.reduce_ms = reduce_ms;
   s.step_ms = step_ms + reduce_ms;

@@ -101,13 +101,18 @@ struct Phys {
   double cn;       // N_A / M
   double kv;       // (2.0*EV) / M_N
   double e_min, w_min;
+  double w_roul;   // roulette survivor weight
+  int32_t vacuum;  // physics variants (R30-R32): vacuum boundary,
+  int32_t analog;  //   sampled absorption,
+  int32_t roulette;//   Russian roulette
+  int32_t pad;
 };
 
 // Step statistics slots (u64 and f64 arrays in global memory).
 enum StatU { SU_ALIVE = 0, SU_FACETS, SU_COLLISIONS, SU_CENSUS, SU_KILLED, SU_XS_RANGE,
-             SU_NONFINITE, SU_EVENT_CAP, SU_REC_OVERFLOW, SU_COUNT };
+             SU_NONFINITE, SU_EVENT_CAP, SU_REC_OVERFLOW, SU_ESCAPED, SU_ABSORBED, SU_COUNT };
 enum StatF { SF_TALLY = 0, SF_CENSUS_E, SF_CENSUS_W, SF_KILLED_E, SF_KILLED_W,
-             SF_ABSORBED_W, SF_COUNT };
+             SF_ABSORBED_W, SF_ESCAPED_E, SF_ESCAPED_W, SF_ABSORBED_E, SF_ROULETTE, SF_COUNT };
 
 // ---- Threefry-2x64-20 (Random123 Threefry) -----------------------------------
 __device__ __forceinline__ uint64_t rotl64(uint64_t x, int r) {

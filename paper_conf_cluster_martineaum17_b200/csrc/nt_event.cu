@@ -363,8 +363,25 @@ ev_step_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, const E
         const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
         ctr += 1u;
         C.nc[i] += 1u;
-        w = w * (1.0 - C.pa[i]);
-        a.f[SF_ABSORBED_W] += w0 - w;
+        double mfp_u = u01(r.b);                    // the draw for the new n_mfp
+        bool absorbed = false;
+        if (!ph.analog) {                           // implicit capture
+          w = w * (1.0 - C.pa[i]);
+          a.f[SF_ABSORBED_W] += w0 - w;
+        } else if (u01(r.b) < C.pa[i]) {           // sampled absorption (R31)
+          absorbed = true;
+        } else {                                    // scatter: n_mfp from the next counter
+          const U64x2 r2 = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+          ctr += 1u;
+          mfp_u = u01(r2.a);
+        }
+        if (absorbed) {
+          ev_flush<kDet>(P, C, i, cx, cy, acc, dstep, a);
+          a.f[SF_ABSORBED_W] += w;
+          a.f[SF_ABSORBED_E] += w * e;
+          a.u[SU_ABSORBED] += 1u;
+          ev_finish(P, C, i, x, y, ox, oy, e, w, mfp, dstep, cx, cy, ctr, false, a);
+        } else {
         const double mu = 1.0 - 2.0 * u01(r.a);
         const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
         const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
@@ -377,7 +394,18 @@ ev_step_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, const E
         oy = noy;
         const double tcen = dcen / speed(e, ph);
         e = e2;
-        if (e < ph.e_min || w < ph.w_min) {
+        bool kill = e < ph.e_min || w < ph.w_min;   // termination
+        if (kill && ph.roulette && !(e < ph.e_min)) {
+          // Russian roulette (R32): survive with probability w / w_s at weight w_s
+          const U64x2 r3 = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+          ctr += 1u;
+          if (u01(r3.a) < w / ph.w_roul) {
+            a.f[SF_ROULETTE] += ph.w_roul - w;
+            w = ph.w_roul;
+            kill = false;
+          }
+        }
+        if (kill) {
           ev_flush<kDet>(P, C, i, cx, cy, acc, dstep, a);
           a.f[SF_KILLED_E] += w * e;
           a.f[SF_KILLED_W] += w;
@@ -391,7 +419,7 @@ ev_step_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, const E
           const Mat m = refresh_xs(P.xs, ph, e, nrange);
           a.u[SU_XS_RANGE] += nrange;
           const double iox = 1.0 / ox, ioy = 1.0 / oy;
-          mfp = -log(u01(r.b));
+          mfp = -log(mfp_u);
           P.p.x[i] = x;
           P.p.y[i] = y;
           P.p.ox[i] = ox;
@@ -412,6 +440,7 @@ ev_step_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, const E
           next = ev_classify<kDet>(P, C, i, x, y, ox, oy, iox, ioy, mfp, dcen, nd, m.st, exn,
                                    eyn, a);
         }
+        }
       } else if (seg == 1) {
         // ---- facet ----
         const bool ax = C.evax[i] != 0;
@@ -428,6 +457,16 @@ ev_step_kernel(const TrackParams* __restrict__ Pp, EvCols C, EvQueues Q, const E
         const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
         const int32_t last = (ax ? nx : ny) - 1;
         const bool refl = pos ? (c == last) : (c == 0);
+        if (refl && ph.vacuum) {
+          // ---- vacuum boundary (R30): the facet ends the history (escape) ----
+          C.nf[i] += 1u;
+          a.u[SU_ESCAPED] += 1u;
+          a.f[SF_ESCAPED_E] += w0 * P.p.e[i];
+          a.f[SF_ESCAPED_W] += w0;
+          ev_finish(P, C, i, x, y, ox, oy, P.p.e[i], w0, mfp, dstep, cx, cy, P.p.ctr[i], false, a);
+          C.evtype[i] = 3u;
+          continue;
+        }
         const int32_t c2 = refl ? c : (pos ? c + 1 : c - 1);
         cx = ax ? c2 : cx;
         cy = ax ? cy : c2;

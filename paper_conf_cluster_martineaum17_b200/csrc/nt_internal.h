@@ -23,7 +23,6 @@ struct TrackParams {
   // history kernel regime parking
   int32_t phase;              // 1: track [lo, hi); >= 2: resume resume_q[0, *resume_count)
   int32_t park_coll_below;    // park a colliding lane while fewer lanes of its warp collide
-  int32_t park_fac_below;     // park a facet lane while fewer lanes of its warp cross facets
   const int32_t* resume_q;
   const unsigned long long* resume_count;
   int32_t* park_q;            // out-queue of parked local indices

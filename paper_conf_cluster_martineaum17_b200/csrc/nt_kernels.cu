@@ -79,7 +79,8 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg, bool kXsWalk>
+template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg, bool kXsWalk,
+          bool kVar>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
   static_assert(!kBlk || kFmt == kDensU8, "the block map indexes u8 material codes");
@@ -154,17 +155,15 @@ history_kernel(const __grid_constant__ TrackParams P) {
   uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
   int32_t bin_s = 0, bin_a = 0;   // kXsWalk: the bins of the last lookup
 
-  // Regime parking: phase 1 tracks particles [lo, hi); later phases resume
-  // the particles the previous phase parked.  A phase parks a lane whose next event is a
-  // collision (park_coll_below) or a facet (park_fac_below) while fewer lanes of its warp
-  // have an event of that kind: its state goes to the particle store, its index to the
-  // out-queue, and the lane takes a new particle.  So phase 1 sends the particles that
-  // reach dense matter to phase 2, where they collide warp-converged, and phase 2 sends the
-  // few that scatter back into vacuum on to phase 3.  Per-particle results are unchanged.
+  // Regime parking: phase 1 tracks particles [lo, hi); phase 2 resumes the
+  // particles phase 1 parked.  Phase 1 parks a lane whose next event is a collision while
+  // fewer than park_coll_below lanes of its warp collide: its state goes to the particle
+  // store, its index to the out-queue, and the lane takes a new particle.  So the particles
+  // that reach dense matter collide warp-converged in phase 2.  Per-particle results are
+  // unchanged.
   const bool resume = P.phase >= 2;
   const unsigned long long span2 = resume ? *P.resume_count : span;
   const int park_coll_below = P.park_coll_below;
-  const int park_fac_below = P.park_fac_below;
   int thr = refill_min;   // break the event loop once this many lanes are idle (32: all)
   for (;;) {
     // ---- refill idle lanes with new particles: one atomic per warp ----
@@ -326,8 +325,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
           outcome = 2;
         } else if (coll && __popc(__activemask()) < park_coll_below) {
           park();
-        } else if (!coll && df < ds && park_fac_below > 0 && __popc(__activemask()) < park_fac_below) {
-          park();
         } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
           acc += ((w * dc) * sig) * m.H;
@@ -337,38 +334,67 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
           ctr += 1u;
           nc += 1u;
-          const double w_old = w;
-          w = w * (1.0 - m.pa);
-          wabs += w_old - w;
-          const double mu = 1.0 - 2.0 * u01(r.a);
-          const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
-          const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
-          const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
-          const double q = 1.0 - ct * ct;
-          const double stt = sgn * sqrt(q > 0.0 ? q : 0.0);
-          const double nox = ox * ct - oy * stt;
-          const double noy = ox * stt + oy * ct;
-          ox = nox;
-          oy = noy;
-          const double tcen = dcen / speed(e, ph);
-          e = e2;
-          if (e < ph.e_min || w < ph.w_min) {
+          double mfp_u = u01(r.b);                  // the draw for the new n_mfp
+          bool absorbed = false;
+          if (!(kVar && ph.analog)) {               // implicit capture
+            const double w_old = w;
+            w = w * (1.0 - m.pa);
+            wabs += w_old - w;
+          } else if (u01(r.b) < m.pa) {            // sampled absorption (R31)
+            absorbed = true;
+          } else {                                  // scatter branch: n_mfp from the next counter
+            const U64x2 r2 = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+            ctr += 1u;
+            mfp_u = u01(r2.a);
+          }
+          if (absorbed) {
             flush();
-            fsum(SF_KILLED_E, w * e);
-            fsum(SF_KILLED_W, w);
-            cnt(SU_KILLED, 1u);
+            wabs += w;
+            fsum(SF_ABSORBED_E, w * e);
+            cnt(SU_ABSORBED, 1u);
             outcome = 2;
           } else {
-            exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
-            eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
-            dcen = tcen * speed(e, ph);
-            if constexpr (kXsWalk) m = refresh_xs_walk(P.xs, ph, e, nrange, bin_s, bin_a);
-            else m = refresh_xs(P.xs, ph, e, nrange);
-            iox = 1.0 / ox;
-            ioy = 1.0 / oy;
-            if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
-            if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
-            mfp = -log(u01(r.b));
+            const double mu = 1.0 - 2.0 * u01(r.a);
+            const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
+            const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
+            const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
+            const double q = 1.0 - ct * ct;
+            const double stt = sgn * sqrt(q > 0.0 ? q : 0.0);
+            const double nox = ox * ct - oy * stt;
+            const double noy = ox * stt + oy * ct;
+            ox = nox;
+            oy = noy;
+            const double tcen = dcen / speed(e, ph);
+            e = e2;
+            bool kill = e < ph.e_min || w < ph.w_min;   // termination
+            if (kVar && kill && ph.roulette && !(e < ph.e_min)) {
+              // Russian roulette (R32): survive with probability w / w_s at weight w_s
+              const U64x2 r3 = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+              ctr += 1u;
+              if (u01(r3.a) < w / ph.w_roul) {
+                fsum(SF_ROULETTE, ph.w_roul - w);
+                w = ph.w_roul;
+                kill = false;
+              }
+            }
+            if (kill) {
+              flush();
+              fsum(SF_KILLED_E, w * e);
+              fsum(SF_KILLED_W, w);
+              cnt(SU_KILLED, 1u);
+              outcome = 2;
+            } else {
+              exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
+              eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
+              dcen = tcen * speed(e, ph);
+              if constexpr (kXsWalk) m = refresh_xs_walk(P.xs, ph, e, nrange, bin_s, bin_a);
+              else m = refresh_xs(P.xs, ph, e, nrange);
+              iox = 1.0 / ox;
+              ioy = 1.0 / oy;
+              if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
+              if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
+              mfp = -log(mfp_u);
+            }
           }
         } else if (df < ds) {
           // ---- facet: one code path for both axes (no X/Y divergence) ----
@@ -387,7 +413,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
           cx = ax ? c2 : cx;
           cy = ax ? cy : c2;
           if (refl) {                               // rare: a branch beats 8 selects
-            if (ax) { ox = -ox; iox = -iox; } else { oy = -oy; ioy = -ioy; }
+            if (kVar && ph.vacuum) {                // vacuum boundary (R30): escape
+              cnt(SU_ESCAPED, 1u);
+              fsum(SF_ESCAPED_E, w * e);
+              fsum(SF_ESCAPED_W, w);
+              outcome = 3;
+            } else if (ax) {
+              ox = -ox;
+              iox = -iox;
+            } else {
+              oy = -oy;
+              ioy = -ioy;
+            }
           }
           // next edge on the crossed axis and the new cell's density: two independent loads,
           // consumed at the next event
@@ -466,43 +503,55 @@ history_kernel(const __grid_constant__ TrackParams P) {
   }
 }
 
-// Instantiations: deterministic/production x density format x layout x block map; the
-// u8 + block-map kernels also come with the cached-bin linear XS walk (xs_search 2), and the
+// Instantiations: deterministic/production x density format x layout x block map x physics
+// variants (kVar: the code paths of DESIGN.md R30-R32, compiled only into the kernels used
+// when a variant is switched on, so the default kernels carry none of it); the u8 +
+// block-map kernels also come with the cached-bin linear XS walk (xs_search 2), and the
 // production ones with a 72-register cap (7 CTAs per SM, ctas_per_sm = 7; the default is 80
 // registers, 6 CTAs per SM) and with warp-aggregated flushes (tally_mode 1).
-template <bool kDet, bool kTiled>
+template <bool kDet, bool kTiled, bool kVar>
 static void* history_fn(int fmt, bool blk, int minb, int agg, int xs) {
   if (fmt == kDensU8) {
-    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false, false>;
-    if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, true>;
-    if constexpr (!kDet) {
-      if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false, false>;
-      if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false>;
+    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false, false, kVar>;
+    if constexpr (!kVar) {
+      if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, true, false>;
+      if constexpr (!kDet) {
+        if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false, false, false>;
+        if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false, false>;
+      }
     }
-    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, false>;
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, false, kVar>;
   }
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false>;
-  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false, kVar>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false, kVar>;
 }
 
-static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs) {
-  if (det) return tiled ? history_fn<true, true>(fmt, blk, minb, agg, xs)
-                        : history_fn<true, false>(fmt, blk, minb, agg, xs);
-  return tiled ? history_fn<false, true>(fmt, blk, minb, agg, xs)
-               : history_fn<false, false>(fmt, blk, minb, agg, xs);
+template <bool kVar>
+static void* history_select_v(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs) {
+  if (det) return tiled ? history_fn<true, true, kVar>(fmt, blk, minb, agg, xs)
+                        : history_fn<true, false, kVar>(fmt, blk, minb, agg, xs);
+  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, agg, xs)
+               : history_fn<false, false, kVar>(fmt, blk, minb, agg, xs);
+}
+
+static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs,
+                            bool var) {
+  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, agg, xs)
+             : history_select_v<false>(det, fmt, tiled, blk, minb, agg, xs);
 }
 
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
                     int xs_search, cudaStream_t s) {
+  const bool var = tp.ph.vacuum || tp.ph.analog || tp.ph.roulette;
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode, xs_search);
+                            tally_mode, xs_search, var);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
 
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb) {
   int n = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, 0, 0),
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, 0, 0, false),
                                                 kHistoryBlock, 0);
   return n;
 }

@@ -61,9 +61,10 @@ def compare_tally(gpu, orc, rtol=1e-9, floor=1e-9):
 
 def compare_stats(gs: dict, os_: dict, rtol=1e-9):
     for k in ["n_alive_start", "n_facets", "n_collisions", "n_census", "n_killed", "n_xs_range",
-              "n_nonfinite", "n_event_cap"]:
+              "n_nonfinite", "n_event_cap", "n_escaped", "n_absorbed"]:
         assert gs[k] == os_[k], f"stat {k}: gpu {gs[k]} oracle {os_[k]}"
     for k in ["tally_total", "census_energy", "census_weight", "killed_energy", "killed_weight",
-              "absorbed_weight"]:
+              "absorbed_weight", "escaped_energy", "escaped_weight", "absorbed_energy",
+              "roulette_gain"]:
         a, b = gs[k], os_[k]
         assert abs(a - b) <= rtol * max(abs(b), 1e-300) + 1e-300, f"stat {k}: gpu {a} oracle {b}"

@@ -104,7 +104,10 @@ def test_inject_matches_oracle(nt, orc, cfgname):
 # ---------------------------------------------------------------------------------------------
 TINY = ["tiny_csp", "tiny_stream", "tiny_split", "tiny_vacuum", "tiny_vacuum_lo", "tiny_scatter_1g",
         "tiny_wkill", "tiny_A12", "tiny_mid", "tiny_thin", "tiny_absorber", "small_csp", "small_scatter",
-        "tiny_levels", "small_random", "tiny_mosaic", "small_mosaic", "tiny_hotspot"]
+        "tiny_levels", "small_random", "tiny_mosaic", "small_mosaic", "tiny_hotspot",
+        # physics variants (R30-R32)
+        "tiny_vacuum_bc", "tiny_mid_bc", "tiny_analog", "tiny_analog_mid", "tiny_roulette",
+        "small_csp_variants"]
 
 
 @pytest.mark.parametrize("mode", MODES)
@@ -124,7 +127,7 @@ def test_parity_deterministic(nt, orc, cfgname, mode):
 @pytest.mark.parametrize("layout", [0, 1])
 @pytest.mark.parametrize("density_format", [0, 1, 2])
 @pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_split", "tiny_mid", "small_scatter", "tiny_levels",
-                                     "tiny_mosaic"])
+                                     "tiny_mosaic", "tiny_analog_mid", "tiny_roulette"])
 def test_parity_production_atomic(nt, orc, cfgname, mode, density_format, layout):
     cfg = wl.CONFIGS[cfgname]
     gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, density_format=density_format,
