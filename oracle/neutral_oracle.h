@@ -14,7 +14,10 @@
  * injection geometry (P3), vacuum closed form (P4), population (P5), flight
  * length law (P6), scatter kinematics / slowing-down law (P7), implicit-capture
  * weights and weight ledger (P8), XS lookup vs brute force (P9), energy balance
- * (P10), symmetry (P11), printed workload facts (P12).
+ * (P10), symmetry (P11), printed workload facts (P12); variants (R30-R32,
+ * tests/test_oracle_variants.py): vacuum-escape closed form, escape/absorption/
+ * roulette ledgers, the sampled-absorption branch law and counter budget,
+ * roulette unbiasedness.
  * Parity unpinned: absolute per-cell tally values at paper scale (the paper's
  * Fig. 2 plots are absent) -- only P10-P12 constrain them.
  */
