@@ -33,7 +33,7 @@
 extern "C" {
 #endif
 
-#define NT_ABI_VERSION 3
+#define NT_ABI_VERSION 4
 
 typedef struct nt_ctx nt_ctx;
 
@@ -117,7 +117,13 @@ typedef struct {
                                   1 Russian roulette: survive with probability
                                   w / roulette_weight at weight roulette_weight (one RNG
                                   counter)                                                 */
-    int32_t pad1;
+    int32_t decomposition;     /* 0: replicated mesh, particles split by global id, tally
+                                  allreduced; 1: x-slabs (SURVEY §8(f) row
+                                  1) -- rank r owns the mesh columns [floor(r nx/P),
+                                  floor((r+1) nx/P)) and tracks the particles inside them;
+                                  a particle crossing a slab edge migrates to the
+                                  neighbour (nt_run_timestep exchanges them over NCCL, or
+                                  the caller drives nt_slab_*).  Production tally only.   */
     double roulette_weight;    /* survivor weight (0 -> 2 w_min)                           */
 } nt_options;
 
@@ -156,6 +162,7 @@ typedef struct {
     uint8_t *status;           /* 1 alive (at census), 0 dead                             */
     uint32_t *nfac, *ncol, *ncen; /* cumulative facet / collision / census events         */
     double *dep;               /* cumulative energy this particle deposited in the tally  */
+    int64_t *gid;              /* global particle id (the RNG key)             */
 } nt_particles;
 
 /* Library identity. */
@@ -220,6 +227,26 @@ nt_status nt_read_particles(nt_ctx *ctx, int64_t first, int64_t count,
  * is counter based, so a restored particle continues bit-exactly). */
 nt_status nt_write_particles(nt_ctx *ctx, int64_t first, int64_t count,
                              const nt_particles *src);
+
+/* ---- slab decomposition driven by the caller (decomposition = 1) -------------------
+ * One timestep = nt_slab_begin, then rounds until no rank has emigrants: nt_slab_round
+ * tracks this rank's particles (the first round: its own; later rounds: the arrivals)
+ * until census, death or a slab edge; nt_slab_export hands over the emigrants as packed
+ * records (those leaving to the left first, n_left + n_right of them), which the caller
+ * delivers to the neighbours' nt_slab_import; nt_slab_end returns this rank's statistics
+ * (sum them over ranks; the tally is read with nt_read_tally(reduced = 0) and summed).
+ * Per-particle results equal the replicated run's (the RNG is keyed by global id).
+ * Local slots of emigrated particles keep status 4 (moved); arrivals are appended. */
+int64_t   nt_slab_record_bytes(void);
+nt_status nt_slab_begin(nt_ctx *ctx, double dt);
+nt_status nt_slab_round(nt_ctx *ctx, int64_t *n_emigrants);
+nt_status nt_slab_export(nt_ctx *ctx, void *dst, int64_t capacity, int64_t *n_left,
+                         int64_t *n_right);
+nt_status nt_slab_import(nt_ctx *ctx, const void *src, int64_t n);
+nt_status nt_slab_end(nt_ctx *ctx, nt_step_stats *stats);
+/* Local particle slots in use (the range nt_read_particles accepts): n_local at
+ * injection, growing when slab arrivals find no free slot. */
+nt_status nt_particle_slots(nt_ctx *ctx, int64_t *n_slots);
 
 /* Verification entry points (run the device code paths in isolation). */
 /* out[2i], out[2i+1] = threefry2x64_20(ctr = {in[4i], in[4i+1]}, key = {in[4i+2], in[4i+3]}). */

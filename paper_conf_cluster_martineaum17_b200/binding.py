@@ -24,7 +24,9 @@ MODES = {"history": 0, "event": 1}
 EXPORTS = ["nt_abi_version", "nt_build_info", "nt_status_string", "nt_options_default",
            "nt_get_unique_id", "nt_create", "nt_destroy", "nt_last_error", "nt_init_mesh",
            "nt_load_cross_sections", "nt_inject_particles", "nt_run_timestep", "nt_read_tally",
-           "nt_read_particles", "nt_write_particles", "nt_debug_threefry", "nt_debug_xs"]
+           "nt_read_particles", "nt_write_particles", "nt_slab_record_bytes", "nt_slab_begin",
+           "nt_slab_round", "nt_slab_export", "nt_slab_import", "nt_slab_end", "nt_particle_slots",
+           "nt_debug_threefry", "nt_debug_xs"]
 
 
 class NeutralError(RuntimeError):
@@ -44,7 +46,8 @@ class Options(C.Structure):
                 ("layout", C.c_int32), ("tally_mode", C.c_int32),
                 ("defer_below", C.c_int32), ("xs_search", C.c_int32),
                 ("boundary", C.c_int32), ("analog_absorption", C.c_int32),
-                ("roulette", C.c_int32), ("pad1", C.c_int32), ("roulette_weight", C.c_double)]
+                ("roulette", C.c_int32), ("decomposition", C.c_int32),
+                ("roulette_weight", C.c_double)]
 
 
 class StepStats(C.Structure):
@@ -65,7 +68,7 @@ PARTICLE_FIELDS = [("x", np.float64), ("y", np.float64), ("ox", np.float64), ("o
                    ("e", np.float64), ("w", np.float64), ("mfp", np.float64), ("cx", np.int32),
                    ("cy", np.int32), ("ctr", np.uint32), ("status", np.uint8),
                    ("nfac", np.uint32), ("ncol", np.uint32), ("ncen", np.uint32),
-                   ("dep", np.float64)]
+                   ("dep", np.float64), ("gid", np.int64)]
 
 
 class ParticlesView(C.Structure):
@@ -100,6 +103,13 @@ def lib():
             "nt_read_tally": ([vp, vp, i32], C.c_int),
             "nt_read_particles": ([vp, i64, i64, C.POINTER(ParticlesView)], C.c_int),
             "nt_write_particles": ([vp, i64, i64, C.POINTER(ParticlesView)], C.c_int),
+            "nt_slab_record_bytes": ([], i64),
+            "nt_slab_begin": ([vp, d], C.c_int),
+            "nt_slab_round": ([vp, C.POINTER(i64)], C.c_int),
+            "nt_slab_export": ([vp, vp, i64, C.POINTER(i64), C.POINTER(i64)], C.c_int),
+            "nt_slab_import": ([vp, vp, i64], C.c_int),
+            "nt_slab_end": ([vp, C.POINTER(StepStats)], C.c_int),
+            "nt_particle_slots": ([vp, C.POINTER(i64)], C.c_int),
             "nt_debug_threefry": ([vp, vp, i64, vp], C.c_int),
             "nt_debug_xs": ([vp, vp, i64, vp, vp], C.c_int),
         }
@@ -153,7 +163,8 @@ class Tracker:
                  ctas_per_sm: int = 0, det_batch: int = 0, refill_min: int = 0,
                  density_format: int = 0, layout: int = 0, tally_mode: int = 0,
                  defer_below: int = 0, xs_search: int = 0, boundary: int = 0,
-                 analog: int = 0, roulette: int = 0, roulette_weight: float = 0.0):
+                 analog: int = 0, roulette: int = 0, roulette_weight: float = 0.0,
+                 decomposition: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -178,6 +189,7 @@ class Tracker:
         o.analog_absorption = analog
         o.roulette = roulette
         o.roulette_weight = roulette_weight
+        o.decomposition = decomposition
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:
@@ -237,6 +249,36 @@ class Tracker:
         d["events"] = d["n_facets"] + d["n_collisions"] + d["n_census"]
         return d
 
+    # -- slab decomposition driven by the caller (decomposition = 1) ------------------------
+    def slab_begin(self, dt: float):
+        self._check(lib().nt_slab_begin(self._h, dt), "nt_slab_begin")
+
+    def slab_round(self) -> int:
+        n = C.c_int64()
+        self._check(lib().nt_slab_round(self._h, C.byref(n)), "nt_slab_round")
+        return n.value
+
+    def slab_export(self, n_max: int):
+        rb = lib().nt_slab_record_bytes()
+        buf = np.empty(max(1, n_max) * rb, dtype=np.uint8)
+        nl, nr = C.c_int64(), C.c_int64()
+        self._check(lib().nt_slab_export(self._h, buf.ctypes.data, n_max, C.byref(nl), C.byref(nr)),
+                    "nt_slab_export")
+        return buf[: (nl.value + nr.value) * rb].reshape(-1, rb), nl.value, nr.value
+
+    def slab_import(self, recs: np.ndarray):
+        recs = np.ascontiguousarray(recs, dtype=np.uint8)
+        self._check(lib().nt_slab_import(self._h, recs.ctypes.data, recs.shape[0] if recs.ndim == 2 else 0),
+                    "nt_slab_import")
+
+    def slab_end(self) -> dict:
+        s = StepStats()
+        st = self._check(lib().nt_slab_end(self._h, C.byref(s)), "nt_slab_end", allow=STEP_ANOMALIES)
+        d = {n: getattr(s, n) for n, _ in StepStats._fields_}
+        d["status"] = st
+        d["events"] = d["n_facets"] + d["n_collisions"] + d["n_census"]
+        return d
+
     def read_tally(self, out=None, reduced: bool = True):
         if out is None:
             out = np.empty((self.ny, self.nx), dtype=np.float64)
@@ -245,9 +287,14 @@ class Tracker:
         return out
 
     # -- verification / checkpoint ------------------------------------------------------------
+    def particle_slots(self) -> int:
+        n = C.c_int64()
+        self._check(lib().nt_particle_slots(self._h, C.byref(n)), "nt_particle_slots")
+        return n.value
+
     def read_particles(self, first: int = 0, count: int | None = None) -> dict:
         if count is None:
-            count = self.n_local - first
+            count = self.particle_slots() - first
         out = {n: np.empty(count, dtype=t) for n, t in PARTICLE_FIELDS}
         v = ParticlesView(*[out[n].ctypes.data for n, _ in PARTICLE_FIELDS])
         self._check(lib().nt_read_particles(self._h, first, count, C.byref(v)), "nt_read_particles")

@@ -77,6 +77,18 @@ struct nt_ctx {
   DevBuf soa;
   Soa p{};
   int32_t* defer_q = nullptr;            // regime-parking queue (in soa)
+  // x-slab decomposition (decomposition 1)
+  int64_t n_cap = 0;                     // particle-store capacity (n_total with slabs)
+  int32_t slab_lo = 0, slab_hi = 0;      // owned mesh columns
+  int32_t* arr_q = nullptr;              // arrivals queued for the next round (in soa)
+  int32_t* out_q = nullptr;              // emigrants of the running round (in soa)
+  int64_t n_arr = 0;                     // arrivals waiting for the next round
+  int32_t* free_q = nullptr;             // slots vacated by emigrants, reused by arrivals
+  int64_t n_free = 0;
+  int slab_round = 0;
+  uint32_t slab_launches = 0;
+  double slab_dt = 0.0;
+  DevBuf slab_buf, slab_rbuf;            // packed emigrant / received records
   // step scratch: [counter][stats_u][stats_f]; per-thread f64 statistic slots
   DevBuf scratch, slots;
   // deterministic mode
@@ -241,7 +253,9 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
       opt.density_format > 2 || opt.layout < 0 || opt.layout > 1 || opt.tally_mode < 0 ||
       opt.tally_mode > 1)
     return NT_ERR_ARG;
-  if (opt.nranks > 1 && !opt.nccl_unique_id) return NT_ERR_ARG;
+  // nranks > 1 needs a communicator, except for x-slabs driven by the caller (nt_slab_*)
+  if (opt.nranks > 1 && !opt.nccl_unique_id && opt.decomposition != 1) return NT_ERR_ARG;
+  if (opt.decomposition < 0 || opt.decomposition > 1) return NT_ERR_ARG;
 
   nt_ctx* c = new nt_ctx();
   c->opt = opt;
@@ -263,7 +277,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   }
   for (auto& ev : c->ev) cudaEventCreate(&ev);
   init_phys(c);
-  if (opt.nranks > 1 || opt.nccl_unique_id) {
+  if (opt.nccl_unique_id) {
     ncclUniqueId id;
     std::memcpy(&id, opt.nccl_unique_id, sizeof id);
     ncclResult_t r = ncclCommInitRank(&c->comm, opt.nranks, id, opt.rank);
@@ -281,7 +295,7 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
-  for (DevBuf* b : {&c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
+  for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup})
     b->release();
@@ -499,8 +513,8 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
 static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   const size_t N = (size_t)(n > 0 ? n : 1);
   const size_t b8 = align256(N * 8), b4 = align256(N * 4), b1 = align256(N);
-  // 8 + 3 f64 columns, 6 + 3 u32 columns, the parking queue, status
-  cudaError_t e = c->soa.ensure(11 * b8 + 10 * b4 + b1);
+  // 8 + 3 f64 columns, gid, 6 + 3 u32 columns, parking / arrival / emigrant / free queues, status
+  cudaError_t e = c->soa.ensure(12 * b8 + 13 * b4 + b1);
   if (e != cudaSuccess) return e;
   char* q = c->soa.as<char>();
   double** d8[11] = {&c->p.x, &c->p.y, &c->p.ox, &c->p.oy, &c->p.e, &c->p.w, &c->p.mfp, &c->p.dep,
@@ -511,6 +525,10 @@ static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   c->p.cy = reinterpret_cast<int32_t*>(q); q += b4;
   for (auto d : d4) { *d = reinterpret_cast<uint32_t*>(q); q += b4; }
   c->defer_q = reinterpret_cast<int32_t*>(q); q += b4;
+  c->arr_q = reinterpret_cast<int32_t*>(q); q += b4;
+  c->out_q = reinterpret_cast<int32_t*>(q); q += b4;
+  c->free_q = reinterpret_cast<int32_t*>(q); q += b4;
+  c->p.gid = reinterpret_cast<int64_t*>(q); q += b8;
   c->p.status = reinterpret_cast<uint8_t*>(q);
   return cudaSuccess;
 }
@@ -527,7 +545,20 @@ nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int6
       !(sy + sh <= c->H))
     return fail(c, NT_ERR_ARG, "source rectangle must lie inside the mesh");
   if (!(e0 > 0.0) || !is_fin(e0)) return fail(c, NT_ERR_ARG, "initial_energy must be finite and > 0");
-  NT_CUDA(c, alloc_soa(c, n_local));
+  const bool slab = c->opt.decomposition == 1;
+  if (slab && c->opt.deterministic)
+    return fail(c, NT_ERR_UNSUPPORTED, "x-slab decomposition supports the production tally only");
+  if (slab && c->opt.mode != NT_MODE_HISTORY)
+    return fail(c, NT_ERR_UNSUPPORTED, "x-slab decomposition supports history mode only");
+  c->n_cap = slab ? (n_total > n_local ? n_total : n_local) : n_local;
+  c->n_free = 0;
+  c->n_arr = 0;
+  NT_CUDA(c, alloc_soa(c, c->n_cap));
+  if (slab) {
+    const int64_t P = c->opt.nranks, r = c->opt.rank;
+    c->slab_lo = (int32_t)((r * c->nx) / P);
+    c->slab_hi = (int32_t)(((r + 1) * c->nx) / P);
+  }
   InjectParams ip{};
   ip.p = c->p;
   ip.ex = c->ex.as<double>();
@@ -633,17 +664,15 @@ static nt_status det_snapshot(nt_ctx* c, int64_t lo, int64_t nb, bool restore) {
   return NT_OK;
 }
 
-// Track one batch [bp.lo, bp.hi) in the context's mode (history kernel or event loop).
-static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_t& launches) {
-  if (c->opt.mode == NT_MODE_EVENT) {
-    if (!c->evs) c->evs = event_state_create();
-    if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
-    return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
-  }
-  // Regime parking: phase 1 tracks [lo, hi) and parks lonely collisions; phase 2 resumes
-  // them.  (Measured alternative: 4 phases, even ones parking lonely facets -- split
-  // 132 -> 130 ms but csp 31 -> 35 ms, each phase adding its own tail of long streaming
-  // histories.)  scratch [16, 24): queue length, [32, 40): phase-2 counter.
+// History kernel with regime parking: phase 1 tracks [lo, hi) -- or, with src_count, the
+// parked particles queued in c->arr_q (slab arrivals) -- and parks lonely collisions;
+// phase 2 resumes them.  (Measured alternative: 4 phases, even ones parking lonely facets
+// -- split 132 -> 130 ms but csp 31 -> 35 ms, each phase adding its own tail of long
+// streaming histories.)  With slabs, both phases hand emigrants to out_q.
+// scratch [0, 8): phase-1 counter, [16, 24): parking queue length, [32, 40): phase-2
+// counter, [40, 48): emigrant count, [64, 72): arrivals count.
+static nt_status track_phases(nt_ctx* c, const TrackParams& bp, bool det, uint32_t& launches,
+                              const unsigned long long* src_count, bool slab) {
   char* s = c->scratch.as<char>();
   unsigned long long* qlen = reinterpret_cast<unsigned long long*>(s + 16);
   NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 24, c->stream));
@@ -651,20 +680,41 @@ static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_
   for (int ph = 1; ph <= 2; ++ph) {
     TrackParams p = bp;
     p.phase = ph;
+    if (slab) {
+      p.slab_lo = c->slab_lo;
+      p.slab_hi = c->slab_hi;
+      p.out_q = c->out_q;
+      p.out_count = reinterpret_cast<unsigned long long*>(s + 40);
+    }
     if (ph == 2) {
       p.resume_q = c->defer_q;
       p.resume_count = qlen;
       p.counter = reinterpret_cast<unsigned long long*>(s + 32);
     } else {
+      if (src_count) {
+        p.resume_q = c->arr_q;
+        p.resume_count = src_count;
+      }
       p.park_q = c->defer_q;
       p.park_count = qlen;
       p.park_coll_below = c->opt.defer_below;
     }
-    launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, c->stream);
+    launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, slab,
+                   c->stream);
     ++launches;
   }
   NT_CUDA(c, cudaGetLastError());
   return NT_OK;
+}
+
+// Track one batch [bp.lo, bp.hi) in the context's mode (history kernel or event loop).
+static nt_status track_range(nt_ctx* c, const TrackParams& bp, bool det, uint32_t& launches) {
+  if (c->opt.mode == NT_MODE_EVENT) {
+    if (!c->evs) c->evs = event_state_create();
+    if (!c->evs) return fail(c, NT_ERR_OOM, "event state");
+    return event_run_range(c->evs, bp, det, c->sm_count, c->stream, launches, c->err);
+  }
+  return track_phases(c, bp, det, launches, nullptr, false);
 }
 
 static nt_status run_det(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
@@ -729,25 +779,210 @@ static nt_status run_det(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
   return NT_OK;
 }
 
-nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
-  if (!c) return NT_ERR_ARG;
-  cudaSetDevice(c->device);
+// ---- x-slab decomposition ---------------------------------------------
+// One round: the first round tracks this rank's own particles [0, n_local) (status 1), later
+// rounds the arrivals queued by nt_slab_import; emigrants are left in out_q.
+static nt_status slab_round(nt_ctx* c, const TrackParams& tp, uint32_t& launches, int64_t* n_out) {
+  char* s = c->scratch.as<char>();
+  unsigned long long* out_count = reinterpret_cast<unsigned long long*>(s + 40);
+  unsigned long long* arr_count = reinterpret_cast<unsigned long long*>(s + 64);
+  NT_CUDA(c, cudaMemsetAsync(s, 0, 8, c->stream));                // phase-1 work counter
+  NT_CUDA(c, cudaMemsetAsync(out_count, 0, 8, c->stream));
+  TrackParams bp = tp;
+  bp.hi = c->n_local;
+  nt_status st = NT_OK;
+  if (c->slab_round == 0) {
+    st = track_phases(c, bp, false, launches, nullptr, true);
+  } else if (c->n_arr > 0) {
+    const unsigned long long na = (unsigned long long)c->n_arr;
+    NT_CUDA(c, cudaMemcpyAsync(arr_count, &na, 8, cudaMemcpyHostToDevice, c->stream));
+    st = track_phases(c, bp, false, launches, arr_count, true);
+  }
+  if (st != NT_OK) return st;
+  unsigned long long no = 0;
+  NT_CUDA(c, cudaMemcpyAsync(&no, out_count, 8, cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  c->n_arr = 0;
+  ++c->slab_round;
+  *n_out = (int64_t)no;
+  return NT_OK;
+}
+
+// Pack the round's emigrants into c->slab_buf (left-going first); counts in *nl, *nr.
+static nt_status slab_pack(nt_ctx* c, const TrackParams& tp, int64_t n_out, int64_t* nl,
+                           int64_t* nr) {
+  char* s = c->scratch.as<char>();
+  unsigned long long* cnt = reinterpret_cast<unsigned long long*>(s + 48);
+  NT_CUDA(c, c->slab_buf.ensure((size_t)(n_out > 0 ? n_out : 1) * sizeof(SlabRec)));
+  NT_CUDA(c, cudaMemsetAsync(cnt, 0, 16, c->stream));
+  TrackParams p = tp;
+  p.slab_lo = c->slab_lo;
+  p.slab_hi = c->slab_hi;
+  launch_slab_pack(p, c->out_q, n_out, c->slab_buf.as<SlabRec>(), cnt, c->stream);
+  NT_CUDA(c, cudaGetLastError());
+  unsigned long long h[2] = {0, 0};
+  NT_CUDA(c, cudaMemcpyAsync(h, cnt, 16, cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  *nl = (int64_t)h[0];
+  *nr = (int64_t)h[1];
+  return NT_OK;
+}
+
+// The emigrants' slots (out_q) become free for arrivals.
+static cudaError_t slab_free_slots(nt_ctx* c, int64_t n_out) {
+  if (n_out <= 0) return cudaSuccess;
+  const cudaError_t e = cudaMemcpyAsync(c->free_q + c->n_free, c->out_q, (size_t)n_out * 4,
+                                        cudaMemcpyDeviceToDevice, c->stream);
+  c->n_free += n_out;
+  return e;
+}
+
+// Store n records (device memory) as parked particles queued for the next round: first in
+// free slots, then appended.
+static nt_status slab_unpack(nt_ctx* c, const SlabRec* d, int64_t n) {
+  if (n <= 0) return NT_OK;
+  const int64_t m = n < c->n_free ? n : c->n_free;
+  if (c->n_local + (n - m) > c->n_cap)
+    return fail(c, NT_ERR_ARG, "slab import exceeds the particle store (%lld + %lld > %lld)",
+                (long long)c->n_local, (long long)(n - m), (long long)c->n_cap);
+  c->n_free -= m;
+  launch_slab_unpack(c->p, d, n, c->free_q + c->n_free, m, c->n_local, c->arr_q + c->n_arr,
+                     c->stream);
+  NT_CUDA(c, cudaGetLastError());
+  c->n_local += n - m;
+  c->n_arr += n;
+  return NT_OK;
+}
+
+// nt_run_timestep with slabs: rounds until no rank has emigrants; with a communicator the
+// emigrants go to the neighbouring ranks over NCCL (counts, then records), and an allreduce
+// of the emigrant count ends the loop.
+static nt_status run_slab_nccl(nt_ctx* c, const TrackParams& tp, uint32_t& launches) {
+  c->slab_round = 0;
+  c->n_arr = 0;
+  const int P = c->opt.nranks, r = c->opt.rank;
+  for (int round = 0;; ++round) {
+    if (round > 4 * (c->nx + c->ny) + 16)
+      return fail(c, NT_ERR_STATE, "slab exchange did not terminate");
+    int64_t n_out = 0;
+    nt_status st = slab_round(c, tp, launches, &n_out);
+    if (st != NT_OK) return st;
+    if (!c->comm) {
+      if (n_out != 0) return fail(c, NT_ERR_STATE, "emigrants without a communicator");
+      return NT_OK;
+    }
+    int64_t nl = 0, nr = 0;
+    st = slab_pack(c, tp, n_out, &nl, &nr);
+    if (st != NT_OK) return st;
+    NT_CUDA(c, slab_free_slots(c, n_out));
+    // counts to / from the neighbours, then the records
+    char* s = c->scratch.as<char>();
+    long long* dc = reinterpret_cast<long long*>(s + 128);   // [send l, send r, recv l, recv r, tot]
+    const long long hsend[3] = {(long long)nl, (long long)nr, (long long)n_out};
+    NT_CUDA(c, cudaMemcpyAsync(dc, hsend, 16, cudaMemcpyHostToDevice, c->stream));
+    NT_CUDA(c, cudaMemcpyAsync(dc + 4, hsend + 2, 8, cudaMemcpyHostToDevice, c->stream));
+    NT_CUDA(c, cudaMemsetAsync(dc + 2, 0, 16, c->stream));
+    NT_NCCL(c, ncclGroupStart());
+    if (r > 0) {
+      NT_NCCL(c, ncclSend(dc + 0, 1, ncclInt64, r - 1, c->comm, c->stream));
+      NT_NCCL(c, ncclRecv(dc + 2, 1, ncclInt64, r - 1, c->comm, c->stream));
+    }
+    if (r + 1 < P) {
+      NT_NCCL(c, ncclSend(dc + 1, 1, ncclInt64, r + 1, c->comm, c->stream));
+      NT_NCCL(c, ncclRecv(dc + 3, 1, ncclInt64, r + 1, c->comm, c->stream));
+    }
+    NT_NCCL(c, ncclGroupEnd());
+    NT_NCCL(c, ncclAllReduce(dc + 4, dc + 4, 1, ncclInt64, ncclSum, c->comm, c->stream));
+    long long hrecv[3] = {0, 0, 0};
+    NT_CUDA(c, cudaMemcpyAsync(hrecv, dc + 2, 24, cudaMemcpyDeviceToHost, c->stream));
+    NT_CUDA(c, cudaStreamSynchronize(c->stream));
+    if (hrecv[2] == 0) return NT_OK;                       // nobody moves: step done
+    const int64_t nin = hrecv[0] + hrecv[1];
+    const size_t rb = sizeof(SlabRec);
+    NT_CUDA(c, c->slab_rbuf.ensure((size_t)(nin > 0 ? nin : 1) * rb));
+    char* sb = c->slab_buf.as<char>();
+    char* rbuf = c->slab_rbuf.as<char>();
+    NT_NCCL(c, ncclGroupStart());
+    if (r > 0) {
+      if (nl) NT_NCCL(c, ncclSend(sb, (size_t)nl * rb, ncclUint8, r - 1, c->comm, c->stream));
+      if (hrecv[0]) NT_NCCL(c, ncclRecv(rbuf, (size_t)hrecv[0] * rb, ncclUint8, r - 1, c->comm, c->stream));
+    }
+    if (r + 1 < P) {
+      if (nr) NT_NCCL(c, ncclSend(sb + (size_t)(n_out - nr) * rb, (size_t)nr * rb, ncclUint8, r + 1,
+                                  c->comm, c->stream));
+      if (hrecv[1]) NT_NCCL(c, ncclRecv(rbuf + (size_t)hrecv[0] * rb, (size_t)hrecv[1] * rb, ncclUint8,
+                                        r + 1, c->comm, c->stream));
+    }
+    NT_NCCL(c, ncclGroupEnd());
+    st = slab_unpack(c, c->slab_rbuf.as<SlabRec>(), nin);
+    if (st != NT_OK) return st;
+  }
+}
+
+// Step statistics from the reduced counters; the return status reports device anomalies.
+static nt_status finish_stats(nt_ctx* c, const double* hs, float track_ms, float reduce_ms,
+                              float step_ms, uint32_t launches, nt_step_stats* stats) {
+  nt_step_stats s{};
+  s.n_alive_start = (uint64_t)hs[SU_ALIVE];
+  s.n_facets = (uint64_t)hs[SU_FACETS];
+  s.n_collisions = (uint64_t)hs[SU_COLLISIONS];
+  s.n_census = (uint64_t)hs[SU_CENSUS];
+  s.n_killed = (uint64_t)hs[SU_KILLED];
+  s.n_xs_range = (uint64_t)hs[SU_XS_RANGE];
+  s.n_nonfinite = (uint64_t)hs[SU_NONFINITE];
+  s.n_event_cap = (uint64_t)hs[SU_EVENT_CAP];
+  s.tally_total = hs[SU_COUNT + SF_TALLY];
+  s.census_energy = hs[SU_COUNT + SF_CENSUS_E];
+  s.census_weight = hs[SU_COUNT + SF_CENSUS_W];
+  s.killed_energy = hs[SU_COUNT + SF_KILLED_E];
+  s.killed_weight = hs[SU_COUNT + SF_KILLED_W];
+  s.absorbed_weight = hs[SU_COUNT + SF_ABSORBED_W];
+  s.n_escaped = (uint64_t)hs[SU_ESCAPED];
+  s.n_absorbed = (uint64_t)hs[SU_ABSORBED];
+  s.escaped_energy = hs[SU_COUNT + SF_ESCAPED_E];
+  s.escaped_weight = hs[SU_COUNT + SF_ESCAPED_W];
+  s.absorbed_energy = hs[SU_COUNT + SF_ABSORBED_E];
+  s.roulette_gain = hs[SU_COUNT + SF_ROULETTE];
+  s.track_ms = track_ms;
+  s.reduce_ms = reduce_ms;
+  s.step_ms = step_ms + reduce_ms;
+  s.n_launches = launches;
+  if (stats) *stats = s;
+  c->stage = ST_STEPPED;
+  if (hs[SU_REC_OVERFLOW] > 0) return fail(c, NT_ERR_UNSUPPORTED, "flush sequence overflow (>2^24 flushes in one history)");
+  if (s.n_nonfinite) return fail(c, NT_ERR_NONFINITE, "%llu particles ended non-finite", (unsigned long long)s.n_nonfinite);
+  if (s.n_event_cap) return fail(c, NT_ERR_EVENT_CAP, "%llu histories hit max_events_per_history", (unsigned long long)s.n_event_cap);
+  if (s.n_xs_range) return fail(c, NT_ERR_XS_RANGE, "%llu lookups outside the table range", (unsigned long long)s.n_xs_range);
+  return NT_OK;
+}
+
+static nt_status step_prologue(nt_ctx* c, double dt) {
   if (c->stage < ST_PARTICLES) return fail(c, NT_ERR_STATE, "nt_inject_particles must come first");
   if (!(dt > 0.0) || !is_fin(dt)) return fail(c, NT_ERR_ARG, "dt must be finite and > 0");
   NT_CUDA(c, c->scratch.ensure(1024));
   // per-thread statistic slots for the largest persistent grid (16 CTAs per SM)
   NT_CUDA(c, c->slots.ensure((size_t)c->sm_count * 16 * kHistoryBlock * SF_COUNT * 8));
+  NT_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
+  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, (size_t)c->cells_st * 8, c->stream));
+  NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 1024, c->stream));
+  NT_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
+  return NT_OK;
+}
+
+nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  {
+    const nt_status st = step_prologue(c, dt);
+    if (st != NT_OK) return st;
+  }
   const size_t cells = (size_t)c->cells_st;   // storage layout (tiles padded with zeros)
   uint32_t launches = 0;
   const bool det = c->opt.deterministic != 0;
-
-  NT_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
-  NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, cells * 8, c->stream));
-  NT_CUDA(c, cudaMemsetAsync(c->scratch.p, 0, 1024, c->stream));
-  NT_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
   const TrackParams tp = make_params(c, dt);
   {
-    const nt_status st = det ? run_det(c, tp, launches) : track_range(c, tp, false, launches);
+    const nt_status st = c->opt.decomposition == 1 ? run_slab_nccl(c, tp, launches)
+                         : det ? run_det(c, tp, launches) : track_range(c, tp, false, launches);
     if (st != NT_OK) return st;
   }
   NT_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
@@ -788,37 +1023,92 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   float track_ms = 0.f, step_ms = 0.f;
   cudaEventElapsedTime(&track_ms, c->ev[1], c->ev[2]);
   cudaEventElapsedTime(&step_ms, c->ev[0], c->ev[2]);
-  nt_step_stats s{};
-  s.n_alive_start = (uint64_t)hs[SU_ALIVE];
-  s.n_facets = (uint64_t)hs[SU_FACETS];
-  s.n_collisions = (uint64_t)hs[SU_COLLISIONS];
-  s.n_census = (uint64_t)hs[SU_CENSUS];
-  s.n_killed = (uint64_t)hs[SU_KILLED];
-  s.n_xs_range = (uint64_t)hs[SU_XS_RANGE];
-  s.n_nonfinite = (uint64_t)hs[SU_NONFINITE];
-  s.n_event_cap = (uint64_t)hs[SU_EVENT_CAP];
-  s.tally_total = hs[SU_COUNT + SF_TALLY];
-  s.census_energy = hs[SU_COUNT + SF_CENSUS_E];
-  s.census_weight = hs[SU_COUNT + SF_CENSUS_W];
-  s.killed_energy = hs[SU_COUNT + SF_KILLED_E];
-  s.killed_weight = hs[SU_COUNT + SF_KILLED_W];
-  s.absorbed_weight = hs[SU_COUNT + SF_ABSORBED_W];
-  s.n_escaped = (uint64_t)hs[SU_ESCAPED];
-  s.n_absorbed = (uint64_t)hs[SU_ABSORBED];
-  s.escaped_energy = hs[SU_COUNT + SF_ESCAPED_E];
-  s.escaped_weight = hs[SU_COUNT + SF_ESCAPED_W];
-  s.absorbed_energy = hs[SU_COUNT + SF_ABSORBED_E];
-  s.roulette_gain = hs[SU_COUNT + SF_ROULETTE];
-  s.track_ms = track_ms;
-  s.reduce_ms = reduce_ms;
-  s.step_ms = step_ms + reduce_ms;
-  s.n_launches = launches;
-  if (stats) *stats = s;
-  c->stage = ST_STEPPED;
-  if (hs[SU_REC_OVERFLOW] > 0) return fail(c, NT_ERR_UNSUPPORTED, "flush sequence overflow (>2^24 flushes in one history)");
-  if (s.n_nonfinite) return fail(c, NT_ERR_NONFINITE, "%llu particles ended non-finite", (unsigned long long)s.n_nonfinite);
-  if (s.n_event_cap) return fail(c, NT_ERR_EVENT_CAP, "%llu histories hit max_events_per_history", (unsigned long long)s.n_event_cap);
-  if (s.n_xs_range) return fail(c, NT_ERR_XS_RANGE, "%llu lookups outside the table range", (unsigned long long)s.n_xs_range);
+  return finish_stats(c, hs, track_ms, reduce_ms, step_ms, launches, stats);
+}
+
+// ---- x-slab decomposition driven by the caller ---------------------------------------------
+int64_t nt_slab_record_bytes(void) { return (int64_t)sizeof(SlabRec); }
+
+static nt_status slab_check(nt_ctx* c) {
+  if (!c) return NT_ERR_ARG;
+  cudaSetDevice(c->device);
+  if (c->opt.decomposition != 1) return fail(c, NT_ERR_STATE, "the context was not created with decomposition = 1");
+  return NT_OK;
+}
+
+nt_status nt_slab_begin(nt_ctx* c, double dt) {
+  nt_status st = slab_check(c);
+  if (st != NT_OK) return st;
+  st = step_prologue(c, dt);
+  if (st != NT_OK) return st;
+  c->slab_dt = dt;
+  c->slab_round = 0;
+  c->n_arr = 0;
+  c->slab_launches = 0;
+  return NT_OK;
+}
+
+nt_status nt_slab_round(nt_ctx* c, int64_t* n_emigrants) {
+  nt_status st = slab_check(c);
+  if (st != NT_OK) return st;
+  if (!n_emigrants) return fail(c, NT_ERR_ARG, "n_emigrants is NULL");
+  if (!(c->slab_dt > 0.0)) return fail(c, NT_ERR_STATE, "nt_slab_begin must come first");
+  const TrackParams tp = make_params(c, c->slab_dt);
+  return slab_round(c, tp, c->slab_launches, n_emigrants);
+}
+
+nt_status nt_slab_export(nt_ctx* c, void* dst, int64_t capacity, int64_t* n_left, int64_t* n_right) {
+  nt_status st = slab_check(c);
+  if (st != NT_OK) return st;
+  if (!dst || !n_left || !n_right) return fail(c, NT_ERR_ARG, "NULL argument");
+  unsigned long long n_out = 0;
+  NT_CUDA(c, cudaMemcpy(&n_out, c->scratch.as<char>() + 40, 8, cudaMemcpyDeviceToHost));
+  if ((int64_t)n_out > capacity) return fail(c, NT_ERR_ARG, "capacity %lld < %llu emigrants", (long long)capacity, n_out);
+  const TrackParams tp = make_params(c, c->slab_dt);
+  st = slab_pack(c, tp, (int64_t)n_out, n_left, n_right);
+  if (st != NT_OK) return st;
+  NT_CUDA(c, cudaMemcpyAsync(dst, c->slab_buf.p, (size_t)n_out * sizeof(SlabRec), cudaMemcpyDefault, c->stream));
+  NT_CUDA(c, slab_free_slots(c, (int64_t)n_out));
+  NT_CUDA(c, cudaMemsetAsync(c->scratch.as<char>() + 40, 0, 8, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  return NT_OK;
+}
+
+nt_status nt_slab_import(nt_ctx* c, const void* src, int64_t n) {
+  nt_status st = slab_check(c);
+  if (st != NT_OK) return st;
+  if (n < 0 || (n > 0 && !src)) return fail(c, NT_ERR_ARG, "bad import");
+  if (n == 0) return NT_OK;
+  NT_CUDA(c, c->slab_rbuf.ensure((size_t)n * sizeof(SlabRec)));
+  NT_CUDA(c, cudaMemcpyAsync(c->slab_rbuf.p, src, (size_t)n * sizeof(SlabRec), cudaMemcpyDefault, c->stream));
+  st = slab_unpack(c, c->slab_rbuf.as<SlabRec>(), n);
+  if (st != NT_OK) return st;
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  return NT_OK;
+}
+
+nt_status nt_slab_end(nt_ctx* c, nt_step_stats* stats) {
+  nt_status st = slab_check(c);
+  if (st != NT_OK) return st;
+  NT_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
+  unsigned long long hu[SU_COUNT];
+  double hf[SF_COUNT], hs[SU_COUNT + SF_COUNT];
+  char* s = c->scratch.as<char>();
+  NT_CUDA(c, cudaMemcpyAsync(hu, s + 256, sizeof hu, cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaMemcpyAsync(hf, s + 512, sizeof hf, cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  for (int k = 0; k < SU_COUNT; ++k) hs[k] = (double)hu[k];
+  for (int k = 0; k < SF_COUNT; ++k) hs[SU_COUNT + k] = hf[k];
+  float track_ms = 0.f, step_ms = 0.f;
+  cudaEventElapsedTime(&track_ms, c->ev[1], c->ev[2]);
+  cudaEventElapsedTime(&step_ms, c->ev[0], c->ev[2]);
+  c->slab_dt = 0.0;
+  return finish_stats(c, hs, track_ms, 0.f, step_ms, c->slab_launches, stats);
+}
+
+nt_status nt_particle_slots(nt_ctx* c, int64_t* n_slots) {
+  if (!c || !n_slots) return NT_ERR_ARG;
+  *n_slots = c->n_local;
   return NT_OK;
 }
 
@@ -859,7 +1149,7 @@ static nt_status copy_particles(nt_ctx* c, int64_t first, int64_t count, const n
       {v->e, c->p.e, 8}, {v->w, c->p.w, 8}, {v->mfp, c->p.mfp, 8}, {v->cx, c->p.cx, 4},
       {v->cy, c->p.cy, 4}, {v->ctr, c->p.ctr, 4}, {v->status, c->p.status, 1},
       {v->nfac, c->p.nfac, 4}, {v->ncol, c->p.ncol, 4}, {v->ncen, c->p.ncen, 4},
-      {v->dep, c->p.dep, 8}};
+      {v->dep, c->p.dep, 8}, {v->gid, c->p.gid, 8}};
   for (const F& x : f) {
     if (!x.host) continue;
     char* d = static_cast<char*>(x.dev) + (size_t)first * x.sz;

@@ -28,6 +28,16 @@ struct Soa {
   // mid-step state of a particle parked by the history kernel's collision deferral
   double *dcen, *acc, *dstep;  // census distance left, pending deposit, deposits flushed
   uint32_t *nf_s, *nc_s, *seq_s;   // facets, collisions, flush records so far this step
+  int64_t *gid;                // global id (RNG key); = first_id + local index unless slabs
+};
+
+// A particle migrating between x-slabs (decomposition 1): its store fields plus the
+// mid-step state of a parked particle.
+struct SlabRec {
+  int64_t gid;
+  double x, y, ox, oy, e, w, mfp, dcen, acc, dstep, dep;
+  int32_t cx, cy;
+  uint32_t ctr, nf, nc, seq, nfac, ncol, ncen, pad;
 };
 
 // Density storage (lossless): the f64 map, or -- when the map holds <= 256 (65536) distinct

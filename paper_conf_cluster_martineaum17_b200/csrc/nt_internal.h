@@ -21,12 +21,16 @@ struct TrackParams {
   int64_t max_events;
   int32_t refill_min;         // refill a warp's idle lanes once at least this many are idle
   // history kernel regime parking
-  int32_t phase;              // 1: track [lo, hi); >= 2: resume resume_q[0, *resume_count)
+  int32_t phase;              // 1: track [lo, hi) (resume_q null); 2: resume resume_q
   int32_t park_coll_below;    // park a colliding lane while fewer lanes of its warp collide
   const int32_t* resume_q;
   const unsigned long long* resume_count;
   int32_t* park_q;            // out-queue of parked local indices
   unsigned long long* park_count;
+  // x-slab decomposition (decomposition 1): particles leaving columns [slab_lo, slab_hi)
+  int32_t slab_lo, slab_hi;
+  int32_t* out_q;             // emigrant local indices
+  unsigned long long* out_count;
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]
@@ -61,7 +65,14 @@ void launch_inject(const InjectParams& ip, cudaStream_t s);
 // xs_search 2 (u8 + block map only): the cached-bin linear walk; 1 is a data change (the
 // caller passes tables without bucket index, nb = 0).
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
-                    int xs_search, cudaStream_t s);
+                    int xs_search, bool slab, cudaStream_t s);
+// Slab decomposition: pack the emigrants (out_q[0, n)) into records, those left of slab_lo
+// first (counter cnt[0]), the others from the end (cnt[1]); unpack n records into the slots
+// free_slots[0, n_free) and then [base, ...), status 2, and queue them in arr_q.
+void launch_slab_pack(const TrackParams& tp, const int32_t* out_q, int64_t n, SlabRec* dst,
+                      unsigned long long* cnt, cudaStream_t s);
+void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32_t* free_slots,
+                        int64_t n_free, int64_t base, int32_t* arr_q, cudaStream_t s);
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);

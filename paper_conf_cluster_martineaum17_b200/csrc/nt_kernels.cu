@@ -57,6 +57,7 @@ __global__ void __launch_bounds__(256) inject_kernel(const __grid_constant__ Inj
   P.p.ncol[i] = 0u;
   P.p.ncen[i] = 0u;
   P.p.dep[i] = 0.0;
+  P.p.gid[i] = (int64_t)pid;
 }
 
 void launch_inject(const InjectParams& ip, cudaStream_t s) {
@@ -80,9 +81,10 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
 template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg, bool kXsWalk,
-          bool kVar>
+          bool kVar, bool kSlab>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
+  static_assert(!(kSlab && kDet), "slab decomposition: production tally only");
   static_assert(!kBlk || kFmt == kDensU8, "the block map indexes u8 material codes");
   static_assert(!(kAgg && kDet), "aggregation reorders the sum: production tally only");
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
@@ -135,6 +137,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
   const uint64_t pol_keep = l2_evict_last();     // tally REDs, density gathers
   const uint64_t pol_stream = l2_evict_first();  // particle store (read / written once)
+  // global id of local particle i (the RNG key)
+  auto pid_of = [&](int32_t i_) -> uint64_t {
+    if constexpr (kSlab) return (uint64_t)__ldg(P.p.gid + i_);
+    else return (uint64_t)(P.first_id + i_);
+  };
   // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather
   auto dload = [&](int32_t cx_, int32_t cy_, uint32_t ci_) {
     if constexpr (kBlk) return dens_load_blk(P.mesh, s_blk, cx_, cy_, ci_, pol_keep);
@@ -161,9 +168,41 @@ history_kernel(const __grid_constant__ TrackParams P) {
   // store, its index to the out-queue, and the lane takes a new particle.  So the particles
   // that reach dense matter collide warp-converged in phase 2.  Per-particle results are
   // unchanged.
-  const bool resume = P.phase >= 2;
+  const bool resume = P.resume_q != nullptr;
   const unsigned long long span2 = resume ? *P.resume_count : span;
   const int park_coll_below = P.park_coll_below;
+  // Park this lane: the state before its next event to the particle store (status st), the
+  // index to queue q (one atomicAdd per group of converged lanes); the lane goes idle and
+  // takes a new particle.  Used for regime parking (status 2, park_q) and, with x-slabs,
+  // for emigrants (status 4, out_q).
+  auto park_to = [&](uint8_t st, int32_t* q, unsigned long long* qn) {
+    P.p.x[i] = x;
+    P.p.y[i] = y;
+    P.p.ox[i] = ox;
+    P.p.oy[i] = oy;
+    P.p.e[i] = e;
+    P.p.w[i] = w;
+    P.p.mfp[i] = mfp;
+    P.p.cx[i] = cx;
+    P.p.cy[i] = cy;
+    P.p.ctr[i] = ctr;
+    P.p.dcen[i] = dcen;
+    P.p.acc[i] = acc;
+    P.p.dstep[i] = dstep;
+    P.p.nf_s[i] = nf;
+    P.p.nc_s[i] = nc;
+    P.p.seq_s[i] = seq;
+    P.p.status[i] = st;
+    const unsigned am = __activemask();
+    const int ld = __ffs(am) - 1;
+    unsigned long long k = 0;
+    if (lane == ld) k = atomicAdd(qn, (unsigned long long)__popc(am));
+    k = __shfl_sync(am, k, ld) + (unsigned long long)__popc(am & lt_mask);
+    q[k] = i;
+    active = false;
+  };
+  auto outside_slab = [&](int32_t cx_) { return cx_ < P.slab_lo || cx_ >= P.slab_hi; };
+
   int thr = refill_min;   // break the event loop once this many lanes are idle (32: all)
   for (;;) {
     // ---- refill idle lanes with new particles: one atomic per warp ----
@@ -224,6 +263,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
               nc = P.p.nc_s[i];
               seq = P.p.seq_s[i];
             }
+            if constexpr (kSlab) {
+              // born (or resumed) outside this rank's slab: hand over before any event
+              if (outside_slab(cx)) park_to(4u, P.out_q, P.out_count);
+            }
           }
         }
       }
@@ -265,35 +308,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
           coll = dc < df && dc < ds;
         }
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
-        // park this lane: the state before this event to the particle store, the index to
-        // the out-queue (one atomicAdd per group of converged lanes), take a new particle
-        auto park = [&]() {
-          P.p.x[i] = x;
-          P.p.y[i] = y;
-          P.p.ox[i] = ox;
-          P.p.oy[i] = oy;
-          P.p.e[i] = e;
-          P.p.w[i] = w;
-          P.p.mfp[i] = mfp;
-          P.p.cx[i] = cx;
-          P.p.cy[i] = cy;
-          P.p.ctr[i] = ctr;
-          P.p.dcen[i] = dcen;
-          P.p.acc[i] = acc;
-          P.p.dstep[i] = dstep;
-          P.p.nf_s[i] = nf;
-          P.p.nc_s[i] = nc;
-          P.p.seq_s[i] = seq;
-          P.p.status[i] = 2u;
-          const unsigned am = __activemask();
-          const int ld = __ffs(am) - 1;
-          unsigned long long q = 0;
-          if (lane == ld) q = atomicAdd(P.park_count, (unsigned long long)__popc(am));
-          q = __shfl_sync(am, q, ld) + (unsigned long long)__popc(am & lt_mask);
-          P.park_q[q] = i;
-          active = false;
-        };
-
         auto flush = [&]() {
           const uint32_t cell = cidx;                // storage index of the current cell
           if constexpr (kDet) {
@@ -324,14 +338,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_KILLED_W, w);
           outcome = 2;
         } else if (coll && __popc(__activemask()) < park_coll_below) {
-          park();
+          park_to(2u, P.park_q, P.park_count);
         } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
           acc += ((w * dc) * sig) * m.H;
           x = x + dc * ox;
           y = y + dc * oy;
           dcen = dcen - dc;
-          const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+          const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, pid_of(i), P.seed);
           ctr += 1u;
           nc += 1u;
           double mfp_u = u01(r.b);                  // the draw for the new n_mfp
@@ -343,7 +357,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           } else if (u01(r.b) < m.pa) {            // sampled absorption (R31)
             absorbed = true;
           } else {                                  // scatter branch: n_mfp from the next counter
-            const U64x2 r2 = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+            const U64x2 r2 = threefry2x64_20((uint64_t)ctr, 0, pid_of(i), P.seed);
             ctr += 1u;
             mfp_u = u01(r2.a);
           }
@@ -369,7 +383,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
             bool kill = e < ph.e_min || w < ph.w_min;   // termination
             if (kVar && kill && ph.roulette && !(e < ph.e_min)) {
               // Russian roulette (R32): survive with probability w / w_s at weight w_s
-              const U64x2 r3 = threefry2x64_20((uint64_t)ctr, 0, (uint64_t)(P.first_id + i), P.seed);
+              const U64x2 r3 = threefry2x64_20((uint64_t)ctr, 0, pid_of(i), P.seed);
               ctr += 1u;
               if (u01(r3.a) < w / ph.w_roul) {
                 fsum(SF_ROULETTE, ph.w_roul - w);
@@ -434,6 +448,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
           cidx = cidx_of(cx, cy);
           draw = dload(cx, cy, cidx);                 // new cell's density
           nf += 1u;
+          if constexpr (kSlab) {
+            // entered the neighbour's slab: the facet is done, the neighbour continues
+            if (ax && !refl && outside_slab(cx)) park_to(4u, P.out_q, P.out_count);
+          }
         } else {
           // ---- census ----
           acc += ((w * ds) * sig) * m.H;
@@ -512,18 +530,28 @@ history_kernel(const __grid_constant__ TrackParams P) {
 template <bool kDet, bool kTiled, bool kVar>
 static void* history_fn(int fmt, bool blk, int minb, int agg, int xs) {
   if (fmt == kDensU8) {
-    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false, false, kVar>;
+    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false, false, kVar, false>;
     if constexpr (!kVar) {
-      if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, true, false>;
+      if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, true, false, false>;
       if constexpr (!kDet) {
-        if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false, false, false>;
-        if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false, false>;
+        if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false, false, false, false>;
+        if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false, false, false>;
       }
     }
-    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, false, kVar>;
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, false, kVar, false>;
   }
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false, kVar>;
-  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false, kVar>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false, kVar, false>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false, kVar, false>;
+}
+
+// x-slab decomposition kernels: production tally, physics variants compiled in.
+template <bool kTiled>
+static void* history_slab_fn(int fmt, bool blk) {
+  if (fmt == kDensU8)
+    return blk ? (void*)history_kernel<false, kDensU8, kTiled, true, 6, false, false, true, true>
+               : (void*)history_kernel<false, kDensU8, kTiled, false, 6, false, false, true, true>;
+  if (fmt == kDensU16) return (void*)history_kernel<false, kDensU16, kTiled, false, 6, false, false, true, true>;
+  return (void*)history_kernel<false, kDensF64, kTiled, false, 6, false, false, true, true>;
 }
 
 template <bool kVar>
@@ -535,16 +563,17 @@ static void* history_select_v(bool det, int fmt, bool tiled, bool blk, int minb,
 }
 
 static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs,
-                            bool var) {
+                            bool var, bool slab = false) {
+  if (slab) return tiled ? history_slab_fn<true>(fmt, blk) : history_slab_fn<false>(fmt, blk);
   return var ? history_select_v<true>(det, fmt, tiled, blk, minb, agg, xs)
              : history_select_v<false>(det, fmt, tiled, blk, minb, agg, xs);
 }
 
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
-                    int xs_search, cudaStream_t s) {
+                    int xs_search, bool slab, cudaStream_t s) {
   const bool var = tp.ph.vacuum || tp.ph.analog || tp.ph.roulette;
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode, xs_search, var);
+                            tally_mode, xs_search, var, slab);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
@@ -585,6 +614,56 @@ cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long*
                        unsigned long long n, int end_bit, cudaStream_t s) {
   return cub::DeviceRadixSort::SortPairs(temp, temp_bytes, kin, kout, vin, vout,
                                          (int64_t)n, 0, end_bit, s);
+}
+
+// ---------------------------------------------------------------------------------------
+// x-slab decomposition: emigrant records.
+__global__ void slab_pack_kernel(const __grid_constant__ TrackParams P, const int32_t* __restrict__ out_q,
+                                 int64_t n, SlabRec* __restrict__ dst, unsigned long long* cnt) {
+  const int64_t k = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (k >= n) return;
+  const int32_t i = out_q[k];
+  const bool left = P.p.cx[i] < P.slab_lo;
+  const unsigned long long slot = atomicAdd(cnt + (left ? 0 : 1), 1ull);
+  SlabRec& r = dst[left ? (int64_t)slot : n - 1 - (int64_t)slot];
+  r.gid = P.p.gid[i];
+  r.x = P.p.x[i]; r.y = P.p.y[i]; r.ox = P.p.ox[i]; r.oy = P.p.oy[i];
+  r.e = P.p.e[i]; r.w = P.p.w[i]; r.mfp = P.p.mfp[i];
+  r.dcen = P.p.dcen[i]; r.acc = P.p.acc[i]; r.dstep = P.p.dstep[i]; r.dep = P.p.dep[i];
+  r.cx = P.p.cx[i]; r.cy = P.p.cy[i]; r.ctr = P.p.ctr[i];
+  r.nf = P.p.nf_s[i]; r.nc = P.p.nc_s[i]; r.seq = P.p.seq_s[i];
+  r.nfac = P.p.nfac[i]; r.ncol = P.p.ncol[i]; r.ncen = P.p.ncen[i]; r.pad = 0u;
+}
+
+__global__ void slab_unpack_kernel(const Soa p, const SlabRec* __restrict__ src, int64_t n,
+                                   const int32_t* __restrict__ free_slots, int64_t n_free,
+                                   int64_t base, int32_t* __restrict__ arr_q) {
+  const int64_t k = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (k >= n) return;
+  const SlabRec& r = src[k];
+  const int64_t i = k < n_free ? (int64_t)free_slots[k] : base + (k - n_free);
+  p.gid[i] = r.gid;
+  p.x[i] = r.x; p.y[i] = r.y; p.ox[i] = r.ox; p.oy[i] = r.oy;
+  p.e[i] = r.e; p.w[i] = r.w; p.mfp[i] = r.mfp;
+  p.dcen[i] = r.dcen; p.acc[i] = r.acc; p.dstep[i] = r.dstep; p.dep[i] = r.dep;
+  p.cx[i] = r.cx; p.cy[i] = r.cy; p.ctr[i] = r.ctr;
+  p.nf_s[i] = r.nf; p.nc_s[i] = r.nc; p.seq_s[i] = r.seq;
+  p.nfac[i] = r.nfac; p.ncol[i] = r.ncol; p.ncen[i] = r.ncen;
+  p.status[i] = 2u;
+  arr_q[k] = (int32_t)i;
+}
+
+void launch_slab_pack(const TrackParams& tp, const int32_t* out_q, int64_t n, SlabRec* dst,
+                      unsigned long long* cnt, cudaStream_t s) {
+  if (n <= 0) return;
+  slab_pack_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(tp, out_q, n, dst, cnt);
+}
+
+void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32_t* free_slots,
+                        int64_t n_free, int64_t base, int32_t* arr_q, cudaStream_t s) {
+  if (n <= 0) return;
+  slab_unpack_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(p, src, n, free_slots, n_free,
+                                                                  base, arr_q);
 }
 
 // ---------------------------------------------------------------------------------------

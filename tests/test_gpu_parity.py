@@ -360,3 +360,60 @@ def test_nccl_allreduce_path_single_rank(nt, orc, mode):
     compare_tally(red, ot)
     compare_stats(s, os_)
     assert s["reduce_ms"] > 0.0
+
+
+# ---------------------------------------------------------------------------------------------
+# x-slab decomposition: several contexts on this GPU, one per slab,
+# exchanging emigrants through the caller-driven nt_slab_* calls.
+def _run_slabs(nt, cfg, nslabs, **opts):
+    ranks = []
+    for r in range(nslabs):
+        lo, n = wl.shard(cfg.n_particles, r, nslabs)
+        ranks.append(nt.setup(cfg, first_id=lo, n_local=n, rank=r, nranks=nslabs, decomposition=1,
+                              **opts))
+    for t in ranks:
+        t.slab_begin(cfg.dt)
+    rounds = 0
+    while True:
+        outs = [t.slab_round() for t in ranks]
+        rounds += 1
+        if sum(outs) == 0:
+            break
+        exp = [t.slab_export(n) for t, n in zip(ranks, outs)]
+        for r, (recs, nl, nr) in enumerate(exp):
+            assert nl == 0 or r > 0, "emigrant left of slab 0"
+            assert nr == 0 or r < nslabs - 1, "emigrant right of the last slab"
+            if nl:
+                ranks[r - 1].slab_import(recs[:nl])
+            if nr:
+                ranks[r + 1].slab_import(recs[nl:])
+    stats = [t.slab_end() for t in ranks]
+    tally = sum(t.read_tally(reduced=False) for t in ranks)
+    parts = [t.read_particles() for t in ranks]
+    for t in ranks:
+        t.close()
+    # gather the particles by global id (slots of emigrants keep status 4)
+    n = cfg.n_particles
+    out = {k: np.zeros(n, dtype=v.dtype) for k, v in parts[0].items()}
+    seen = np.zeros(n, dtype=np.int64)
+    for p in parts:
+        keep = p["status"] <= 1
+        g = p["gid"][keep]
+        seen[g] += 1
+        for k in out:
+            out[k][g] = p[k][keep]
+    assert np.all(seen == 1), "every particle ends on exactly one slab"
+    tot = {k: sum(s[k] for s in stats) for k in stats[0] if k not in ("status",)}
+    return tally, out, tot, rounds
+
+
+@pytest.mark.parametrize("nslabs", [2, 3])
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "tiny_stream", "tiny_split", "tiny_mid_bc", "small_csp"])
+def test_slab_decomposition_matches_oracle(nt, orc, cfgname, nslabs):
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, gs, rounds = _run_slabs(nt, cfg, nslabs)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)                  # per-particle results: identical to replicated
+    compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+    compare_stats(gs, os_, rtol=1e-9)
+    assert rounds >= 2 if cfg.density != "uniform_hi" else True
