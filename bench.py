@@ -184,6 +184,7 @@ def parse():
                     help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
     ap.add_argument("--json-out", default=None)
     ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
+    ap.add_argument("--particles", type=int, default=0, help="experiment: override the particle count")
     return ap.parse_args()
 
 
@@ -246,6 +247,8 @@ def main():
     cfg = wl.CONFIGS[a.config]
     if a.mesh:
         cfg = cfg.with_(nx=a.mesh, ny=a.mesh, name=f"{cfg.name}@{a.mesh}")
+    if a.particles:
+        cfg = cfg.with_(n_particles=a.particles, name=f"{cfg.name}@{a.particles}p")
     if a.table_size:
         cfg = cfg.with_(tables=wl.Tables(n_scatter=a.table_size, n_capture=max(2, 3 * a.table_size // 4)),
                         name=f"{cfg.name}@xs{a.table_size}")

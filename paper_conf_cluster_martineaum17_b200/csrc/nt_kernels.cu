@@ -93,7 +93,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
   constexpr int kWarps = kHistoryBlock / 32;
   __shared__ uint32_t s_u[kWarps][SU_COUNT];
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
-  __shared__ uint8_t s_blk[kBlk ? kBlkMax : 1];
+  __shared__ __align__(16) uint8_t s_blk[kBlk ? kBlkMax : 1];
+  __shared__ double s_wabs[kHistoryBlock];   // weight absorbed by implicit capture, per thread
   const int t = threadIdx.x;
   const int64_t gt = (int64_t)blockIdx.x * kHistoryBlock + t;
   const int64_t sstride = (int64_t)gridDim.x * kHistoryBlock;
@@ -114,7 +115,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const int wid = t >> 5;
   auto cnt = [&](int k, uint32_t v) { atomicAdd(&s_u[wid][k], v); };
   auto fsum = [&](int k, double v) { sf[k * sstride] += v; };
-  double wabs = 0.0;   // weight absorbed by implicit capture, this thread
+  s_wabs[t] = 0.0;
   const double* __restrict__ ndtab = (kFmt == kDensU8) ? s_nd : P.mesh.nd_tab;
 
   const int lane = t & 31;
@@ -124,7 +125,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const double* __restrict__ ey = P.mesh.ey;
   const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
   const Phys& ph = P.ph;
-  const int refill_min = P.refill_min;
   const uint32_t strip = 16u * (uint32_t)P.mesh.ntx;    // tiled: cells per row of tiles
   // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, as nt_device.cuh cell_index
   // (32-bit: nt_init_mesh guarantees the storage fits 2^32 cells)
@@ -159,7 +159,15 @@ history_kernel(const __grid_constant__ TrackParams P) {
   Mat m{0, 0, 0};
   int32_t cx = 0, cy = 0;
   uint32_t cidx = 0;         // storage index of (cx, cy)
-  uint32_t ctr = 0, nf = 0, nc = 0, seq = 0, nrange = 0;
+  uint32_t ctr = 0, nf = 0, nc = 0;
+  uint32_t seq = 0;          // flush sequence number (deterministic records only)
+  // XS clamp counts go straight to the warp's shared counter (rare)
+  auto xs_refresh = [&](double e_) {
+    uint32_t nr = 0;
+    const Mat mm = refresh_xs(P.xs, ph, e_, nr);
+    if (nr) cnt(SU_XS_RANGE, nr);
+    return mm;
+  };
   int32_t bin_s = 0, bin_a = 0;   // kXsWalk: the bins of the last lookup
 
   // Regime parking: phase 1 tracks particles [lo, hi); phase 2 resumes the
@@ -191,7 +199,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
     P.p.dstep[i] = dstep;
     P.p.nf_s[i] = nf;
     P.p.nc_s[i] = nc;
-    P.p.seq_s[i] = seq;
+    if constexpr (kDet) P.p.seq_s[i] = seq;
     P.p.status[i] = st;
     const unsigned am = __activemask();
     const int ld = __ffs(am) - 1;
@@ -203,18 +211,16 @@ history_kernel(const __grid_constant__ TrackParams P) {
   };
   auto outside_slab = [&](int32_t cx_) { return cx_ < P.slab_lo || cx_ >= P.slab_hi; };
 
-  int thr = refill_min;   // break the event loop once this many lanes are idle (32: all)
   for (;;) {
     // ---- refill idle lanes with new particles: one atomic per warp ----
     const unsigned idle = __ballot_sync(kFull, !active);
-    if (!exhausted && idle != 0u && (__popc(idle) >= refill_min || idle == kFull)) {
+    if (!exhausted && idle != 0u && (__popc(idle) >= P.refill_min || idle == kFull)) {
       const int leader = __ffs(idle) - 1;
       unsigned long long base = 0;
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
       base = __shfl_sync(kFull, base, leader);
       if (base + (unsigned long long)__popc(idle) >= span2) {
         exhausted = true;
-        thr = 32;
       }
       if (!active) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
@@ -245,7 +251,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
               bin_a = xs_bin(P.xs.c, clamp_only(e, P.xs.c));
             }
             if (!resume) {
-              m = refresh_xs(P.xs, ph, e, nrange);
+              m = xs_refresh(e);
               dcen = speed(e, ph) * P.dt;
               acc = 0.0;
               dstep = 0.0;
@@ -261,7 +267,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
               dstep = P.p.dstep[i];
               nf = P.p.nf_s[i];
               nc = P.p.nc_s[i];
-              seq = P.p.seq_s[i];
+              if constexpr (kDet) seq = P.p.seq_s[i];
             }
             if constexpr (kSlab) {
               // born (or resumed) outside this rank's slab: hand over before any event
@@ -277,8 +283,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
     }
 
     // ---- events until enough lanes are idle to refill (or none is active) ----
-    for (;;) {
-      if (active) {
+    auto event = [&]() __attribute__((always_inline)) {
         // ---- one event (Listing 1) ----
         // consume the gathers issued by the previous facet (density code, next edge)
         double nd;
@@ -353,7 +358,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           if (!(kVar && ph.analog)) {               // implicit capture
             const double w_old = w;
             w = w * (1.0 - m.pa);
-            wabs += w_old - w;
+            s_wabs[t] += w_old - w;
           } else if (u01(r.b) < m.pa) {            // sampled absorption (R31)
             absorbed = true;
           } else {                                  // scatter branch: n_mfp from the next counter
@@ -363,7 +368,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           }
           if (absorbed) {
             flush();
-            wabs += w;
+            s_wabs[t] += w;
             fsum(SF_ABSORBED_E, w * e);
             cnt(SU_ABSORBED, 1u);
             outcome = 2;
@@ -401,8 +406,13 @@ history_kernel(const __grid_constant__ TrackParams P) {
               exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
               eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
               dcen = tcen * speed(e, ph);
-              if constexpr (kXsWalk) m = refresh_xs_walk(P.xs, ph, e, nrange, bin_s, bin_a);
-              else m = refresh_xs(P.xs, ph, e, nrange);
+              if constexpr (kXsWalk) {
+                uint32_t nr = 0;
+                m = refresh_xs_walk(P.xs, ph, e, nr, bin_s, bin_a);
+                if (nr) cnt(SU_XS_RANGE, nr);
+              } else {
+                m = xs_refresh(e);
+              }
               iox = 1.0 / ox;
               ioy = 1.0 / oy;
               if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
@@ -493,14 +503,24 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_TALLY, dstep);
           active = false;
         }
+    };
+    // Two copies of the loop, so the exit test needs no register for the threshold: while
+    // particles remain, leave once refill_min lanes are idle; after that, once all are.
+    if (!exhausted) {
+      for (;;) {
+        if (active) event();
+        if (__popc(__ballot_sync(kFull, !active)) >= P.refill_min) break;
       }
-      if (__popc(__ballot_sync(kFull, !active)) >= thr) break;
+    } else {
+      for (;;) {
+        if (active) event();
+        if (!__any_sync(kFull, active)) break;
+      }
     }
   }
 
   // ---- CTA reduction of the statistics, one atomic per statistic per CTA ----
-  if (nrange) cnt(SU_XS_RANGE, nrange);
-  fsum(SF_ABSORBED_W, wabs);
+  fsum(SF_ABSORBED_W, s_wabs[t]);
   __syncthreads();
   const int lane2 = t & 31;
   for (int k = wid; k < SU_COUNT + SF_COUNT; k += kWarps) {
