@@ -7,11 +7,16 @@ exceptions.  There is no CPU fallback: if the library is missing, loading fails 
 from __future__ import annotations
 
 import ctypes as C
+import os
 from pathlib import Path
 
 import numpy as np
 
 LIB_PATH = Path(__file__).resolve().parent / "lib" / "libneutral_b200.so"
+# profiling aid: NT_LIB_VARIANT=name loads lib/variants/libneutral_b200_<name>.so (an A/B build
+# of the same sources with different compile-time options, scripts/dev/build_variants.sh)
+if os.environ.get("NT_LIB_VARIANT"):
+    LIB_PATH = LIB_PATH.parent / "variants" / f"libneutral_b200_{os.environ['NT_LIB_VARIANT']}.so"
 
 NT_OK = 0
 STATUS = {0: "NT_OK", 1: "NT_ERR_ARG", 2: "NT_ERR_STATE", 3: "NT_ERR_OOM", 4: "NT_ERR_CUDA",

@@ -283,7 +283,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
     }
 
     // ---- events until enough lanes are idle to refill (or none is active) ----
-    auto event = [&]() __attribute__((always_inline)) {
+    // event(capped): capped = true handles the event-cap kill only (NT_INNER path)
+    auto event = [&](bool capped) __attribute__((always_inline)) {
         // ---- one event (Listing 1) ----
         // consume the gathers issued by the previous facet (density code, next edge)
         double nd;
@@ -292,20 +293,24 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const double sig = nd * m.st;
         // An axis with direction cosine 0 carries exn = iox = +inf (set where the direction
         // changes), so (exn - x) * iox = +inf without a select -- the "ω = 0 -> ∞" of §3.
-        double tx = (exn - x) * iox;
-        tx = tx < 0.0 ? 0.0 : tx;
-        double ty = (eyn - y) * ioy;
-        ty = ty < 0.0 ? 0.0 : ty;
-        const bool ax = tx < ty;
-        const double df = ax ? tx : ty;
+        // §3 clamps tx and ty at 0 and takes X iff clamped tx < clamped ty (tie -> Y).
+        // max(tx,0) < max(ty,0) <=> ty > 0 && tx < ty, and the clamped minimum is the
+        // minimum clamped, so one clamp of the chosen distance gives the same df (±0 and
+        // all; R28).
+        const double tx = (exn - x) * iox;
+        const double ty = (eyn - y) * ioy;
+        const bool ax = ty > 0.0 && tx < ty;
+        double df = ax ? tx : ty;
+        df = df < 0.0 ? 0.0 : df;
         const double ds = dcen;
         // dc = n_mfp / Sigma_t only matters if a collision is possible: when
-        // n_mfp > (min(df, ds) * Sigma_t) * (1 + 2^-50) the rounded quotient provably exceeds
+        // n_mfp > (min(df, ds) * Sigma_t) * (1 + 2^-20) the rounded quotient provably exceeds
         // min(df, ds), so the event is not a collision and dc is never used.
-        // (The relative-error argument needs a normal product: tiny ones take the division.)
+        // (The relative-error argument needs a normal product: below 2^-960 the division is
+        // taken.)  Both constants have a zero low word, so they are instruction immediates.
         const double dmin = df < ds ? df : ds;
         const double dsig = dmin * sig;
-        const bool maybe_coll = !(mfp > dsig * 1.0000000000000009) || dsig < 1e-290;
+        const bool maybe_coll = !(mfp > dsig * 0x1.00001p+0) || dsig < 0x1p-960;
         double dc = d_inf();
         bool coll = false;
         if (__builtin_expect(maybe_coll && sig > 0.0, 0)) {  // branch, not a select
@@ -334,7 +339,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
           acc = 0.0;
         };
 
+#if NT_INNER
+        if (capped) {
+#else
         if (nf + nc >= max_ev) {
+#endif
           // guard (R27): count, flush, kill
           cnt(SU_EVENT_CAP, 1u);
           flush();
@@ -431,9 +440,16 @@ history_kernel(const __grid_constant__ TrackParams P) {
           flush();                                    // deposit of the cell being left
           const int32_t c = ax ? cx : cy;
           const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
+#if NT_REFL2
+          // step, and reflect if the stepped index leaves [0, n): one unsigned compare
+          const int32_t cs = c + (pos ? 1 : -1);
+          const bool refl = (uint32_t)cs >= (uint32_t)(ax ? nx : ny);   // reflective
+          const int32_t c2 = refl ? c : cs;
+#else
           const int32_t last = (ax ? nx : ny) - 1;
           const bool refl = pos ? (c == last) : (c == 0);   // reflective boundary
           const int32_t c2 = refl ? c : (pos ? c + 1 : c - 1);
+#endif
           cx = ax ? c2 : cx;
           cy = ax ? cy : c2;
           if (refl) {                               // rare: a branch beats 8 selects
@@ -504,21 +520,51 @@ history_kernel(const __grid_constant__ TrackParams P) {
           active = false;
         }
     };
-    // Two copies of the loop, so the exit test needs no register for the threshold: while
-    // particles remain, leave once refill_min lanes are idle; after that, once all are.
+#if NT_INNER
+    // Each lane runs up to NT_INNER events between two warp votes; the per-lane bound
+    // lim = min(events so far + NT_INNER, max_events) also enforces the event cap (R27),
+    // whose kill is handled by event(true) once the bound is the cap.
+    auto run_lane = [&]() __attribute__((always_inline)) {
+      if (active) {
+        const uint32_t ne = nf + nc;
+        const uint32_t lim =
+            (ne < max_ev && max_ev - ne > (uint32_t)NT_INNER) ? ne + (uint32_t)NT_INNER : max_ev;
+        while (nf + nc < lim) {
+          event(false);
+          if (!active) break;
+        }
+        if (active && nf + nc >= max_ev) event(true);
+      }
+    };
     if (!exhausted) {
       for (;;) {
-        if (active) event();
+        run_lane();
         if (__popc(__ballot_sync(kFull, !active)) >= P.refill_min) break;
       }
     } else {
       for (;;) {
-        if (active) event();
+        run_lane();
+        if (!__any_sync(kFull, active)) break;
+      }
+    }
+  }
+#else
+    // Two copies of the loop, so the exit test needs no register for the threshold: while
+    // particles remain, leave once refill_min lanes are idle; after that, once all are.
+    if (!exhausted) {
+      for (;;) {
+        if (active) event(false);
+        if (__popc(__ballot_sync(kFull, !active)) >= P.refill_min) break;
+      }
+    } else {
+      for (;;) {
+        if (active) event(false);
         if (!__any_sync(kFull, active)) break;
       }
     }
   }
 
+#endif
   // ---- CTA reduction of the statistics, one atomic per statistic per CTA ----
   fsum(SF_ABSORBED_W, s_wabs[t]);
   __syncthreads();

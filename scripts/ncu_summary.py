@@ -83,19 +83,43 @@ def main():
         lines.append(f"DRAM traffic of this launch (read + write): {tr:.4g} B")
         lines.append("")
     lines.append(f"DRAM traffic of all captured launches: {traffic:.4g} B")
-    # source page: top stall-sampled SASS lines
+    # source page: top stall-sampled SASS lines, per captured kernel (the page repeats a
+    # "Kernel Name" row and a header row for every launch)
     try:
         src = list(csv.reader(io.StringIO(ncu(["-i", a.rep, "--page", "source", "--csv",
                                                 "--print-source", "sass"]))))
-        h = src[1]
-        body = src[2:]
-        iS, iW = h.index("Source"), h.index("Warp Stall Sampling (All Samples)")
-        iE, iT = h.index("Instructions Executed"), h.index("Avg. Threads Executed")
-        tot = sum(int(x[iW]) for x in body) or 1
-        lines += ["", f"### top {a.top} stall-sampled SASS instructions", "",
-                  "| # | share | executed | avg threads | SASS |", "|---|---|---|---|---|"]
-        for k, x in sorted(enumerate(body), key=lambda kx: -int(kx[1][iW]))[:a.top]:
-            lines.append(f"| {k} | {100 * int(x[iW]) / tot:.1f}% | {x[iE]} | {x[iT]} | `{x[iS].strip()}` |")
+        blocks, cur = [], None
+        for row in src:
+            if row and row[0] == "Kernel Name":
+                cur = {"name": row[1] if len(row) > 1 else "", "rows": []}
+                blocks.append(cur)
+            elif cur is not None and row and row[0] == "Address":
+                cur["h"] = row
+            elif cur is not None and row:
+                cur["rows"].append(row)
+        for nb, b in enumerate(blocks):
+            h, body = b["h"], b["rows"]
+            iS, iW = h.index("Source"), h.index("Warp Stall Sampling (All Samples)")
+            iE, iT = h.index("Instructions Executed"), h.index("Avg. Threads Executed")
+            num_ = lambda v: int(v) if v.strip().lstrip("-").isdigit() else 0  # noqa: E731
+            tot = sum(num_(x[iW]) for x in body) or 1
+            ex_tot = sum(num_(x[iE]) for x in body)
+            lines += ["", f"### launch {nb}: top {a.top} stall-sampled SASS instructions "
+                      f"({ex_tot:.4g} warp instructions executed)", "",
+                      "| # | share | executed | avg threads | SASS |", "|---|---|---|---|---|"]
+            for k, x in sorted(enumerate(body), key=lambda kx: -num_(kx[1][iW]))[:a.top]:
+                lines.append(f"| {k} | {100 * num_(x[iW]) / tot:.1f}% | {x[iE]} | {x[iT]} | `{x[iS].strip()}` |")
+            # executed-instruction mix by opcode (what the issue slots go to)
+            mix: dict[str, int] = {}
+            for x in body:
+                op = x[iS].strip().split()
+                if not op:
+                    continue
+                o = op[1] if op[0].startswith("@") and len(op) > 1 else op[0]
+                mix[o.split(".")[0]] = mix.get(o.split(".")[0], 0) + num_(x[iE])
+            lines += ["", f"opcode mix of launch {nb} (share of executed warp instructions): " +
+                      ", ".join(f"{o} {100 * v / max(ex_tot, 1):.1f}%" for o, v in
+                                sorted(mix.items(), key=lambda kv: -kv[1])[:24])]
     except Exception as e:  # noqa: BLE001
         lines.append(f"(source page unavailable: {e})")
     Path(a.out).write_text("\n".join(lines) + "\n")
