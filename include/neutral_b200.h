@@ -75,7 +75,7 @@ typedef struct {
     int32_t ctas_per_sm;       /* persistent CTAs per SM (0 -> occupancy maximum)         */
     int64_t det_batch;         /* deterministic mode: particles per batch (0 -> 65536)    */
     int32_t refill_min;        /* history mode: a warp refills its idle lanes once at least
-                                  this many are idle (0 -> 8)                              */
+                                  this many are idle (0 -> 4)                              */
     int32_t density_format;    /* 0: lossless u8/u16 material codes when the density map
                                   holds <= 256 / 65536 distinct values, else f64; with u8
                                   codes (<= 254 values) also a block map (the code of each

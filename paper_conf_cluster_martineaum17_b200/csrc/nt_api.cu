@@ -204,7 +204,7 @@ nt_status nt_options_default(nt_options* opt) {
   opt->w_min = 1.0e-3;
   opt->max_events_per_history = 1000000000ll;
   opt->det_batch = 65536;
-  opt->refill_min = 8;
+  opt->refill_min = 4;
   opt->defer_below = 8;
   return NT_OK;
 }
@@ -620,7 +620,7 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.seed = c->seed;
   tp.dt = dt;
   tp.max_events = c->opt.max_events_per_history;
-  tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 8;
+  tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 4;
 
   char* s = c->scratch.as<char>();
   tp.counter = reinterpret_cast<unsigned long long*>(s);

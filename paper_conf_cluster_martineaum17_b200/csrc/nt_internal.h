@@ -85,6 +85,9 @@ cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long*
                        unsigned long long n, int end_bit, cudaStream_t s);
 
 constexpr int kHistoryBlock = 128;
+// history kernel: events a lane may run between two warp votes (refill checks); the A/B
+// sweep in profiles/ab/r01_ab4_history_variants.md chose 256
+constexpr int kInnerEvents = 256;
 
 }  // namespace nt
 

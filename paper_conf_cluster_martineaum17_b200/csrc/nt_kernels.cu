@@ -283,7 +283,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
     }
 
     // ---- events until enough lanes are idle to refill (or none is active) ----
-    // event(capped): capped = true handles the event-cap kill only (NT_INNER path)
+    // event(capped): capped = true handles only the event-cap kill (R27)
     auto event = [&](bool capped) __attribute__((always_inline)) {
         // ---- one event (Listing 1) ----
         // consume the gathers issued by the previous facet (density code, next edge)
@@ -339,11 +339,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           acc = 0.0;
         };
 
-#if NT_INNER
         if (capped) {
-#else
-        if (nf + nc >= max_ev) {
-#endif
           // guard (R27): count, flush, kill
           cnt(SU_EVENT_CAP, 1u);
           flush();
@@ -440,16 +436,10 @@ history_kernel(const __grid_constant__ TrackParams P) {
           flush();                                    // deposit of the cell being left
           const int32_t c = ax ? cx : cy;
           const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
-#if NT_REFL2
           // step, and reflect if the stepped index leaves [0, n): one unsigned compare
           const int32_t cs = c + (pos ? 1 : -1);
           const bool refl = (uint32_t)cs >= (uint32_t)(ax ? nx : ny);   // reflective
           const int32_t c2 = refl ? c : cs;
-#else
-          const int32_t last = (ax ? nx : ny) - 1;
-          const bool refl = pos ? (c == last) : (c == 0);   // reflective boundary
-          const int32_t c2 = refl ? c : (pos ? c + 1 : c - 1);
-#endif
           cx = ax ? c2 : cx;
           cy = ax ? cy : c2;
           if (refl) {                               // rare: a branch beats 8 selects
@@ -520,15 +510,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
           active = false;
         }
     };
-#if NT_INNER
-    // Each lane runs up to NT_INNER events between two warp votes; the per-lane bound
-    // lim = min(events so far + NT_INNER, max_events) also enforces the event cap (R27),
+    // Each lane runs up to kInnerEvents events between two warp votes; the per-lane bound
+    // lim = min(events so far + kInnerEvents, max_events) also enforces the event cap (R27),
     // whose kill is handled by event(true) once the bound is the cap.
     auto run_lane = [&]() __attribute__((always_inline)) {
       if (active) {
         const uint32_t ne = nf + nc;
         const uint32_t lim =
-            (ne < max_ev && max_ev - ne > (uint32_t)NT_INNER) ? ne + (uint32_t)NT_INNER : max_ev;
+            (ne < max_ev && max_ev - ne > (uint32_t)kInnerEvents) ? ne + (uint32_t)kInnerEvents : max_ev;
         while (nf + nc < lim) {
           event(false);
           if (!active) break;
@@ -548,23 +537,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
       }
     }
   }
-#else
-    // Two copies of the loop, so the exit test needs no register for the threshold: while
-    // particles remain, leave once refill_min lanes are idle; after that, once all are.
-    if (!exhausted) {
-      for (;;) {
-        if (active) event(false);
-        if (__popc(__ballot_sync(kFull, !active)) >= P.refill_min) break;
-      }
-    } else {
-      for (;;) {
-        if (active) event(false);
-        if (!__any_sync(kFull, active)) break;
-      }
-    }
-  }
-
-#endif
   // ---- CTA reduction of the statistics, one atomic per statistic per CTA ----
   fsum(SF_ABSORBED_W, s_wabs[t]);
   __syncthreads();

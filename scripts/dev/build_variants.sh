@@ -1,6 +1,6 @@
 # usage: bash scripts/dev/build_variants.sh "name:-DFLAG=1 -DOTHER=0" ...
-# Builds nt_kernels.cu with the given -D flags, links it with the other objects of the last
-# full build (build/*.o), and writes lib/variants/libneutral_b200_<name>.so for A/B timing
+# Builds nt_kernels.cu and nt_event.cu with the given -D flags, links them with the other
+# objects of the last full build (build/*.o), and writes lib/variants/libneutral_b200_<name>.so for A/B timing
 # with NT_LIB_VARIANT=<name>.
 set -e
 ROOT=$(cd "$(dirname "$0")/../.." && pwd)
@@ -9,11 +9,16 @@ NCCL=$(python -c "import nvidia.nccl as n, os; print(list(n.__path__)[0])")
 mkdir -p $PKG/lib/variants $ROOT/build/variants
 for spec in "$@"; do
   name=${spec%%:*}; flags=${spec#*:}
-  nvcc -gencode arch=compute_100a,code=sm_100a -O3 -lineinfo -fmad=false -std=c++17 -Xcompiler -fPIC \
-       --expt-relaxed-constexpr -Xptxas -v -I$NCCL/include -I$ROOT/include $flags \
-       -c $PKG/csrc/nt_kernels.cu -o $ROOT/build/variants/nt_kernels_$name.o 2> $ROOT/build/variants/ptxas_$name.log
-  objs=$(ls $ROOT/build/*.o | grep -v nt_kernels.o)
+  for src in nt_kernels nt_event; do
+    nvcc -gencode arch=compute_100a,code=sm_100a -O3 -lineinfo -fmad=false -std=c++17 -Xcompiler -fPIC \
+         --expt-relaxed-constexpr -Xptxas -v -I$NCCL/include -I$ROOT/include $flags \
+         -c $PKG/csrc/$src.cu -o $ROOT/build/variants/${src}_$name.o 2> $ROOT/build/variants/ptxas_${src}_$name.log &
+  done
+  wait
+  cp $ROOT/build/variants/ptxas_nt_kernels_$name.log $ROOT/build/variants/ptxas_$name.log
+  objs=$(ls $ROOT/build/*.o | grep -v "nt_kernels.o\|nt_event.o")
   nvcc -gencode arch=compute_100a,code=sm_100a -shared -o $PKG/lib/variants/libneutral_b200_$name.so \
-       $objs $ROOT/build/variants/nt_kernels_$name.o -L$NCCL/lib -l:libnccl.so.2 -Xlinker -rpath,$NCCL/lib
+       $objs $ROOT/build/variants/nt_kernels_$name.o $ROOT/build/variants/nt_event_$name.o \
+       -L$NCCL/lib -l:libnccl.so.2 -Xlinker -rpath,$NCCL/lib
   echo "$name: $(grep -A2 'history_kernelILb0ELi2ELb1ELb1ELi6ELb0ELb0ELb0ELb0E' $ROOT/build/variants/ptxas_$name.log | sed -n 3p)"
 done

@@ -97,7 +97,13 @@ def main():
                 cur["h"] = row
             elif cur is not None and row:
                 cur["rows"].append(row)
-        for nb, b in enumerate(blocks):
+        seen, uniq = set(), []
+        for b in blocks:                        # the page can repeat a launch; keep one copy
+            key = (b["name"], len(b["rows"]), tuple(b["rows"][0]) if b["rows"] else ())
+            if b["rows"] and "h" in b and key not in seen:
+                seen.add(key)
+                uniq.append(b)
+        for nb, b in enumerate(uniq):
             h, body = b["h"], b["rows"]
             iS, iW = h.index("Source"), h.index("Warp Stall Sampling (All Samples)")
             iE, iT = h.index("Instructions Executed"), h.index("Avg. Threads Executed")
