@@ -34,9 +34,17 @@
 namespace nt {
 
 constexpr int kEvBlock = 256;
-constexpr int kACap = 1024;                 // particle slots per CTA
+#ifndef NT_EV_ACAP
+#define NT_EV_ACAP 1024
+#endif
+#ifndef NT_EV_MINB
+#define NT_EV_MINB 3
+#endif
+constexpr int kACap = NT_EV_ACAP;           // particle slots per CTA
 constexpr int kSlotsPerThread = kACap / kEvBlock;
-static_assert(kACap % kEvBlock == 0, "slots per thread");
+constexpr unsigned kAccBit = 4u;            // type-byte flag: the slot's C_ACC is non-zero
+
+static_assert(kACap % kEvBlock == 0 && kACap / kEvBlock <= 8, "slots per thread");
 
 // slot columns (8-byte words)
 enum Col : int {
@@ -91,6 +99,7 @@ struct EvKernel {
   uint64_t pol;             // L2 evict_last: tally REDs and density gathers
   double* cols;             // this CTA's slot columns
   int slot;                 // the slot being handled
+  const uint8_t* s_type;    // slot type bytes (bit 2: the slot's deposit accumulator is non-zero)
 
   __device__ double& c(int f) { return cols[f * kACap + slot]; }
   __device__ int2 ci2(int f) { return reinterpret_cast<int2*>(cols + f * kACap)[slot]; }
@@ -186,13 +195,15 @@ struct EvKernel {
       return 3;
     }
     const Dist d = dist(s, nd_of(s.cx, s.cy));
-    if (d.dc < d.df && d.dc < d.ds) return 0;
-    return d.df < d.ds ? 1 : 2;
+    const int ab = s.acc != 0.0 ? (int)kAccBit : 0;   // the slot's type bit for load_common
+    if (d.dc < d.df && d.dc < d.ds) return 0 | ab;
+    return (d.df < d.ds ? 1 : 2) | ab;
   }
 
   __device__ void load_common(St& s) {
     s.x = c(C_X); s.y = c(C_Y); s.mfp = c(C_MFP); s.dcen = c(C_DCEN);
-    s.acc = c(C_ACC); s.dstep = c(C_DSTEP);
+    s.acc = (s_type[slot] & kAccBit) ? c(C_ACC) : 0.0;   // most events start with acc == 0
+    s.dstep = c(C_DSTEP);
     s.ox = c(C_OX); s.oy = c(C_OY); s.iox = c(C_IOX); s.ioy = c(C_IOY);
     s.w = c(C_W); s.st = c(C_ST); s.H = c(C_H);
     const int2 cxy = ci2(C_CXY);
@@ -202,7 +213,8 @@ struct EvKernel {
   }
   __device__ void store_moved(const St& s) {     // what every event changes
     c(C_X) = s.x; c(C_Y) = s.y; c(C_MFP) = s.mfp; c(C_DCEN) = s.dcen;
-    c(C_ACC) = s.acc; c(C_DSTEP) = s.dstep;
+    if (s.acc != 0.0) c(C_ACC) = s.acc;          // read back only while the type bit is set
+    c(C_DSTEP) = s.dstep;
     si2(C_CXY, make_int2(s.cx, s.cy));
     si2(C_NFC, make_int2((int)s.nf, (int)s.nc));
   }
@@ -405,7 +417,7 @@ struct EvKernel {
 };
 
 template <bool kDet, int kFmt, bool kBlk>
-__global__ void __launch_bounds__(kEvBlock, 3) ev_loop_kernel(const __grid_constant__ EvParams E) {
+__global__ void __launch_bounds__(kEvBlock, NT_EV_MINB) ev_loop_kernel(const __grid_constant__ EvParams E) {
   const TrackParams& P = E.P;
   __shared__ unsigned long long s_u[SU_COUNT];
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
@@ -444,7 +456,7 @@ __global__ void __launch_bounds__(kEvBlock, 3) ev_loop_kernel(const __grid_const
   }
   __syncthreads();
   EvKernel<kDet, kFmt, kBlk> K{P, P.ph, s_nd, s_blk, s_u, P.slot_f + gt, sstride,
-                              l2_evict_last(), E.slots + (int64_t)bidx * kCols * kACap, 0};
+                              l2_evict_last(), E.slots + (int64_t)bidx * kCols * kACap, 0, s_type};
   const unsigned long long span = (unsigned long long)(P.hi - P.lo);
 
   for (unsigned it = 0;; ++it) {
@@ -487,12 +499,12 @@ __global__ void __launch_bounds__(kEvBlock, 3) ev_loop_kernel(const __grid_const
     __syncthreads();
     // ---- (3) compaction: the queues and the free list in slot order ----
     {
-      unsigned tys = 0u;                          // this thread's kSlotsPerThread type bytes
+      unsigned long long tys = 0ull;              // this thread's kSlotsPerThread (<= 8) type bytes
       unsigned c01 = 0u, c23 = 0u;                // per-type counts, two 16-bit fields each
 #pragma unroll
       for (int k = 0; k < kSlotsPerThread; ++k) {
-        const unsigned ty = s_type[t * kSlotsPerThread + k];
-        tys |= ty << (8 * k);
+        const unsigned ty = s_type[t * kSlotsPerThread + k] & 3u;
+        tys |= (unsigned long long)ty << (8 * k);
         if (ty < 2u) c01 += 1u << (16 * ty); else c23 += 1u << (16 * (ty - 2u));
       }
       unsigned i01 = c01, i23 = c23;              // inclusive warp scans
@@ -523,7 +535,7 @@ __global__ void __launch_bounds__(kEvBlock, 3) ev_loop_kernel(const __grid_const
       unsigned p3 = s_wsum[wid][3] + ((i23 - c23) >> 16);
 #pragma unroll
       for (int k = 0; k < kSlotsPerThread; ++k) {
-        const unsigned ty = (tys >> (8 * k)) & 0xffu;
+        const unsigned ty = (unsigned)(tys >> (8 * k)) & 0xffu;
         const unsigned p = ty == 0u ? p0++ : (ty == 1u ? p1++ : (ty == 2u ? p2++ : p3++));
         s_q[ty][p] = (uint16_t)(t * kSlotsPerThread + k);
       }

@@ -18,8 +18,10 @@ import json; d=json.load(open('$f')); r=d['roofline']
 print('$f'.split('/')[-1], f\"value={d['value']:.3e} ms={d['ms_per_step']:.2f} frac={r['frac']:.3f} clocks={d['clocks']['sm_mhz']}\")"; done
 ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv --log-file $OUT/launches_csp.csv \
     python bench.py --steps 2 --warmup 1 --no-cpu-baseline --no-e2e > $OUT/ncu_launch_bench.log 2>&1
-for c in csp stream; do
+for c in csp stream scatter; do
   ncu --set full --clock-control none --import-source on -k regex:history -s 2 -c 2 \
       -o $OUT/prof_${c} python bench.py --config $c --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > $OUT/ncu_$c.log 2>&1
 done
+ncu --set full --clock-control none --import-source on -k regex:ev_loop -c 1 \
+    -o $OUT/prof_csp_event python bench.py --mode event --steps 1 --warmup 0 --no-cpu-baseline --no-e2e > $OUT/ncu_csp_event.log 2>&1
 ls $OUT
