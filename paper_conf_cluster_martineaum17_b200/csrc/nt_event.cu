@@ -38,7 +38,7 @@ constexpr int kEvBlock = 256;
 #define NT_EV_ACAP 1024
 #endif
 #ifndef NT_EV_MINB
-#define NT_EV_MINB 3
+#define NT_EV_MINB 4
 #endif
 constexpr int kACap = NT_EV_ACAP;           // particle slots per CTA
 constexpr int kSlotsPerThread = kACap / kEvBlock;
