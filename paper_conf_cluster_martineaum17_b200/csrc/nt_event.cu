@@ -459,23 +459,25 @@ __global__ void __launch_bounds__(kEvBlock, NT_EV_MINB) ev_loop_kernel(const __g
                               l2_evict_last(), E.slots + (int64_t)bidx * kCols * kACap, 0, s_type};
   const unsigned long long span = (unsigned long long)(P.hi - P.lo);
 
-  for (unsigned it = 0;; ++it) {
-    // ---- (1) refill: new particles for the free slots once a block-size of them is free ----
-    if (t == 0) {
-      const unsigned nfree = s_n[3];
-      unsigned nnew = 0;
-      if (!s_exhausted && (nfree >= (unsigned)kEvBlock || nfree == (unsigned)kACap)) {
-        const unsigned long long base = atomicAdd(&E.ctl->counter, (unsigned long long)nfree);
-        if (base >= span) {
-          s_exhausted = 1;
-        } else {
-          nnew = (unsigned)(span - base < nfree ? span - base : nfree);
-          if (base + nfree >= span) s_exhausted = 1;
-          s_newbase = base;
-        }
+  // (1) refill: new particles for the free slots once a block-size of them is free (one
+  // thread; published by the barrier that follows.  Folding it into the compaction's
+  // barriers measured 11% slower: profiles/ab/r01_ab7_event_refill.md)
+  auto refill = [&](unsigned nfree) {
+    unsigned nnew = 0;
+    if (!s_exhausted && (nfree >= (unsigned)kEvBlock || nfree == (unsigned)kACap)) {
+      const unsigned long long base = atomicAdd(&E.ctl->counter, (unsigned long long)nfree);
+      if (base >= span) {
+        s_exhausted = 1;
+      } else {
+        nnew = (unsigned)(span - base < nfree ? span - base : nfree);
+        if (base + nfree >= span) s_exhausted = 1;
+        s_newbase = base;
       }
-      s_nnew = nnew;
     }
+    s_nnew = nnew;
+  };
+  for (unsigned it = 0;; ++it) {
+    if (t == 0) refill(s_n[3]);
     __syncthreads();
     const unsigned n0 = s_n[0], n1 = s_n[1], n2 = s_n[2], nnew = s_nnew;
     const unsigned n012 = n0 + n1 + n2, total = n012 + nnew;

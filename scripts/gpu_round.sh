@@ -24,4 +24,10 @@ for c in csp stream scatter; do
 done
 ncu --set full --clock-control none --import-source on -k regex:ev_loop -c 1 \
     -o $OUT/prof_csp_event python bench.py --mode event --steps 1 --warmup 0 --no-cpu-baseline --no-e2e > $OUT/ncu_csp_event.log 2>&1
+# summaries on the box (the reports themselves would exceed gpurun's 64 MiB return limit)
+for r in csp stream scatter csp_event; do
+  k=$(echo $r | sed 's/_event/\/event/; t; s/$/\/history/')
+  python scripts/ncu_summary.py $OUT/prof_$r.ncu-rep $OUT/ncu_${r}.md --traffic-key $k > /dev/null 2>&1
+done
+for r in stream scatter csp_event; do rm -f $OUT/prof_$r.ncu-rep; done
 ls $OUT

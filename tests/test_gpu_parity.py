@@ -417,3 +417,22 @@ def test_slab_decomposition_matches_oracle(nt, orc, cfgname, nslabs):
     compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
     compare_stats(gs, os_, rtol=1e-9)
     assert rounds >= 2 if cfg.density != "uniform_hi" else True
+
+
+@pytest.mark.parametrize("mode", ["history", "event"])
+@pytest.mark.parametrize("cap", [1, 255, 256, 257, 300, 600])
+@pytest.mark.parametrize("det", [True, False])
+def test_event_cap_across_vote_rounds(nt, orc, mode, cap, det):
+    """The event cap (R27) at, below and above the history kernel's 256-event bound between
+    warp votes: the bound that ends a lane's round also enforces the cap."""
+    c = wl.CONFIGS["tiny_stream"].with_(nx=256, ny=256, n_particles=400)   # ~450 facets each
+    gt, gp, (gs,) = _gpu_run(nt, c, deterministic=det, mode=mode, max_events=cap)
+    prob = orc.Problem(c, wl.density(c), wl.tables(c), max_events=cap)
+    op = orc.inject(prob, 0, c.n_particles)
+    ot = np.zeros((c.ny, c.nx))
+    os_ = orc.step(prob, op, 0, ot)
+    assert os_["n_event_cap"] > 0 if cap < 400 else True
+    assert gs["n_event_cap"] == os_["n_event_cap"]
+    compare_particles(gp, op)
+    compare_stats(gs, os_)
+    compare_tally(gt, ot, rtol=1e-9 if det else 1e-6, floor=1e-9 if det else 1e-12)
