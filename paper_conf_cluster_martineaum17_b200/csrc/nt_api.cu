@@ -334,6 +334,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   ml.ny = ny;
   ml.tiled = tiled;
   ml.ntx = ntx;
+  ml.strip = 16 * ntx;
   NT_CUDA(c, c->rho.ensure((size_t)cells * 8));
   NT_CUDA(c, c->tally.ensure((size_t)cells_st * 8));
   NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
@@ -504,6 +505,8 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     T[t]->nb = nbk[t];
     T[t]->shift = shift[t];
     T[t]->base = base[t];
+    T[t]->kfirst = h[2 * t][0];
+    T[t]->klast = h[2 * t][(size_t)len[2 * t] - 1];
   }
   c->stage = ST_XS;
   return NT_OK;
@@ -592,6 +595,7 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.mesh.rho = (c->tiled && c->dens_fmt == kDensF64) ? c->rho_st.as<double>() : c->rho.as<double>();
   tp.mesh.tiled = c->tiled;
   tp.mesh.ntx = c->ntx;
+  tp.mesh.strip = 16 * c->ntx;
   tp.mesh.rho8 = c->rho_code.as<uint8_t>();
   tp.mesh.rho16 = c->rho_code.as<uint16_t>();
   tp.mesh.nd_tab = c->nd_tab.as<double>();
@@ -1128,6 +1132,7 @@ nt_status nt_read_tally(nt_ctx* c, double* dst, int32_t reduced) {
     ml.ny = c->ny;
     ml.tiled = 1;
     ml.ntx = c->ntx;
+    ml.strip = 16 * c->ntx;
     NT_CUDA(c, launch_relayout(src, c->tally_rm.as<double>(), cells, ml, false, c->stream));
     src = c->tally_rm.as<double>();
   }

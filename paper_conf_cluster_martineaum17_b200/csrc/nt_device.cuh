@@ -63,7 +63,8 @@ struct Mesh {
   // code, kBlkMixed otherwise.  The history kernel keeps it in shared memory, so a facet
   // into a uniform block needs no global gather.  blk == nullptr: no block map.
   const uint8_t* __restrict__ blk;
-  int32_t bshift, nbx, nblk, pad2;
+  int32_t bshift, nbx, nblk;
+  int32_t strip;                      // 16 * ntx: cells per row of tiles (tiled layout)
 };
 
 constexpr uint32_t kBlkMixed = 255u;   // block-map entry: block holds more than one code
@@ -90,6 +91,7 @@ struct Table {
   const uint32_t* __restrict__ idx; // [nb + 1]
   uint64_t base;
   int32_t n, nb, shift, pad;
+  double kfirst, klast;             // k[0] and k[n-1], as kernel parameters (no load latency)
 };
 
 struct Tables {
@@ -320,7 +322,7 @@ __device__ __forceinline__ double xs_lookup(const Table& T, double e) {
   const double* __restrict__ k = T.k;
   const int32_t n = T.n;
   int32_t lo, hi;                             // k[lo] <= e < k[hi]
-  if (e >= __ldg(k + n - 1)) {
+  if (e >= T.klast) {
     lo = n - 2;
     hi = n - 1;
   } else if (T.nb > 0) {
@@ -347,18 +349,16 @@ struct Mat {
   double H;    // E - (sigma_s/sigma_t) * (E*f): expected heating response
 };
 
-__device__ __forceinline__ double clamp_count(double e, const double* __restrict__ k,
-                                              int32_t n, uint32_t& nrange) {
-  const double lo = __ldg(k), hi = __ldg(k + n - 1);
-  if (e < lo) { ++nrange; return lo; }
-  if (e > hi) { ++nrange; return hi; }
+__device__ __forceinline__ double clamp_count(double e, const Table& T, uint32_t& nrange) {
+  if (e < T.kfirst) { ++nrange; return T.kfirst; }
+  if (e > T.klast) { ++nrange; return T.klast; }
   return e;
 }
 
 __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, double e,
                                           uint32_t& nrange) {
-  const double es = clamp_count(e, T.s.k, T.s.n, nrange);
-  const double ea = clamp_count(e, T.c.k, T.c.n, nrange);
+  const double es = clamp_count(e, T.s, nrange);
+  const double ea = clamp_count(e, T.c, nrange);
   const double ss = xs_lookup(T.s, es);
   const double sa = xs_lookup(T.c, ea);
   const double t = ss + sa;
@@ -374,15 +374,14 @@ __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, doubl
 // the new bin is found by a linear walk from it (energies only fall in elastic scatter
 // off a target at rest, so the walk goes down).  Same bin as xs_lookup by definition.
 __device__ __forceinline__ double clamp_only(double e, const Table& T) {
-  const double lo = __ldg(T.k), hi = __ldg(T.k + T.n - 1);
-  return e < lo ? lo : (e > hi ? hi : e);
+  return e < T.kfirst ? T.kfirst : (e > T.klast ? T.klast : e);
 }
 
 // Bin of e (already in [k0, k_{N-1}]) by the bucketed binary search of xs_lookup.
 __device__ __forceinline__ int32_t xs_bin(const Table& T, double e) {
   const double* __restrict__ k = T.k;
   const int32_t n = T.n;
-  if (e >= __ldg(k + n - 1)) return n - 2;
+  if (e >= T.klast) return n - 2;
   int32_t lo = 0, hi = n - 1;
   if (T.nb > 0) {
     const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
@@ -410,8 +409,8 @@ __device__ __forceinline__ double xs_walk(const Table& T, double e, int32_t& bin
 
 __device__ __forceinline__ Mat refresh_xs_walk(const Tables& T, const Phys& ph, double e,
                                                uint32_t& nrange, int32_t& bin_s, int32_t& bin_a) {
-  const double es = clamp_count(e, T.s.k, T.s.n, nrange);
-  const double ea = clamp_count(e, T.c.k, T.c.n, nrange);
+  const double es = clamp_count(e, T.s, nrange);
+  const double ea = clamp_count(e, T.c, nrange);
   const double ss = xs_walk(T.s, es, bin_s);
   const double sa = xs_walk(T.c, ea, bin_a);
   const double t = ss + sa;

@@ -125,7 +125,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const double* __restrict__ ey = P.mesh.ey;
   const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
   const Phys& ph = P.ph;
-  const uint32_t strip = 16u * (uint32_t)P.mesh.ntx;    // tiled: cells per row of tiles
+  const uint32_t strip = (uint32_t)P.mesh.strip;        // tiled: cells per row of tiles
   // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, as nt_device.cuh cell_index
   // (32-bit: nt_init_mesh guarantees the storage fits 2^32 cells)
   auto cidx_of = [&](int32_t cx_, int32_t cy_) -> uint32_t {
@@ -725,8 +725,8 @@ __global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, in
   const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
   if (i >= n) return;
   uint32_t dummy = 0;
-  const double es = clamp_count(e[i], T.s.k, T.s.n, dummy);
-  const double ea = clamp_count(e[i], T.c.k, T.c.n, dummy);
+  const double es = clamp_count(e[i], T.s, dummy);
+  const double ea = clamp_count(e[i], T.c, dummy);
   os[i] = xs_lookup(T.s, es);
   oa[i] = xs_lookup(T.c, ea);
 }
