@@ -87,7 +87,7 @@ cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long*
 constexpr int kHistoryBlock = 128;
 // history kernel: events a lane may run between two warp votes (refill checks); the A/B
 // sweep in profiles/ab/r01_ab4_history_variants.md chose 256
-constexpr int kInnerEvents = 256;
+constexpr int kInnerEvents = 256;   // (also best for the parked-particle phase: ab9, ab10)
 
 }  // namespace nt
 

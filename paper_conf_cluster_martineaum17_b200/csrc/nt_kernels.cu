@@ -513,11 +513,12 @@ history_kernel(const __grid_constant__ TrackParams P) {
     // Each lane runs up to kInnerEvents events between two warp votes; the per-lane bound
     // lim = min(events so far + kInnerEvents, max_events) also enforces the event cap (R27),
     // whose kill is handled by event(true) once the bound is the cap.
+    constexpr uint32_t inner = (uint32_t)kInnerEvents;
     auto run_lane = [&]() __attribute__((always_inline)) {
       if (active) {
         const uint32_t ne = nf + nc;
         const uint32_t lim =
-            (ne < max_ev && max_ev - ne > (uint32_t)kInnerEvents) ? ne + (uint32_t)kInnerEvents : max_ev;
+            (ne < max_ev && max_ev - ne > inner) ? ne + inner : max_ev;
         while (nf + nc < lim) {
           event(false);
           if (!active) break;

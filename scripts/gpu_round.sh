@@ -6,6 +6,8 @@ mkdir -p $OUT
 python -c "import __graft_entry__ as g; g.build()"
 timeout 1200 python -m pytest tests -m gpu -x -q -p no:cacheprovider > $OUT/pytest_gpu.log 2>&1
 tail -1 $OUT/pytest_gpu.log | sed "s/^/PYTEST: /"
+timeout 600 python -c "import __graft_entry__ as g; g.smoke()" > $OUT/smoke.log 2>&1; echo "SMOKE rc=$?: $(tail -1 $OUT/smoke.log)"
+timeout 600 python bench.py --impl reference --steps 2 --warmup 1 > $OUT/bench_reference.log 2>&1; echo "REFERENCE: $(tail -1 $OUT/bench_reference.log | cut -c1-200)"
 python bench.py --json-out $OUT/bench_csp.json > $OUT/bench_csp.log 2>&1
 for c in stream scatter split stream_8m; do
   python bench.py --config $c --no-cpu-baseline --no-e2e --steps 5 --json-out $OUT/bench_$c.json > $OUT/bench_$c.log 2>&1
