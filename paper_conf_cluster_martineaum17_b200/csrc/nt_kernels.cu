@@ -566,6 +566,9 @@ history_kernel(const __grid_constant__ TrackParams P) {
 // block-map kernels also come with the cached-bin linear XS walk (xs_search 2), and the
 // production ones with a 72-register cap (7 CTAs per SM, ctas_per_sm = 7; the default is 80
 // registers, 6 CTAs per SM) and with warp-aggregated flushes (tally_mode 1).
+#ifndef NT_HIST_MINB
+#define NT_HIST_MINB 6   // resident CTAs per SM the default kernel is compiled for (A/B ab11)
+#endif
 template <bool kDet, bool kTiled, bool kVar>
 static void* history_fn(int fmt, bool blk, int minb, int agg, int xs) {
   if (fmt == kDensU8) {
@@ -577,7 +580,7 @@ static void* history_fn(int fmt, bool blk, int minb, int agg, int xs) {
         if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false, false, false>;
       }
     }
-    return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, false, kVar, false>;
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, false, false, kVar, false>;
   }
   if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false, kVar, false>;
   return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false, kVar, false>;
