@@ -177,8 +177,8 @@ struct EvKernel {
     Dist d;
     d.ax = tx < ty;
     d.df = d.ax ? tx : ty;
-    d.dc = sig > 0.0 ? s.mfp / sig : ev_inf();
     d.ds = s.dcen;
+    d.dc = sig > 0.0 ? s.mfp / sig : ev_inf();
     return d;
   }
 
