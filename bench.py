@@ -54,6 +54,16 @@ def measured_peaks() -> dict:
     return {"hbm_gbs": 6650.0, "source": "fallback (B200_PROFILING.md)"}
 
 
+def l2_red_peak():
+    """Scattered fp64 RED throughput of the L2 (REDs/s), measured by scripts/dev/red_microbench.cu
+    on a B200 (profiles/r01_v16_red_microbench.json): the best L2-resident footprint."""
+    p = ROOT / "profiles" / "r01_v16_red_microbench.json"
+    if not p.exists():
+        return None
+    d = json.loads(p.read_text())
+    return max(r["reds_per_s"] for r in d["results"] if r["footprint_MB"] < 100)
+
+
 def ncu_traffic(config: str, mode: str):
     """Per-launch DRAM bytes of the tracking kernel from a committed ncu --set full capture."""
     p = ROOT / "profiles" / "ncu_traffic.json"
@@ -309,6 +319,10 @@ def main():
     peaks = measured_peaks()
     achieved = ab / (track_ms / 1e3) / 1e9
     traffic = ncu_traffic(cfg.name, a.mode)
+    # one fp64 tally RED per flush: every facet, census and kill
+    reds = statistics.mean(s["n_facets"] + s["n_census"] + s["n_killed"] for s in stats) / world
+    red_peak = l2_red_peak()
+    red_rate = reds / (track_ms / 1e3)
     status = {s["status"] for s in stats}
     launches = sum(s["n_launches"] + 1 for s in stats)          # + inject kernel per step
 
@@ -378,6 +392,10 @@ def main():
                          "algorithmic_bytes_per_launch": ab, "kernel_ms": track_ms,
                          "kernel_share_of_step": track_ms / (ms / a.steps),
                          "peak_source": peaks["source"]},
+            "l2_red_roofline": None if red_peak is None else {
+                "bound": "l2_red", "achieved": red_rate, "peak": red_peak, "unit": "RED/s",
+                "frac": red_rate / red_peak, "reds_per_launch": reds,
+                "peak_source": "measured: scripts/dev/red_microbench.cu (profiles/r01_v16_red_microbench.json)"},
             "cpu_baseline": cpu,
             "e2e": e2e,
             "gpu_launches": launches,
