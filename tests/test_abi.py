@@ -94,3 +94,15 @@ def test_missing_library_fails_loudly(tmp_path, monkeypatch):
     monkeypatch.setattr(binding, "LIB_PATH", tmp_path / "nope.so")
     with pytest.raises(ImportError):
         binding.lib()
+
+
+def test_bench_roofline_inputs():
+    """bench.py's two roofline denominators load from committed, driver- or B200-measured files
+    (MEASURED_PEAKS.json; profiles/r01_v16_red_microbench.json), and its byte and
+    RED counts follow SURVEY §8(d) (24 B per facet, 16 B per flush, 138 B per particle)."""
+    import bench
+    assert bench.measured_peaks()["hbm_gbs"] > 1000.0
+    peak = bench.l2_red_peak()
+    assert peak is not None and 1e10 < peak < 1e12
+    s = {"n_facets": 10, "n_census": 2, "n_killed": 1, "n_alive_start": 3}
+    assert bench.algorithmic_bytes(s) == 24 * 10 + 16 * 3 + 138 * 3
