@@ -430,8 +430,20 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   if (!sk || !sv || !ck || !cv) return fail(c, NT_ERR_ARG, "table pointer is NULL");
   const double* src[4] = {sk, sv, ck, cv};
   const int64_t len[4] = {ns, ns, nc, nc};
-  std::vector<double> h[4];
-  for (int k = 0; k < 4; ++k) NT_CUDA(c, fetch(h[k], src[k], len[k], c->stream));
+  // host (pageable, pinned or managed) tables are validated and indexed in place and copied
+  // once; device tables are fetched to the host first
+  std::vector<double> hv[4];
+  const double* h[4];
+  for (int k = 0; k < 4; ++k) {
+    cudaPointerAttributes pa;
+    if (cudaPointerGetAttributes(&pa, src[k]) == cudaSuccess && pa.type == cudaMemoryTypeDevice) {
+      NT_CUDA(c, fetch(hv[k], src[k], len[k], c->stream));
+      h[k] = hv[k].data();
+    } else {
+      cudaGetLastError();   // clear a failed attribute query (plain host pointer on old drivers)
+      h[k] = src[k];
+    }
+  }
   for (int k = 0; k < 4; k += 2) {
     for (int64_t j = 0; j < len[k]; ++j) {
       if (!is_fin(h[k][j])) return fail(c, NT_ERR_ARG, "table %d key %lld not finite", k / 2, (long long)j);
@@ -446,7 +458,7 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   uint64_t base[2] = {0, 0};
   int32_t shift[2] = {0, 0}, nbk[2] = {0, 0};
   for (int t = 0; t < 2; ++t) {
-    const std::vector<double>& k = h[2 * t];
+    const double* k = h[2 * t];
     const int64_t n = len[2 * t];
     if (!(k[0] > 0.0)) continue;                       // index needs positive keys
     uint64_t b0, b1;
@@ -489,8 +501,8 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
-    NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k].data(), (size_t)len[k] * 8,
-                               cudaMemcpyHostToDevice, c->stream));
+    NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k], (size_t)len[k] * 8,
+                               cudaMemcpyDefault, c->stream));
   for (int t = 0; t < 2; ++t)
     if (!idx[t].empty())
       NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[4 + t], idx[t].data(), idx[t].size() * 4,
