@@ -53,7 +53,8 @@ class _Problem(C.Structure):
 _PFIELDS = [("x", np.float64), ("y", np.float64), ("ox", np.float64), ("oy", np.float64),
             ("e", np.float64), ("w", np.float64), ("mfp", np.float64), ("cx", np.int32),
             ("cy", np.int32), ("ctr", np.uint32), ("status", np.uint8), ("nfac", np.uint32),
-            ("ncol", np.uint32), ("ncen", np.uint32), ("dep", np.float64)]
+            ("ncol", np.uint32), ("ncen", np.uint32), ("dep", np.float64),
+            ("tfl", np.float64)]   # tfl: the oracle's flight-time ledger (no GPU counterpart)
 
 
 class _Particles(C.Structure):

@@ -167,6 +167,7 @@ void or_inject(const or_problem *pb, or_particles *pt, int64_t first_id,
         pt->ncol[i] = 0;
         pt->ncen[i] = 0;
         pt->dep[i] = 0.0;
+        pt->tfl[i] = 0.0;
     }
 }
 
@@ -193,6 +194,7 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
     int32_t cx = pt->cx[i], cy = pt->cy[i];
     uint32_t c = pt->ctr[i];
     double dep = pt->dep[i];
+    double tfl = pt->tfl[i];           /* flight-time ledger: += segment / speed */
     double acc = 0.0;
 
     or_mat m = or_refresh_xs(pb, e, &st->n_xs_range);
@@ -229,6 +231,7 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
         if (dc < df && dc < ds) {
             /* ---- collision ---- */
             acc += ((w * dc) * sig) * m.H;
+            tfl += dc / v;
             x = x + dc * ox;
             y = y + dc * oy;
             dcen = dcen - dc;
@@ -293,7 +296,6 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
                 break;
             }
             v = or_speed(e);
-            dcen = tcen * v;
             m = or_refresh_xs(pb, e, &st->n_xs_range);
             sig = nd * m.st;
             iox = 1.0 / ox;
@@ -303,6 +305,7 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
             /* ---- facet ---------------------------- */
             int escaped = 0;
             acc += ((w * df) * sig) * m.H;
+            tfl += df / v;
             double nm = mfp - df * sig;
             mfp = nm > 0.0 ? nm : 0.0;
             dcen = dcen - df;
@@ -343,6 +346,7 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
         } else {
             /* ---- census ------------------------------------ */
             acc += ((w * ds) * sig) * m.H;
+            tfl += ds / v;
             x = x + ds * ox;
             y = y + ds * oy;
             double nm = mfp - ds * sig;
@@ -359,6 +363,7 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
     pt->x[i] = x; pt->y[i] = y; pt->ox[i] = ox; pt->oy[i] = oy;
     pt->e[i] = e; pt->w[i] = w; pt->mfp[i] = mfp;
     pt->cx[i] = cx; pt->cy[i] = cy; pt->ctr[i] = c; pt->dep[i] = dep;
+    pt->tfl[i] = tfl;
 }
 
 void or_step(const or_problem *pb, or_particles *pt, int64_t first_id,

@@ -17,7 +17,10 @@
  * (P10), symmetry (P11), printed workload facts (P12); variants (R30-R32,
  * tests/test_oracle_variants.py): vacuum-escape closed form, escape/absorption/
  * roulette ledgers, the sampled-absorption branch law and counter budget,
- * roulette unbiasedness.
+ * roulette unbiasedness; census clock (tests/test_oracle_census.py): the flight-time
+ * ledger tfl equals k*dt at the k-th census (R21's distance-timer conversion through a
+ * collision), the first-flight law across a census (census n_mfp carry-over, R23), and
+ * the invariance of a history under splitting its timestep at a census.
  * Parity unpinned: absolute per-cell tally values at paper scale (the paper's
  * Fig. 2 plots are absent) -- only P10-P12 constrain them.
  */
@@ -63,6 +66,10 @@ typedef struct {
     uint8_t *status;               /* 1 = alive (at census), 0 = dead */
     uint32_t *nfac, *ncol, *ncen;  /* cumulative event counters */
     double *dep;                   /* cumulative energy this particle tallied */
+    double *tfl;                   /* cumulative flight time (s): sum over segments of
+                                    * length / speed -- an instrument of the oracle only
+                                    * (pins the census clock); it
+                                    * feeds back into nothing */
 } or_particles;
 
 /* Ledger of one step (sums over the particles stepped). */

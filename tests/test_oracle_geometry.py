@@ -134,3 +134,27 @@ def test_sharding_invariance(orc):
         assert np.array_equal(cat, getattr(p_all, name)), name
     tsum = tallies[0] + tallies[1] + tallies[2]
     assert np.allclose(tsum, t_all, rtol=1e-12, atol=0)
+
+
+def test_facet_axis_tie_goes_to_y(orc):
+    """Reading R16 (Listing 1 order; X-facet iff tx < ty): a particle
+    whose two facet distances are exactly equal crosses Y first, then X at distance ~0 (a
+    corner is two facets, R17).  Constructed input: a cell centre, direction (s, s)."""
+    cfg = wl.CONFIGS["tiny_vacuum"]
+    dx = cfg.width / cfg.nx
+    s = math.sqrt(0.5)
+    for cap, want in [(1, (3, 4, 1)), (2, (4, 4, 2))]:
+        prob = orc.Problem(cfg, wl.density(cfg), wl.tables(cfg), max_events=cap)
+        p = orc.Particles(4)
+        for k, (c0, ox, oy) in enumerate([(3, s, s), (3, -s, -s), (3, s, -s), (3, -s, s)]):
+            p.x[k] = p.y[k] = (c0 + 0.5) * dx
+            p.cx[k] = p.cy[k] = c0
+            p.ox[k], p.oy[k] = ox, oy
+            p.e[k], p.w[k], p.mfp[k], p.ctr[k], p.status[k] = cfg.e0, 1.0, 1.0, 2, 1
+        orc.step(prob, p, 0, np.zeros(cfg.nx * cfg.ny))
+        assert np.all(p.nfac == want[2])
+        # k = 0 moves +x +y: after the tie the first crossing is Y
+        assert (p.cx[0], p.cy[0]) == (want[0], want[1])
+        if cap == 1:
+            assert np.array_equal(p.cx, [3, 3, 3, 3])
+            assert np.array_equal(p.cy, [4, 2, 2, 4])
