@@ -216,8 +216,10 @@ nt_status nt_inject_particles(nt_ctx *ctx, int64_t n_total, int64_t first_id,
 nt_status nt_run_timestep(nt_ctx *ctx, double dt, nt_step_stats *stats);
 
 /* Copy the per-cell tally [ny][nx] (f64) of the last step into dst (host or device).
- * reduced = 1: the cross-rank sum (equal to the local tally when nranks == 1);
- * reduced = 0: this rank's own partial tally (kept only when nranks > 1). */
+ * reduced = 1: the cross-rank sum (equal to the local tally without a communicator);
+ * reduced = 0: this rank's own partial tally.  With a communicator the step allreduces
+ * out of place (local partial -> a second tally buffer), so both stay readable without a
+ * copy. */
 nt_status nt_read_tally(nt_ctx *ctx, double *dst, int32_t reduced);
 
 /* Copy local particles [first, first+count) (local indices) into dst's arrays. */
@@ -249,6 +251,9 @@ nt_status nt_slab_end(nt_ctx *ctx, nt_step_stats *stats);
 nt_status nt_particle_slots(nt_ctx *ctx, int64_t *n_slots);
 
 /* Verification entry points (run the device code paths in isolation). */
+/* Device allocations the library has made so far, process-wide (every cudaMalloc goes
+ * through one counter).  A timestep on a context whose buffers exist allocates nothing. */
+int64_t nt_debug_alloc_count(void);
 /* out[2i], out[2i+1] = threefry2x64_20(ctr = {in[4i], in[4i+1]}, key = {in[4i+2], in[4i+3]}). */
 nt_status nt_debug_threefry(nt_ctx *ctx, const uint64_t *in, int64_t n, uint64_t *out);
 /* Microscopic XS from the loaded tables: out_s[i], out_a[i] at energies[i] (no clamp

@@ -31,7 +31,7 @@ EXPORTS = ["nt_abi_version", "nt_build_info", "nt_status_string", "nt_options_de
            "nt_load_cross_sections", "nt_inject_particles", "nt_run_timestep", "nt_read_tally",
            "nt_read_particles", "nt_write_particles", "nt_slab_record_bytes", "nt_slab_begin",
            "nt_slab_round", "nt_slab_export", "nt_slab_import", "nt_slab_end", "nt_particle_slots",
-           "nt_debug_threefry", "nt_debug_xs"]
+           "nt_debug_threefry", "nt_debug_xs", "nt_debug_alloc_count"]
 
 
 class NeutralError(RuntimeError):
@@ -117,6 +117,7 @@ def lib():
             "nt_particle_slots": ([vp, C.POINTER(i64)], C.c_int),
             "nt_debug_threefry": ([vp, vp, i64, vp], C.c_int),
             "nt_debug_xs": ([vp, vp, i64, vp, vp], C.c_int),
+            "nt_debug_alloc_count": ([], i64),
         }
         for name, (args, res) in sigs.items():
             f = getattr(L, name)
@@ -124,6 +125,11 @@ def lib():
             f.restype = res
         _lib = L
     return _lib
+
+
+def alloc_count() -> int:
+    """Device allocations the library has made so far (process-wide)."""
+    return int(lib().nt_debug_alloc_count())
 
 
 def get_unique_id() -> bytes:
@@ -159,7 +165,16 @@ def _f64(a):
 
 
 class Tracker:
-    """One nt_ctx: a 2D mesh, two XS tables, this rank's particles, and its tally."""
+    """One nt_ctx: a 2D mesh, two XS tables, this rank's particles, and its tally.
+
+    Streams: the context orders its work on ``stream`` (a cudaStream_t handle, e.g.
+    ``torch.cuda.current_stream().cuda_stream``) or, when None, on a stream of its own.
+    CUDA tensors passed in or out are produced / consumed on torch's current stream: when
+    that is not the context's stream, the binding synchronises torch's current stream
+    before handing the pointer over (so a tensor is never read before its producer wrote
+    it, nor overwritten while a kernel still reads it); the library synchronises its own
+    stream before returning from every call that reads or writes caller memory.
+    """
 
     def __init__(self, device: int = 0, stream=None, mode: str = "history",
                  deterministic: bool = False, rank: int = 0, nranks: int = 1,
@@ -200,10 +215,20 @@ class Tracker:
         if st != NT_OK:
             raise NeutralError(st, "nt_create failed")
         self._h = h
+        self._stream = stream or 0
         self.nx = self.ny = 0
         self.n_local = 0
 
     # -- helpers ---------------------------------------------------------------------------
+    def _order(self, *arrays):
+        """Synchronise torch's current stream for CUDA tensors not on the context stream."""
+        for a in arrays:
+            if getattr(a, "is_cuda", False):
+                import torch
+                cur = torch.cuda.current_stream(a.device)
+                if self._stream == 0 or cur.cuda_stream != self._stream:
+                    cur.synchronize()
+
     def _check(self, st: int, what: str, allow=()):
         if st != NT_OK and st not in allow:
             raise NeutralError(st, f"{what}: {lib().nt_last_error(self._h).decode()}")
@@ -228,12 +253,15 @@ class Tracker:
 
     # -- the five calls of the boundary -------------------------------------------------------
     def init_mesh(self, nx: int, ny: int, width: float, height: float, density):
-        p, keep = _ptr(_f64(density))
+        dens = _f64(density)
+        self._order(dens)
+        p, keep = _ptr(dens)
         self._check(lib().nt_init_mesh(self._h, nx, ny, width, height, p), "nt_init_mesh")
         self.nx, self.ny = nx, ny
 
     def load_cross_sections(self, scatter_keys, scatter_vals, capture_keys, capture_vals):
         arrs = [_f64(a) for a in (scatter_keys, scatter_vals, capture_keys, capture_vals)]
+        self._order(*arrs)
         ps = [_ptr(a)[0] for a in arrs]
         self._check(lib().nt_load_cross_sections(self._h, ps[0], ps[1], len(arrs[0]), ps[2], ps[3],
                                                  len(arrs[2])), "nt_load_cross_sections")
@@ -287,6 +315,7 @@ class Tracker:
     def read_tally(self, out=None, reduced: bool = True):
         if out is None:
             out = np.empty((self.ny, self.nx), dtype=np.float64)
+        self._order(out)
         p, _ = _ptr(out)
         self._check(lib().nt_read_tally(self._h, p, int(reduced)), "nt_read_tally")
         return out

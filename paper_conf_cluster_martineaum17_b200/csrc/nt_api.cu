@@ -5,6 +5,7 @@
 // nt_kernels.cu / nt_event.cu.
 #include <nccl.h>
 
+#include <atomic>
 #include <cmath>
 #include <cstdarg>
 #include <cstdio>
@@ -23,6 +24,10 @@ namespace {
 
 enum Stage { ST_CREATED = 0, ST_MESH = 1, ST_XS = 2, ST_PARTICLES = 3, ST_STEPPED = 4 };
 
+// Device buffer that only grows.  ensure() frees the old allocation before it allocates
+// the new one, so a caller whose state points into the buffer lowers its stage first
+// (nt_load_cross_sections, nt_inject_particles): after a failed ensure nothing refers to
+// freed memory.
 struct DevBuf {
   void* p = nullptr;
   size_t bytes = 0;
@@ -32,7 +37,7 @@ struct DevBuf {
     p = nullptr;
     bytes = 0;
     if (b == 0) return cudaSuccess;
-    cudaError_t e = cudaMalloc(&p, b);
+    cudaError_t e = nt::device_malloc(&p, b);
     if (e == cudaSuccess) bytes = b;
     return e;
   }
@@ -46,6 +51,14 @@ struct DevBuf {
 
 }  // namespace
 
+namespace nt {
+static std::atomic<long long> g_device_allocs{0};
+cudaError_t device_malloc(void** p, size_t bytes) {
+  ++g_device_allocs;
+  return cudaMalloc(p, bytes);
+}
+}  // namespace nt
+
 struct nt_ctx {
   nt_options opt{};
   std::string err;
@@ -57,10 +70,14 @@ struct nt_ctx {
   cudaEvent_t ev[6] = {};
   ncclComm_t comm = nullptr;
   Phys ph{};
+  // step statistics as doubles: [SU_COUNT u64 counts][SF_COUNT sums] (device, and a
+  // pinned host copy read once per step)
+  DevBuf stats_d;
+  double* stats_h = nullptr;
   // mesh
   int32_t nx = 0, ny = 0;
   double W = 0, H = 0;
-  DevBuf rho, tally, tally_local, ex, ey;
+  DevBuf rho, tally, tally_red, ex, ey;  // tally_red: the cross-rank sum (comm only)
   DevBuf rho_code, nd_tab, enc_keys;     // lossless density encoding
   DevBuf blk;                            // block map of the u8 codes (Mesh::blk)
   int blk_shift = 0, blk_nbx = 0, blk_n = 0;   // blk_n = 0: no block map
@@ -276,6 +293,12 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
     c->own_stream = true;
   }
   for (auto& ev : c->ev) cudaEventCreate(&ev);
+  if (cudaHostAlloc(reinterpret_cast<void**>(&c->stats_h), (SU_COUNT + SF_COUNT) * sizeof(double),
+                    cudaHostAllocDefault) != cudaSuccess ||
+      c->stats_d.ensure((SU_COUNT + SF_COUNT) * sizeof(double)) != cudaSuccess) {
+    nt_destroy(c);
+    return NT_ERR_OOM;
+  }
   init_phys(c);
   if (opt.nccl_unique_id) {
     ncclUniqueId id;
@@ -295,10 +318,11 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
-  for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_local, &c->ex, &c->ey, &c->xs, &c->soa,
+  for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
-                    &c->sort_tmp, &c->backup})
+                    &c->sort_tmp, &c->backup, &c->stats_d})
     b->release();
+  if (c->stats_h) cudaFreeHost(c->stats_h);
   for (auto& ev : c->ev)
     if (ev) cudaEventDestroy(ev);
   if (c->comm) ncclCommDestroy(c->comm);
@@ -337,6 +361,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   ml.strip = 16 * ntx;
   NT_CUDA(c, c->rho.ensure((size_t)cells * 8));
   NT_CUDA(c, c->tally.ensure((size_t)cells_st * 8));
+  if (c->comm) NT_CUDA(c, c->tally_red.ensure((size_t)cells_st * 8));
   NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
   NT_CUDA(c, c->ey.ensure(((size_t)ny + 1) * 8));
   NT_CUDA(c, c->scratch.ensure(1024));
@@ -400,6 +425,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
     NT_CUDA(c, launch_relayout(c->rho.as<double>(), c->rho_st.as<double>(), cells, ml, true, c->stream));
   }
   NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, (size_t)cells_st * 8, c->stream));
+  if (c->comm) NT_CUDA(c, cudaMemsetAsync(c->tally_red.p, 0, (size_t)cells_st * 8, c->stream));
   launch_edges(c->ex.as<double>(), nx, width, c->ey.as<double>(), ny, height, c->stream);
   NT_CUDA(c, cudaGetLastError());
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
@@ -428,15 +454,18 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   if (ns < 2 || nc < 2 || ns > (1ll << 30) || nc > (1ll << 30))
     return fail(c, NT_ERR_ARG, "table sizes must be in [2, 2^30]");
   if (!sk || !sv || !ck || !cv) return fail(c, NT_ERR_ARG, "table pointer is NULL");
+  c->stage = ST_MESH;           // the tables are replaced: later stages are invalid from here
   const double* src[4] = {sk, sv, ck, cv};
   const int64_t len[4] = {ns, ns, nc, nc};
-  // host (pageable, pinned or managed) tables are validated and indexed in place and copied
-  // once; device tables are fetched to the host first
+  // host (pageable or pinned) tables are validated and indexed in place and copied once;
+  // device and managed tables are fetched to the host first (the fetch is ordered behind
+  // earlier work on the context stream, which may still be writing a managed table)
   std::vector<double> hv[4];
   const double* h[4];
   for (int k = 0; k < 4; ++k) {
     cudaPointerAttributes pa;
-    if (cudaPointerGetAttributes(&pa, src[k]) == cudaSuccess && pa.type == cudaMemoryTypeDevice) {
+    if (cudaPointerGetAttributes(&pa, src[k]) == cudaSuccess &&
+        (pa.type == cudaMemoryTypeDevice || pa.type == cudaMemoryTypeManaged)) {
       NT_CUDA(c, fetch(hv[k], src[k], len[k], c->stream));
       h[k] = hv[k].data();
     } else {
@@ -568,6 +597,7 @@ nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int6
   c->n_cap = slab ? (n_total > n_local ? n_total : n_local) : n_local;
   c->n_free = 0;
   c->n_arr = 0;
+  c->stage = ST_XS;             // the particle store is replaced: no step until it is rebuilt
   NT_CUDA(c, alloc_soa(c, c->n_cap));
   if (slab) {
     const int64_t P = c->opt.nranks, r = c->opt.rank;
@@ -1002,35 +1032,34 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
     if (st != NT_OK) return st;
   }
   NT_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
-  // stats: u64 slots then f64 slots, reduced over ranks as doubles (counts < 2^53 exact)
-  double hs[SU_COUNT + SF_COUNT];
+  // statistics -> one f64 vector on the device (u64 counts < 2^53 convert exactly); with a
+  // communicator the tally (out of place: the local partial stays in c->tally) and the
+  // statistics are summed over ranks in one NCCL group; one D2H copy, one synchronisation.
+  // Nothing here allocates (stats_d, stats_h and tally_red exist since nt_create /
+  // nt_init_mesh).
+  double* sd = c->stats_d.as<double>();
   {
-    unsigned long long hu[SU_COUNT];
-    double hf[SF_COUNT];
     char* s = c->scratch.as<char>();
-    NT_CUDA(c, cudaMemcpyAsync(hu, s + 256, sizeof hu, cudaMemcpyDeviceToHost, c->stream));
-    NT_CUDA(c, cudaMemcpyAsync(hf, s + 512, sizeof hf, cudaMemcpyDeviceToHost, c->stream));
-    if (c->comm) {
-      NT_CUDA(c, c->tally_local.ensure(cells * 8));
-      NT_CUDA(c, cudaMemcpyAsync(c->tally_local.p, c->tally.p, cells * 8, cudaMemcpyDeviceToDevice, c->stream));
-      NT_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
-      NT_NCCL(c, ncclAllReduce(c->tally.p, c->tally.p, cells, ncclFloat64, ncclSum, c->comm, c->stream));
-      NT_CUDA(c, cudaEventRecord(c->ev[4], c->stream));
-    }
-    NT_CUDA(c, cudaStreamSynchronize(c->stream));
-    for (int k = 0; k < SU_COUNT; ++k) hs[k] = (double)hu[k];
-    for (int k = 0; k < SF_COUNT; ++k) hs[SU_COUNT + k] = hf[k];
+    launch_stats_to_f64(reinterpret_cast<const unsigned long long*>(s + 256),
+                        reinterpret_cast<const double*>(s + 512), sd, c->stream);
+    ++launches;
+    NT_CUDA(c, cudaGetLastError());
   }
+  if (c->comm) {
+    NT_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    NT_NCCL(c, ncclGroupStart());
+    NT_NCCL(c, ncclAllReduce(c->tally.p, c->tally_red.p, cells, ncclFloat64, ncclSum, c->comm, c->stream));
+    NT_NCCL(c, ncclAllReduce(sd, sd, SU_COUNT + SF_COUNT, ncclFloat64, ncclSum, c->comm, c->stream));
+    NT_NCCL(c, ncclGroupEnd());
+    NT_CUDA(c, cudaEventRecord(c->ev[4], c->stream));
+  }
+  NT_CUDA(c, cudaMemcpyAsync(c->stats_h, sd, (SU_COUNT + SF_COUNT) * sizeof(double),
+                             cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  double hs[SU_COUNT + SF_COUNT];
+  std::memcpy(hs, c->stats_h, sizeof hs);
   float reduce_ms = 0.f;
   if (c->comm) {
-    // small stats allreduce through the same communicator
-    DevBuf tmp;
-    NT_CUDA(c, tmp.ensure(sizeof hs));
-    NT_CUDA(c, cudaMemcpyAsync(tmp.p, hs, sizeof hs, cudaMemcpyHostToDevice, c->stream));
-    NT_NCCL(c, ncclAllReduce(tmp.p, tmp.p, SU_COUNT + SF_COUNT, ncclFloat64, ncclSum, c->comm, c->stream));
-    NT_CUDA(c, cudaMemcpyAsync(hs, tmp.p, sizeof hs, cudaMemcpyDeviceToHost, c->stream));
-    NT_CUDA(c, cudaStreamSynchronize(c->stream));
-    tmp.release();
     cudaEventElapsedTime(&reduce_ms, c->ev[3], c->ev[4]);
     ncclResult_t async_err;
     ncclCommGetAsyncError(c->comm, &async_err);
@@ -1135,8 +1164,8 @@ nt_status nt_read_tally(nt_ctx* c, double* dst, int32_t reduced) {
   if (c->stage < ST_MESH) return fail(c, NT_ERR_STATE, "no mesh");
   if (!dst) return fail(c, NT_ERR_ARG, "dst is NULL");
   const int64_t cells = (int64_t)c->nx * (int64_t)c->ny;
-  const double* src = (!reduced && c->comm) ? c->tally_local.as<double>() : c->tally.as<double>();
-  if (!src) return fail(c, NT_ERR_STATE, "no local tally yet");
+  const double* src = (reduced && c->comm) ? c->tally_red.as<double>() : c->tally.as<double>();
+  if (!src) return fail(c, NT_ERR_STATE, "no tally yet");
   if (c->tiled) {            // storage layout -> row-major [ny][nx]
     NT_CUDA(c, c->tally_rm.ensure((size_t)cells * 8));
     Mesh ml{};
@@ -1188,6 +1217,8 @@ nt_status nt_write_particles(nt_ctx* c, int64_t first, int64_t count, const nt_p
 }
 
 // ---- verification entry points -----------------------------------------------------------
+int64_t nt_debug_alloc_count(void) { return (int64_t)nt::g_device_allocs.load(); }
+
 nt_status nt_debug_threefry(nt_ctx* c, const uint64_t* in, int64_t n, uint64_t* out) {
   if (!c || !in || !out || n < 0) return NT_ERR_ARG;
   cudaSetDevice(c->device);

@@ -597,14 +597,14 @@ nt_status event_run_range(EventState* s, const TrackParams& tp, bool det, int sm
   const int grid = sm_count * per_sm;
   cudaError_t e = cudaSuccess;
   if (!s->ctl) {
-    e = cudaMalloc(&s->ctl, sizeof(EvCtl));
+    e = device_malloc(reinterpret_cast<void**>(&s->ctl), sizeof(EvCtl));
     if (e != cudaSuccess) { s->ctl = nullptr; err = cudaGetErrorString(e); return NT_ERR_OOM; }
   }
   if (grid > s->slot_blocks) {
     if (s->slots) cudaFree(s->slots);
     s->slots = nullptr;
     s->slot_blocks = 0;
-    e = cudaMalloc(&s->slots, (size_t)grid * kCols * kACap * 8);
+    e = device_malloc(reinterpret_cast<void**>(&s->slots), (size_t)grid * kCols * kACap * 8);
     if (e != cudaSuccess) { s->slots = nullptr; err = cudaGetErrorString(e); return NT_ERR_OOM; }
     s->slot_blocks = grid;
   }
@@ -613,7 +613,7 @@ nt_status event_run_range(EventState* s, const TrackParams& tp, bool det, int sm
     if (s->slot_f) cudaFree(s->slot_f);
     s->slot_f = nullptr;
     s->slot_cap = 0;
-    e = cudaMalloc(&s->slot_f, (size_t)nslot * 8);
+    e = device_malloc(reinterpret_cast<void**>(&s->slot_f), (size_t)nslot * 8);
     if (e != cudaSuccess) { s->slot_f = nullptr; err = cudaGetErrorString(e); return NT_ERR_OOM; }
     s->slot_cap = nslot;
   }

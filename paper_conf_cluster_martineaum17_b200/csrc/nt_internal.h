@@ -84,6 +84,14 @@ cudaError_t sort_pairs(void* temp, size_t& temp_bytes, const unsigned long long*
                        unsigned long long* kout, const double* vin, double* vout,
                        unsigned long long n, int end_bit, cudaStream_t s);
 
+// Every device allocation of the library goes through device_malloc (nt_api.cu), which
+// counts them: nt_debug_alloc_count lets the tests assert that a timestep allocates
+// nothing once the context's buffers exist.
+cudaError_t device_malloc(void** p, size_t bytes);
+// out[k] = (double)su[k] for k < SU_COUNT, out[SU_COUNT + k] = sf[k] for k < SF_COUNT.
+void launch_stats_to_f64(const unsigned long long* su, const double* sf, double* out,
+                         cudaStream_t s);
+
 constexpr int kHistoryBlock = 128;
 // history kernel: events a lane may run between two warp votes (refill checks); the A/B
 // sweep in profiles/ab/r01_ab4_history_variants.md chose 256

@@ -709,6 +709,20 @@ void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32
 }
 
 // ---------------------------------------------------------------------------------------
+// Step statistics as one f64 vector (the NCCL allreduce and the single D2H read).
+__global__ void stats_to_f64_kernel(const unsigned long long* __restrict__ su,
+                                    const double* __restrict__ sf, double* __restrict__ out) {
+  const int k = threadIdx.x;
+  if (k < SU_COUNT) out[k] = (double)su[k];
+  else if (k < SU_COUNT + SF_COUNT) out[k] = sf[k - SU_COUNT];
+}
+
+void launch_stats_to_f64(const unsigned long long* su, const double* sf, double* out,
+                         cudaStream_t s) {
+  stats_to_f64_kernel<<<1, 32, 0, s>>>(su, sf, out);
+}
+
+// ---------------------------------------------------------------------------------------
 // Verification kernels.
 __global__ void threefry_debug_kernel(const uint64_t* __restrict__ in, int64_t n,
                                       uint64_t* __restrict__ out) {
