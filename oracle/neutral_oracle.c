@@ -296,6 +296,7 @@ static void or_history(const or_problem *pb, or_particles *pt, int64_t i,
                 break;
             }
             v = or_speed(e);
+            dcen = tcen * v;
             m = or_refresh_xs(pb, e, &st->n_xs_range);
             sig = nd * m.st;
             iox = 1.0 / ox;

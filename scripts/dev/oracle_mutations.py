@@ -1,6 +1,7 @@
 #!/usr/bin/env python
 """Mutation check of the oracle's pins: apply one plausible mistake at a time to
-oracle/neutral_oracle.c, rebuild, run the CPU pin suite (-m "not gpu"), restore.
+oracle/neutral_oracle.c, rebuild, run the CPU pin suite (-m "not gpu").  Works on a copy
+of the repository under /tmp, so the tree itself is never mutated.
 
 Every mutation must turn at least one pin red.  Output: one line per mutation with the
 failing test count (profiles/r02_oracle_mutations.txt holds the committed run).
@@ -8,13 +9,13 @@ failing test count (profiles/r02_oracle_mutations.txt holds the committed run).
     python scripts/dev/oracle_mutations.py [--out profiles/r02_oracle_mutations.txt]
 """
 import argparse
+import shutil
 import subprocess
 import sys
+import tempfile
 from pathlib import Path
 
-ROOT = Path(__file__).resolve().parents[2]
-SRC = ROOT / "oracle" / "neutral_oracle.c"
-LIB = ROOT / "oracle" / "liboracle.so"
+REPO = Path(__file__).resolve().parents[2]
 
 MUTATIONS = {
     "census timer not converted at a collision (drop dcen = tcen * v)":
@@ -57,6 +58,12 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--out", default=None)
     a = ap.parse_args()
+    tmp = Path(tempfile.mkdtemp(prefix="oracle_mut_"))
+    ROOT = tmp / "repo"
+    shutil.copytree(REPO, ROOT, ignore=shutil.ignore_patterns(".git", "gpurun_out", "profiles", "build",
+                                                              "__pycache__"))
+    SRC = ROOT / "oracle" / "neutral_oracle.c"
+    LIB = ROOT / "oracle" / "liboracle.so"
     orig = SRC.read_text()
     lines = []
     try:
@@ -73,8 +80,7 @@ def main():
             print(line, flush=True)
             lines.append(line)
     finally:
-        SRC.write_text(orig)
-        LIB.unlink(missing_ok=True)
+        shutil.rmtree(tmp, ignore_errors=True)
     if a.out:
         Path(a.out).write_text("\n".join(lines) + "\n")
     return 0 if all(l.startswith("RED") for l in lines) else 1
