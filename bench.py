@@ -193,6 +193,8 @@ def parse():
     ap.add_argument("--table-size", type=int, default=0,
                     help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
     ap.add_argument("--json-out", default=None)
+    ap.add_argument("--no-extras", action="store_true",
+                    help="skip the short runs of the other configs / modes added to the JSON line")
     ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
     ap.add_argument("--particles", type=int, default=0, help="experiment: override the particle count")
     return ap.parse_args()
@@ -238,6 +240,52 @@ def run_reference(a):
           "cpu_baseline": cpu,
           "e2e": {"value": v, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}},
          a.json_out)
+
+
+# Short runs of the other BASELINE.json workloads and variants, reported next to the headline
+# in the same JSON line (extra keys; the headline value stays csp / history mode).
+EXTRAS = [
+    ("stream", "history", {}), ("scatter", "history", {}), ("split", "history", {}),
+    ("csp", "event", {}), ("stream", "event", {}), ("scatter", "event", {}), ("split", "event", {}),
+    ("csp", "history", {"density_format": 1}),
+]
+
+
+def measure_extra(binding, torch, cfgname, mode, opts, local, steps=3, warmup=2):
+    cfg = wl.CONFIGS[cfgname]
+    stream = torch.cuda.current_stream()
+    tr = binding.Tracker(device=local, stream=stream.cuda_stream, mode=mode, A=cfg.A,
+                         molar_mass=cfg.molar_mass, e_min=cfg.e_min, w_min=cfg.w_min, **opts)
+    tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, wl.density(cfg))
+    tr.load_cross_sections(*wl.tables(cfg))
+
+    def step():
+        tr.inject_particles(cfg.n_particles, 0, cfg.n_particles, cfg.source, cfg.e0, cfg.seed)
+        return tr.run_timestep(cfg.dt)
+
+    for _ in range(warmup):
+        step()
+    torch.cuda.synchronize()
+    e0 = torch.cuda.Event(enable_timing=True)
+    e1 = torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    stats = [step() for _ in range(steps)]
+    e1.record(stream)
+    torch.cuda.synchronize()
+    tr.close()
+    ms = e0.elapsed_time(e1) / steps
+    events = statistics.mean(s["events"] for s in stats)
+    track_ms = statistics.mean(s["track_ms"] for s in stats)
+    ab = statistics.mean(algorithmic_bytes(s) for s in stats)
+    reds = statistics.mean(s["n_facets"] + s["n_census"] + s["n_killed"] for s in stats)
+    red_peak = l2_red_peak()
+    return {"workload": cfgname, "mode": mode, "opts": opts, "value": events / (ms / 1e3), "unit": UNIT,
+            "ms_per_step": ms, "steps": steps, "warmup": warmup, "events_per_step": events,
+            "kernel_ms": track_ms,
+            "hbm_roofline_frac": ab / (track_ms / 1e3) / 1e9 / measured_peaks()["hbm_gbs"],
+            "l2_red_frac": None if red_peak is None else reds / (track_ms / 1e3) / red_peak,
+            "grind_ns_per_event": track_ms * 1e6 / max(1.0, events),
+            "status": sorted({s["status"] for s in stats})}
 
 
 def main():
@@ -356,9 +404,22 @@ def main():
                        "run_timestep + read_tally"}
     tr.close()
 
+    extras = None
+    if rank == 0 and world == 1 and not a.no_extras and a.config == "csp" and a.mode == "history":
+        extras = {}
+        for c, m, o in EXTRAS:
+            key = f"{c}/{m}" + "".join(f"/{k}={v}" for k, v in o.items())
+            try:
+                extras[key] = measure_extra(binding, torch, c, m, o, local)
+            except Exception as ex:          # reported, never fatal for the headline
+                extras[key] = {"error": str(ex)[:200]}
+
     cpu = None
     if rank == 0 and world == 1 and not a.no_cpu_baseline:
         cpu = oracle_host_rate(cfg)
+        one = oracle_host_rate(cfg, budget_s=8.0, max_procs=1)
+        cpu["one_core"] = {"value": one["value"], "cores": 1, "sample": one["sample"]}
+        cpu["gpu_over_oracle"] = {"all_cores": value / cpu["value"], "one_core": value / one["value"]}
 
     if rank == 0:
         s0 = stats[-1]
@@ -386,7 +447,13 @@ def main():
             "grind_ns": {"per_event": track_ms * 1e6 * world / max(1.0, events / a.steps),
                          "per_facet_if_all_facets": track_ms * 1e6 * world / max(1, s0["n_facets"]),
                          "per_collision_if_all_collisions": track_ms * 1e6 * world / max(1, s0["n_collisions"])},
-            "roofline": {"bound": "hbm", "kernel": f"history_kernel<false>" if a.mode == "history" else "event kernels",
+            "roofline": {"bound": "hbm", "basis": "algorithmic bytes of the paper's fp64 format (SURVEY §8(d): "
+                         "24 B/facet, 16 B/census or kill flush, 138 B/particle) / tracking-kernel time; the "
+                         "kernel reads u8 codes and its tally REDs stay in L2, so this is an algorithmic-byte "
+                         "rate, not DRAM utilisation (that is traffic / kernel time, dram_frac); the binding "
+                         "ceiling is l2_red_roofline",
+                         "dram_frac": None if not traffic else traffic / (track_ms / 1e3) / 1e9 / peaks["hbm_gbs"],
+                         "kernel": f"history_kernel<false>" if a.mode == "history" else "ev_loop_kernel",
                          "achieved": achieved, "peak": peaks["hbm_gbs"], "unit": "GB/s",
                          "frac": achieved / peaks["hbm_gbs"], "traffic": traffic,
                          "algorithmic_bytes_per_launch": ab, "kernel_ms": track_ms,
@@ -397,6 +464,7 @@ def main():
                 "frac": red_rate / red_peak, "reds_per_launch": reds,
                 "peak_source": "measured: scripts/dev/red_microbench.cu (profiles/r01_v16_red_microbench.json)"},
             "cpu_baseline": cpu,
+            "extra_configs": extras,
             "e2e": e2e,
             "gpu_launches": launches,
             "clocks": clk.summary(),

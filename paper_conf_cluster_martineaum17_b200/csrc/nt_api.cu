@@ -87,6 +87,7 @@ struct nt_ctx {
   int64_t cells_st = 0;                  // cells in the storage layout (tiles padded)
   // tables
   DevBuf xs;
+  size_t xs_bytes = 0;                   // bytes of xs in use (keys, values, indexes, pairs)
   Tables tables{};
   // particles
   int64_t n_total = 0, first_id = 0, n_local = 0;
@@ -494,9 +495,11 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     std::memcpy(&b0, &k[0], 8);
     std::memcpy(&b1, &k[n - 1], 8);
     const uint64_t range = b1 - b0;
-    int64_t target = n / 4;
-    if (target < 1) target = 1;
-    if (target > 16384) target = 16384;
+    // about four buckets per key (the bit patterns of log-spaced keys are linear within a
+    // binade, so the keys per bucket vary by 2x): a bucket then almost always spans at most
+    // one key and the lookup needs no search loop (xs_lookup)
+    int64_t target = 4 * n;
+    if (target > (1ll << 22)) target = 1ll << 22;
     int s = 0;
     while ((range >> s) >= (uint64_t)target) ++s;
     const int64_t nb = (int64_t)(range >> s) + 1;
@@ -519,7 +522,18 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     shift[t] = s;
     nbk[t] = (int32_t)nb;
   }
-  size_t off[6], total = 0;
+  // interleaved (key, value) pairs, one padding pair (a copy of the last) at the end
+  std::vector<double> kvh[2];
+  for (int t = 0; t < 2; ++t) {
+    const int64_t n = len[2 * t];
+    kvh[t].resize(2 * ((size_t)n + 1));
+    for (int64_t j = 0; j <= n; ++j) {
+      const int64_t q = j < n ? j : n - 1;
+      kvh[t][2 * (size_t)j] = h[2 * t][q];
+      kvh[t][2 * (size_t)j + 1] = h[2 * t + 1][q];
+    }
+  }
+  size_t off[8], total = 0;
   for (int k = 0; k < 4; ++k) {
     off[k] = total;
     total += align256((size_t)len[k] * 8);
@@ -528,20 +542,29 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     off[4 + t] = total;
     total += align256(idx[t].size() * 4 + 4);
   }
+  for (int t = 0; t < 2; ++t) {
+    off[6 + t] = total;
+    total += align256(kvh[t].size() * 8);
+  }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k], (size_t)len[k] * 8,
                                cudaMemcpyDefault, c->stream));
-  for (int t = 0; t < 2; ++t)
+  for (int t = 0; t < 2; ++t) {
     if (!idx[t].empty())
       NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[4 + t], idx[t].data(), idx[t].size() * 4,
                                  cudaMemcpyHostToDevice, c->stream));
+    NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[6 + t], kvh[t].data(), kvh[t].size() * 8,
+                               cudaMemcpyHostToDevice, c->stream));
+  }
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  c->xs_bytes = total;
   Table* T[2] = {&c->tables.s, &c->tables.c};
   for (int t = 0; t < 2; ++t) {
     T[t]->k = reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t]);
     T[t]->v = reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t + 1]);
     T[t]->idx = reinterpret_cast<const uint32_t*>(c->xs.as<char>() + off[4 + t]);
+    T[t]->kv = reinterpret_cast<const double2*>(c->xs.as<char>() + off[6 + t]);
     T[t]->n = (int32_t)len[2 * t];
     T[t]->nb = nbk[t];
     T[t]->shift = shift[t];
@@ -626,7 +649,6 @@ nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int6
   c->first_id = first_id;
   c->n_local = n_local;
   c->seed = seed;
-  if (c->evs) event_state_invalidate(c->evs);
   c->stage = ST_PARTICLES;
   return NT_OK;
 }

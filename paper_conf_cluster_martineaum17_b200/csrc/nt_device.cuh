@@ -88,6 +88,8 @@ __device__ __forceinline__ int64_t cell_index(const Mesh& M, int32_t cx, int32_t
 struct Table {
   const double* __restrict__ k;     // keys, eV, strictly increasing
   const double* __restrict__ v;     // values, barns
+  const double2* __restrict__ kv;   // (k[i], v[i]) interleaved, [n + 1] (last entry repeats
+                                    // n - 1): one 48 B run holds the two bins a bucket spans
   const uint32_t* __restrict__ idx; // [nb + 1]
   uint64_t base;
   int32_t n, nb, shift, pad;
@@ -315,30 +317,73 @@ __device__ __forceinline__ double dens_nd(typename DensRaw<kFmt>::type raw,
 }
 
 // ---- microscopic cross sections -----------------------------------------------
+// Table loads.  NT_XS_HINT=1 (A/B option) gives them an L2 evict_last policy, the priority
+// of the tally lines, so the 128 MB tally cannot push the (~5 MB) tables out of L2.
+#ifndef NT_XS_HINT
+#define NT_XS_HINT 0
+#endif
+__device__ __forceinline__ double2 xs_ld2(const double2* p) {
+#if NT_XS_HINT
+  double2 v;
+  asm volatile("{ .reg .b64 pol; createpolicy.fractional.L2::evict_last.b64 pol, 1.0;\n\t"
+               "ld.global.nc.L2::cache_hint.v2.f64 {%0, %1}, [%2], pol; }"
+               : "=d"(v.x), "=d"(v.y) : "l"(p));
+  return v;
+#else
+  return __ldg(p);
+#endif
+}
+__device__ __forceinline__ uint32_t xs_ldu(const uint32_t* p) {
+#if NT_XS_HINT
+  uint32_t v;
+  asm volatile("{ .reg .b64 pol; createpolicy.fractional.L2::evict_last.b64 pol, 1.0;\n\t"
+               "ld.global.nc.L2::cache_hint.u32 %0, [%1], pol; }" : "=r"(v) : "l"(p));
+  return v;
+#else
+  return __ldg(p);
+#endif
+}
+
 // Bin i = max{i in [0,N-2]: k[i] <= e} for e already in [k0, k_{N-1}] (the energy-bin
-// search), then linear interpolation.  The bucket index narrows the binary search to a
-// few keys; it returns the same bin as a full binary search by construction.
+// search), then linear interpolation.  The bucket index is fine enough (about four buckets
+// per key, nt_load_cross_sections) that a bucket nearly always spans at most one key: then
+// the bin is idx[b] or idx[b] + 1, decided by one compare against k[idx[b] + 1], and the
+// three (key, value) pairs that can be needed come from one 48 B run of the interleaved
+// table -- two dependent loads per lookup (the index pair, then the run).  A bucket holding
+// more keys falls back to a binary search inside it.  Same bin as a full binary search by
+// construction.
 __device__ __forceinline__ double xs_lookup(const Table& T, double e) {
-  const double* __restrict__ k = T.k;
-  const int32_t n = T.n;
   int32_t lo, hi;                             // k[lo] <= e < k[hi]
   if (e >= T.klast) {
-    lo = n - 2;
-    hi = n - 1;
+    lo = T.n - 2;
+    hi = T.n - 1;
   } else if (T.nb > 0) {
     const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
-    lo = (int32_t)__ldg(T.idx + b);
-    hi = (int32_t)__ldg(T.idx + b + 1) + 1;
+    lo = (int32_t)xs_ldu(T.idx + b);
+    hi = (int32_t)xs_ldu(T.idx + b + 1) + 1;
   } else {
     lo = 0;
-    hi = n - 1;
+    hi = T.n - 1;
   }
-  while (hi - lo > 1) {
-    const int32_t mid = (lo + hi) >> 1;
-    if (__ldg(k + mid) <= e) lo = mid; else hi = mid;
+  double k0, k1, v0, v1;
+  if (hi - lo <= 2) {
+    const double2 a = xs_ld2(T.kv + lo), b = xs_ld2(T.kv + lo + 1), c = xs_ld2(T.kv + lo + 2);
+    const bool up = hi - lo == 2 && b.x <= e;
+    k0 = up ? b.x : a.x;
+    v0 = up ? b.y : a.y;
+    k1 = up ? c.x : b.x;
+    v1 = up ? c.y : b.y;
+  } else {
+    while (hi - lo > 1) {
+      const int32_t mid = (lo + hi) >> 1;
+      if (__ldg(T.k + mid) <= e) lo = mid; else hi = mid;
+    }
+    const double2 a = __ldg(T.kv + lo), b = __ldg(T.kv + lo + 1);
+    k0 = a.x;
+    v0 = a.y;
+    k1 = b.x;
+    v1 = b.y;
   }
-  const double k0 = __ldg(k + lo), k1 = __ldg(k + lo + 1);
-  const double v0 = __ldg(T.v + lo), v1 = __ldg(T.v + lo + 1);
   const double t = (e - k0) / (k1 - k0);
   return v0 + t * (v1 - v0);
 }

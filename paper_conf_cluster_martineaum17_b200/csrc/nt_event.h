@@ -11,7 +11,6 @@ namespace nt {
 struct EventState;
 EventState* event_state_create();
 void event_state_destroy(EventState* s);
-void event_state_invalidate(EventState* s);
 // Track local particles [tp.lo, tp.hi) for one timestep with the event queues; adds the
 // range's statistics into tp.stats_*.  Deterministic mode (det) writes flush records.
 nt_status event_run_range(EventState* s, const TrackParams& tp, bool det, int sm_count,
