@@ -33,7 +33,7 @@
 extern "C" {
 #endif
 
-#define NT_ABI_VERSION 4
+#define NT_ABI_VERSION 5
 
 typedef struct nt_ctx nt_ctx;
 
@@ -254,6 +254,10 @@ nt_status nt_particle_slots(nt_ctx *ctx, int64_t *n_slots);
 /* Device allocations the library has made so far, process-wide (every cudaMalloc goes
  * through one counter).  A timestep on a context whose buffers exist allocates nothing. */
 int64_t nt_debug_alloc_count(void);
+/* Device bytes the context holds for the mesh: density (f64 and codes, block map) and the
+ * tally buffers.  With x-slabs (decomposition 1) only the rank's columns plus a one-column
+ * halo are stored, so this scales as 1/nranks.  -1 for a NULL context. */
+int64_t nt_debug_mesh_bytes(const nt_ctx *ctx);
 /* out[2i], out[2i+1] = threefry2x64_20(ctr = {in[4i], in[4i+1]}, key = {in[4i+2], in[4i+3]}). */
 nt_status nt_debug_threefry(nt_ctx *ctx, const uint64_t *in, int64_t n, uint64_t *out);
 /* Microscopic XS from the loaded tables: out_s[i], out_a[i] at energies[i] (no clamp

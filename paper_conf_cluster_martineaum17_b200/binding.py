@@ -31,7 +31,8 @@ EXPORTS = ["nt_abi_version", "nt_build_info", "nt_status_string", "nt_options_de
            "nt_load_cross_sections", "nt_inject_particles", "nt_run_timestep", "nt_read_tally",
            "nt_read_particles", "nt_write_particles", "nt_slab_record_bytes", "nt_slab_begin",
            "nt_slab_round", "nt_slab_export", "nt_slab_import", "nt_slab_end", "nt_particle_slots",
-           "nt_debug_threefry", "nt_debug_xs", "nt_debug_alloc_count"]
+           "nt_debug_threefry", "nt_debug_xs", "nt_debug_alloc_count",
+           "nt_debug_mesh_bytes"]
 
 
 class NeutralError(RuntimeError):
@@ -118,6 +119,7 @@ def lib():
             "nt_debug_threefry": ([vp, vp, i64, vp], C.c_int),
             "nt_debug_xs": ([vp, vp, i64, vp, vp], C.c_int),
             "nt_debug_alloc_count": ([], i64),
+            "nt_debug_mesh_bytes": ([vp], i64),
         }
         for name, (args, res) in sigs.items():
             f = getattr(L, name)
@@ -339,6 +341,10 @@ class Tracker:
         keep = {n: np.ascontiguousarray(fields[n], dtype=t) for n, t in PARTICLE_FIELDS if n in fields}
         v = ParticlesView(*[keep[n].ctypes.data if n in keep else None for n, _ in PARTICLE_FIELDS])
         self._check(lib().nt_write_particles(self._h, first, count, C.byref(v)), "nt_write_particles")
+
+    def mesh_bytes(self) -> int:
+        """Device bytes held for the mesh (density + tally buffers)."""
+        return int(lib().nt_debug_mesh_bytes(self._h))
 
     def debug_threefry(self, inputs: np.ndarray) -> np.ndarray:
         inp = np.ascontiguousarray(inputs, dtype=np.uint64).reshape(-1, 4)

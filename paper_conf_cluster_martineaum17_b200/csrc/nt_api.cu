@@ -14,6 +14,8 @@
 #include <string>
 #include <vector>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "../../include/neutral_b200.h"
 #include "nt_event.h"
 #include "nt_internal.h"
@@ -49,6 +51,13 @@ struct DevBuf {
   template <class T> T* as() const { return static_cast<T*>(p); }
 };
 
+// NVTX range over a C-ABI call (nsys / ncu --nvtx show the library's phases by name; the
+// header-only NVTX v3 costs nothing without a tool attached).
+struct NvtxRange {
+  explicit NvtxRange(const char* name) { nvtxRangePushA(name); }
+  ~NvtxRange() { nvtxRangePop(); }
+};
+
 }  // namespace
 
 namespace nt {
@@ -76,12 +85,14 @@ struct nt_ctx {
   double* stats_h = nullptr;
   // mesh
   int32_t nx = 0, ny = 0;
+  int32_t x0 = 0, nxs = 0;               // stored columns [x0, x0 + nxs) (x-slabs: own + halo)
   double W = 0, H = 0;
   DevBuf rho, tally, tally_red, ex, ey;  // tally_red: the cross-rank sum (comm only)
   DevBuf rho_code, nd_tab, enc_keys;     // lossless density encoding
   DevBuf blk;                            // block map of the u8 codes (Mesh::blk)
   int blk_shift = 0, blk_nbx = 0, blk_n = 0;   // blk_n = 0: no block map
   DevBuf rho_st, tally_rm;               // f64 density in storage layout; row-major staging
+  DevBuf tally_full;                     // x-slabs: the whole-mesh tally assembled at read time
   int dens_fmt = kDensF64, dens_codes = 0;
   int tiled = 0, ntx = 0;                // storage layout of tally / density (cell_index)
   int64_t cells_st = 0;                  // cells in the storage layout (tiles padded)
@@ -319,7 +330,7 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
-  for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
+  for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->tally_full, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup, &c->stats_d})
     b->release();
@@ -339,6 +350,7 @@ nt_status nt_destroy(nt_ctx* c) {
 // 8 B and the map stays L2-resident.
 nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double height,
                        const double* density) {
+  NvtxRange nvtx_("nt_init_mesh");
   if (!c) return NT_ERR_ARG;
   cudaSetDevice(c->device);
   if (nx < 1 || ny < 1) return fail(c, NT_ERR_ARG, "nx, ny must be >= 1 (got %d, %d)", nx, ny);
@@ -347,26 +359,42 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   if (!(width > 0.0) || !(height > 0.0) || !is_fin(width) || !is_fin(height))
     return fail(c, NT_ERR_ARG, "width, height must be finite and > 0");
   if (!density) return fail(c, NT_ERR_ARG, "density is NULL");
-  const int64_t cells = (int64_t)nx * (int64_t)ny;
+  // x-slabs (decomposition 1): this rank stores only its columns [floor(r nx/P),
+  // floor((r+1) nx/P)) plus a one-column halo on each side (the density of the cell a
+  // particle steps into before it is handed over), so mesh memory scales as 1/P
+  int32_t x0 = 0, nxs = nx;
+  if (c->opt.decomposition == 1) {
+    const int64_t P = c->opt.nranks, r = c->opt.rank;
+    const int32_t lo = (int32_t)((r * nx) / P), hi = (int32_t)(((r + 1) * nx) / P);
+    x0 = lo > 0 ? lo - 1 : 0;
+    nxs = (hi < nx ? hi + 1 : nx) - x0;
+  }
+  const int64_t cells = (int64_t)nxs * (int64_t)ny;   // stored cells
   c->stage = ST_CREATED;
   const int tiled = c->opt.layout == 0 ? 1 : 0;
-  const int ntx = (nx + 3) / 4, nty = (ny + 3) / 4;
+  const int ntx = (nxs + 3) / 4, nty = (ny + 3) / 4;
   const int64_t cells_st = tiled ? (int64_t)ntx * nty * 16 : cells;
   if (cells_st >= (1ll << 32))
     return fail(c, NT_ERR_ARG, "the tiled mesh storage must hold < 2^32 cells");
-  Mesh ml{};
-  ml.nx = nx;
+  Mesh ml{};                              // the stored sub-mesh, in its own columns
+  ml.nx = nxs;
+  ml.gnx = nxs;
   ml.ny = ny;
   ml.tiled = tiled;
   ml.ntx = ntx;
   ml.strip = 16 * ntx;
   NT_CUDA(c, c->rho.ensure((size_t)cells * 8));
   NT_CUDA(c, c->tally.ensure((size_t)cells_st * 8));
-  if (c->comm) NT_CUDA(c, c->tally_red.ensure((size_t)cells_st * 8));
+  const bool reduce_in_step = c->comm && c->opt.decomposition != 1;
+  if (reduce_in_step) NT_CUDA(c, c->tally_red.ensure((size_t)cells_st * 8));
   NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
   NT_CUDA(c, c->ey.ensure(((size_t)ny + 1) * 8));
   NT_CUDA(c, c->scratch.ensure(1024));
-  NT_CUDA(c, cudaMemcpyAsync(c->rho.p, density, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
+  if (nxs == nx)
+    NT_CUDA(c, cudaMemcpyAsync(c->rho.p, density, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
+  else
+    NT_CUDA(c, cudaMemcpy2DAsync(c->rho.p, (size_t)nxs * 8, density + x0, (size_t)nx * 8,
+                                 (size_t)nxs * 8, (size_t)ny, cudaMemcpyDefault, c->stream));
   unsigned long long* bad = c->scratch.as<unsigned long long>();
   NT_CUDA(c, cudaMemsetAsync(bad, 0, 16, c->stream));
   NT_CUDA(c, launch_density_check(c->rho.as<double>(), cells, bad, c->stream));
@@ -405,7 +433,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   int blk_shift = 0, blk_nbx = 0, blk_n = 0;
   if (fmt == kDensU8 && nu < (int)kBlkMixed && c->opt.density_format == 0) {
     for (int s = 2; s < 31; ++s) {
-      const int64_t bx = ((int64_t)nx + (1 << s) - 1) >> s, by = ((int64_t)ny + (1 << s) - 1) >> s;
+      const int64_t bx = ((int64_t)nxs + (1 << s) - 1) >> s, by = ((int64_t)ny + (1 << s) - 1) >> s;
       if (bx * by <= kBlkMax) {
         blk_shift = s;
         blk_nbx = (int)bx;
@@ -426,7 +454,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
     NT_CUDA(c, launch_relayout(c->rho.as<double>(), c->rho_st.as<double>(), cells, ml, true, c->stream));
   }
   NT_CUDA(c, cudaMemsetAsync(c->tally.p, 0, (size_t)cells_st * 8, c->stream));
-  if (c->comm) NT_CUDA(c, cudaMemsetAsync(c->tally_red.p, 0, (size_t)cells_st * 8, c->stream));
+  if (reduce_in_step) NT_CUDA(c, cudaMemsetAsync(c->tally_red.p, 0, (size_t)cells_st * 8, c->stream));
   launch_edges(c->ex.as<double>(), nx, width, c->ey.as<double>(), ny, height, c->stream);
   NT_CUDA(c, cudaGetLastError());
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
@@ -440,6 +468,8 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   c->cells_st = cells_st;
   c->nx = nx;
   c->ny = ny;
+  c->x0 = x0;
+  c->nxs = nxs;
   c->W = width;
   c->H = height;
   c->stage = ST_MESH;
@@ -449,6 +479,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
 // ---- cross sections ---------------------------------------------------------
 nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, int64_t ns,
                                  const double* ck, const double* cv, int64_t nc) {
+  NvtxRange nvtx_("nt_load_cross_sections");
   if (!c) return NT_ERR_ARG;
   cudaSetDevice(c->device);
   if (c->stage < ST_MESH) return fail(c, NT_ERR_STATE, "nt_init_mesh must come first");
@@ -603,6 +634,7 @@ static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
 nt_status nt_inject_particles(nt_ctx* c, int64_t n_total, int64_t first_id, int64_t n_local,
                               double sx, double sy, double sw, double sh, double e0,
                               uint64_t seed) {
+  NvtxRange nvtx_("nt_inject_particles");
   if (!c) return NT_ERR_ARG;
   cudaSetDevice(c->device);
   if (c->stage < ST_XS) return fail(c, NT_ERR_STATE, "mesh and cross sections must be loaded first");
@@ -672,7 +704,11 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.mesh.tally = c->tally.as<double>();
   tp.mesh.ex = c->ex.as<double>();
   tp.mesh.ey = c->ey.as<double>();
-  tp.mesh.nx = c->nx;
+  tp.mesh.nx = c->nxs;
+  tp.mesh.gnx = c->nx;
+  tp.mesh.x0 = c->x0;
+  tp.mesh.wx = c->W;
+  tp.mesh.wy = c->H;
   tp.mesh.ny = c->ny;
   tp.xs = c->tables;
   if (c->opt.xs_search == 1) {          // plain binary search over the whole table
@@ -737,10 +773,14 @@ static nt_status det_snapshot(nt_ctx* c, int64_t lo, int64_t nb, bool restore) {
 // phase 2 resumes them.  (Measured alternative: 4 phases, even ones parking lonely facets
 // -- split 132 -> 130 ms but csp 31 -> 35 ms, each phase adding its own tail of long
 // streaming histories.)  With slabs, both phases hand emigrants to out_q.
+// (Measured and rejected in round 2: a third phase for the streamers phase 2 finds --
+// particles scattered back out of dense matter -- csp 27.1 -> 27.8-29.6 ms: too few of them
+// to fill the GPU, so the third launch is one long latency-bound tail; profiles/ab.)
 // scratch [0, 8): phase-1 counter, [16, 24): parking queue length, [32, 40): phase-2
 // counter, [40, 48): emigrant count, [64, 72): arrivals count.
 static nt_status track_phases(nt_ctx* c, const TrackParams& bp, bool det, uint32_t& launches,
                               const unsigned long long* src_count, bool slab) {
+  NvtxRange nvtx_("history phases");
   char* s = c->scratch.as<char>();
   unsigned long long* qlen = reinterpret_cast<unsigned long long*>(s + 16);
   NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 24, c->stream));
@@ -1038,6 +1078,7 @@ static nt_status step_prologue(nt_ctx* c, double dt) {
 }
 
 nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
+  NvtxRange nvtx_("nt_run_timestep");
   if (!c) return NT_ERR_ARG;
   cudaSetDevice(c->device);
   {
@@ -1068,9 +1109,12 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
     NT_CUDA(c, cudaGetLastError());
   }
   if (c->comm) {
+    NvtxRange nvtx_("tally + stats allreduce");
+    // (x-slabs own disjoint columns: their tallies are assembled at read time, nt_read_tally)
     NT_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
     NT_NCCL(c, ncclGroupStart());
-    NT_NCCL(c, ncclAllReduce(c->tally.p, c->tally_red.p, cells, ncclFloat64, ncclSum, c->comm, c->stream));
+    if (c->opt.decomposition != 1)
+      NT_NCCL(c, ncclAllReduce(c->tally.p, c->tally_red.p, cells, ncclFloat64, ncclSum, c->comm, c->stream));
     NT_NCCL(c, ncclAllReduce(sd, sd, SU_COUNT + SF_COUNT, ncclFloat64, ncclSum, c->comm, c->stream));
     NT_NCCL(c, ncclGroupEnd());
     NT_CUDA(c, cudaEventRecord(c->ev[4], c->stream));
@@ -1116,6 +1160,7 @@ nt_status nt_slab_begin(nt_ctx* c, double dt) {
 }
 
 nt_status nt_slab_round(nt_ctx* c, int64_t* n_emigrants) {
+  NvtxRange nvtx_("nt_slab_round");
   nt_status st = slab_check(c);
   if (st != NT_OK) return st;
   if (!n_emigrants) return fail(c, NT_ERR_ARG, "n_emigrants is NULL");
@@ -1125,6 +1170,7 @@ nt_status nt_slab_round(nt_ctx* c, int64_t* n_emigrants) {
 }
 
 nt_status nt_slab_export(nt_ctx* c, void* dst, int64_t capacity, int64_t* n_left, int64_t* n_right) {
+  NvtxRange nvtx_("nt_slab_export");
   nt_status st = slab_check(c);
   if (st != NT_OK) return st;
   if (!dst || !n_left || !n_right) return fail(c, NT_ERR_ARG, "NULL argument");
@@ -1142,6 +1188,7 @@ nt_status nt_slab_export(nt_ctx* c, void* dst, int64_t capacity, int64_t* n_left
 }
 
 nt_status nt_slab_import(nt_ctx* c, const void* src, int64_t n) {
+  NvtxRange nvtx_("nt_slab_import");
   nt_status st = slab_check(c);
   if (st != NT_OK) return st;
   if (n < 0 || (n > 0 && !src)) return fail(c, NT_ERR_ARG, "bad import");
@@ -1181,17 +1228,20 @@ nt_status nt_particle_slots(nt_ctx* c, int64_t* n_slots) {
 
 // ---- read-back ---------------------------------------------------------------------------
 nt_status nt_read_tally(nt_ctx* c, double* dst, int32_t reduced) {
+  NvtxRange nvtx_("nt_read_tally");
   if (!c) return NT_ERR_ARG;
   cudaSetDevice(c->device);
   if (c->stage < ST_MESH) return fail(c, NT_ERR_STATE, "no mesh");
   if (!dst) return fail(c, NT_ERR_ARG, "dst is NULL");
-  const int64_t cells = (int64_t)c->nx * (int64_t)c->ny;
-  const double* src = (reduced && c->comm) ? c->tally_red.as<double>() : c->tally.as<double>();
+  const bool slab = c->opt.decomposition == 1;
+  const int64_t cells = (int64_t)c->nxs * (int64_t)c->ny;         // stored cells
+  const double* src = (reduced && c->comm && !slab) ? c->tally_red.as<double>() : c->tally.as<double>();
   if (!src) return fail(c, NT_ERR_STATE, "no tally yet");
-  if (c->tiled) {            // storage layout -> row-major [ny][nx]
+  if (c->tiled) {            // storage layout -> row-major [ny][nxs]
     NT_CUDA(c, c->tally_rm.ensure((size_t)cells * 8));
     Mesh ml{};
-    ml.nx = c->nx;
+    ml.nx = c->nxs;
+    ml.gnx = c->nxs;
     ml.ny = c->ny;
     ml.tiled = 1;
     ml.ntx = c->ntx;
@@ -1199,7 +1249,21 @@ nt_status nt_read_tally(nt_ctx* c, double* dst, int32_t reduced) {
     NT_CUDA(c, launch_relayout(src, c->tally_rm.as<double>(), cells, ml, false, c->stream));
     src = c->tally_rm.as<double>();
   }
-  NT_CUDA(c, cudaMemcpyAsync(dst, src, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
+  if (slab) {
+    // the stored columns into a whole-mesh map (zero elsewhere); reduced with a
+    // communicator: the sum over the ranks' disjoint slabs
+    const int64_t all = (int64_t)c->nx * (int64_t)c->ny;
+    NT_CUDA(c, c->tally_full.ensure((size_t)all * 8));
+    double* full = c->tally_full.as<double>();
+    NT_CUDA(c, cudaMemsetAsync(full, 0, (size_t)all * 8, c->stream));
+    NT_CUDA(c, cudaMemcpy2DAsync(full + c->x0, (size_t)c->nx * 8, src, (size_t)c->nxs * 8,
+                                 (size_t)c->nxs * 8, (size_t)c->ny, cudaMemcpyDeviceToDevice, c->stream));
+    if (reduced && c->comm)
+      NT_NCCL(c, ncclAllReduce(full, full, (size_t)all, ncclFloat64, ncclSum, c->comm, c->stream));
+    NT_CUDA(c, cudaMemcpyAsync(dst, full, (size_t)all * 8, cudaMemcpyDefault, c->stream));
+  } else {
+    NT_CUDA(c, cudaMemcpyAsync(dst, src, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
+  }
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   return NT_OK;
 }
@@ -1240,6 +1304,14 @@ nt_status nt_write_particles(nt_ctx* c, int64_t first, int64_t count, const nt_p
 
 // ---- verification entry points -----------------------------------------------------------
 int64_t nt_debug_alloc_count(void) { return (int64_t)nt::g_device_allocs.load(); }
+
+int64_t nt_debug_mesh_bytes(const nt_ctx* c) {
+  if (!c) return -1;
+  int64_t b = 0;
+  for (const DevBuf* d : {&c->rho, &c->tally, &c->tally_red, &c->rho_code, &c->blk, &c->rho_st})
+    b += (int64_t)d->bytes;
+  return b;
+}
 
 nt_status nt_debug_threefry(nt_ctx* c, const uint64_t* in, int64_t n, uint64_t* out) {
   if (!c || !in || !out || n < 0) return NT_ERR_ARG;

@@ -52,9 +52,14 @@ struct Mesh {
   const uint16_t* __restrict__ rho16; // [ny][nx] material code     (kDensU16)
   const double* __restrict__ nd_tab;  // [codes] rho_k * cn, atoms/m^3
   double* __restrict__ tally;         // [ny][nx] eV*weight
-  const double* __restrict__ ex;      // [nx+1] edge(i) = (i*W)/nx
+  const double* __restrict__ ex;      // [gnx+1] edge(i) = (i*W)/gnx
   const double* __restrict__ ey;      // [ny+1]
-  int32_t nx, ny;
+  int32_t nx, ny;                     // cells in storage (the columns this rank holds x rows)
+  int32_t gnx;                        // cells per row of the whole mesh (reflection bound)
+  int32_t x0;                         // whole-mesh column of storage column 0 (x-slabs: the
+                                      // rank's first column minus a one-column halo; else 0)
+  double wx, wy;                      // mesh extents W, H: edge(i) = (i*W)/gnx in place of a
+                                      // load (bit-identical to ex[i], DESIGN.md §3 MESH)
   int32_t fmt, ncodes;
   int32_t tiled;                      // 1: 4x4-cell tiles (one 128 B tally line per tile)
   int32_t ntx;                        // tiles per row = ceil(nx / 4)
@@ -75,10 +80,14 @@ constexpr int kBlkMax = 16384;         // max block-map entries (bytes of shared
 // (cy/4)*(16*ntx) + 4*cx + cy%4 -- so the 16 f64 tally cells of a tile fill one 128 B line
 // and a particle's consecutive facets (x or y) mostly stay in it; the index costs one shift
 // and two integer multiply-adds.
+// kOff (x-slab storage): cx is a whole-mesh column, the storage column is cx - x0; without
+// it cx is the storage column (x0 = 0: replicated meshes and mesh preparation).
+template <bool kOff = false>
 __device__ __forceinline__ int64_t cell_index(const Mesh& M, int32_t cx, int32_t cy) {
+  const int64_t lx = kOff ? (int64_t)(cx - M.x0) : (int64_t)cx;
   if (M.tiled)
-    return (int64_t)(cy >> 2) * (16 * (int64_t)M.ntx) + ((int64_t)cx << 2) + (int64_t)(cy & 3);
-  return (int64_t)cy * M.nx + cx;
+    return (int64_t)(cy >> 2) * (16 * (int64_t)M.ntx) + (lx << 2) + (int64_t)(cy & 3);
+  return (int64_t)cy * M.nx + lx;
 }
 
 // One microscopic cross-section table with its bucket index: bucket b covers the IEEE bit
@@ -289,10 +298,12 @@ __device__ __forceinline__ typename DensRaw<kFmt>::type dens_load(const Mesh& M,
 
 // u8 code of cell (cx, cy) via the shared-memory block map: the block's code when the block
 // is uniform, else the cell's own code from the global map (storage index cidx).
+template <bool kOff = false>
 __device__ __forceinline__ uint32_t dens_load_blk(const Mesh& M, const uint8_t* s_blk,
                                                   int32_t cx, int32_t cy, uint32_t cidx,
                                                   uint64_t pol) {
-  uint32_t code = s_blk[(cy >> M.bshift) * M.nbx + (cx >> M.bshift)];
+  const int32_t lx = kOff ? cx - M.x0 : cx;
+  uint32_t code = s_blk[(cy >> M.bshift) * M.nbx + (lx >> M.bshift)];
   if (code == kBlkMixed) code = ldg_u8_hint(M.rho8 + cidx, pol);
   return code;
 }

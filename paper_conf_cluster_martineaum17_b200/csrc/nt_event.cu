@@ -42,19 +42,23 @@ constexpr int kEvBlock = kEvWarps * 32;
 constexpr int kWSlots = 64;                  // slots per warp: two per lane
 constexpr int kSlots = kEvWarps * kWSlots;   // slots per CTA
 constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many slots are free
+#ifndef NT_EV_EDGE_DIV
+#define NT_EV_EDGE_DIV 0
+#endif
 
-// event types (low 3 bits of a slot's type byte); bit 3: the facet crosses an X edge
-enum : uint32_t { T_COLL = 0, T_FACET = 1, T_CENSUS = 2, T_BIRTH = 3, T_FREE = 4, T_AXBIT = 8 };
+// Type byte of a slot: bits 0-2 the next event (or free / birth), bit 3 the facet crosses
+// an X edge, bit 4 the slot's deposit accumulator is non-zero (it is zero after every
+// flush, so most events neither load nor store it).
+enum : uint32_t { T_COLL = 0, T_FACET = 1, T_CENSUS = 2, T_BIRTH = 3, T_FREE = 4, T_AXBIT = 8,
+                  T_ACCBIT = 16 };
 
-// f64 slot columns
+// 8-byte slot columns (three of them pack two i32 fields) and one 4-byte column
 enum Col8 : int {
   C_X = 0, C_Y, C_OX, C_OY, C_IOX, C_IOY, C_EXN, C_EYN, C_MFP, C_DCEN, C_ACC, C_DSTEP,
-  C_W, C_E, C_ST, C_H, C_PA, C_ND, C_D, kCol8
+  C_W, C_E, C_ST, C_H, C_PA, C_ND, C_D, C_CXY, C_NFC, C_CTRSEQ, kCol8
 };
-// i32 slot columns
-enum Col4 : int { C_CX = 0, C_CY, C_NF, C_NC, C_CTR, C_SEQ, C_PID, kCol4 };
 
-constexpr size_t kSmemCols = (size_t)kSlots * (kCol8 * 8 + kCol4 * 4);
+constexpr size_t kSmemCols = (size_t)kSlots * (kCol8 * 8 + 4);
 constexpr size_t ev_smem_bytes(bool blk) {
   return kSmemCols + 2 * (size_t)kSlots /* types, per-warp queues */ + (blk ? (size_t)kBlkMax : 0);
 }
@@ -78,6 +82,13 @@ struct EvParams {
 
 __device__ __forceinline__ double ev_inf() { return __longlong_as_double(0x7ff0000000000000ll); }
 
+// A particle's state in registers while one of its events is handled.
+struct St {
+  double x, y, ox, oy, iox, ioy, exn, eyn, mfp, dcen, acc, dstep, w, e, st, H, nd;
+  int32_t cx, cy;
+  uint32_t nf, nc, ctr;
+};
+
 template <bool kDet, int kFmt, bool kBlk>
 struct EvKernel {
   const TrackParams& P;
@@ -89,15 +100,33 @@ struct EvKernel {
   int64_t sstride;
   uint64_t pol;             // L2 evict_last: tally REDs and density gathers
   double* c8;               // [kCol8][kSlots]
-  int32_t* c4;              // [kCol4][kSlots]
+  int32_t* cpid;            // [kSlots] local particle index
 
   __device__ double& d(int f, int s) { return c8[f * kSlots + s]; }
-  __device__ int32_t& i(int f, int s) { return c4[f * kSlots + s]; }
+  __device__ int2& i2(int f, int s) { return reinterpret_cast<int2*>(c8 + f * kSlots)[s]; }
 
   __device__ void cnt(int k, uint32_t v) { atomicAdd(s_u + k, (unsigned long long)v); }
   __device__ void fsum(int k, double v) { sf[k * sstride] += v; }
 
   __device__ uint32_t cidx(int32_t cx, int32_t cy) { return (uint32_t)cell_index(P.mesh, cx, cy); }
+
+  // Mesh edges (DESIGN.md §3 MESH): edge(i) = (i*W)/n.  NT_EV_EDGE_DIV evaluates the
+  // expression in place -- the same IEEE operations as the edge tables, so bit-identical --
+  // instead of a dependent global load on every facet (16 warps per SM hide little latency).
+  __device__ double edge_x(int32_t k) {
+#if NT_EV_EDGE_DIV
+    return ((double)k * P.mesh.wx) / (double)P.mesh.gnx;
+#else
+    return __ldg(P.mesh.ex + k);
+#endif
+  }
+  __device__ double edge_y(int32_t k) {
+#if NT_EV_EDGE_DIV
+    return ((double)k * P.mesh.wy) / (double)P.mesh.ny;
+#else
+    return __ldg(P.mesh.ey + k);
+#endif
+  }
 
   // number density of cell (cx, cy)
   __device__ double nd_of(int32_t cx, int32_t cy) {
@@ -108,275 +137,317 @@ struct EvKernel {
   }
 
   // the flush of DESIGN.md §3: production RED or deterministic record
-  __device__ void flush(int s, int32_t cx, int32_t cy, double& acc, double& dstep) {
-    const uint32_t cell = cidx(cx, cy);
+  __device__ void flush(int s, St& v) {
+    const uint32_t cell = cidx(v.cx, v.cy);
     if constexpr (kDet) {
-      const int32_t pi = i(C_PID, s);
-      const uint32_t seq = (uint32_t)i(C_SEQ, s);
+      const int32_t pi = cpid[s];
+      int2 cs = i2(C_CTRSEQ, s);
+      const uint32_t seq = (uint32_t)cs.y;
       const unsigned long long rs = atomicAdd(P.rec_count, 1ull);
       if (rs < P.rec_cap) {
         P.rec_key[rs] = ((unsigned long long)cell << 40) |
                         ((unsigned long long)((int64_t)pi - P.lo) << 24) |
                         (unsigned long long)(seq & 0xffffffu);
-        P.rec_val[rs] = acc;
+        P.rec_val[rs] = v.acc;
       }
       if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
-      i(C_SEQ, s) = (int32_t)(seq + 1u);
+      cs.y = (int)(seq + 1u);
+      i2(C_CTRSEQ, s) = cs;
     } else {
-      red_add_hint(P.mesh.tally + cell, acc, pol);
+      red_add_hint(P.mesh.tally + cell, v.acc, pol);
     }
-    dstep += acc;
-    acc = 0.0;
+    v.dstep += v.acc;
+    v.acc = 0.0;
   }
 
   // A history ended in slot s: write the particle store (census: alive; otherwise dead).
-  __device__ uint32_t finish(int s, double x, double y, double ox, double oy, double e, double w,
-                             double mfp, double dstep, int32_t cx, int32_t cy, uint32_t ctr,
-                             uint32_t nf, uint32_t nc, bool alive) {
-    const int32_t pi = i(C_PID, s);
-    if (!(isfinite(x) && isfinite(y) && isfinite(e) && isfinite(w))) cnt(SU_NONFINITE, 1u);
-    P.p.x[pi] = x;
-    P.p.y[pi] = y;
-    P.p.ox[pi] = ox;
-    P.p.oy[pi] = oy;
-    P.p.e[pi] = e;
-    P.p.w[pi] = w;
-    P.p.mfp[pi] = mfp;
-    P.p.dep[pi] += dstep;
-    P.p.cx[pi] = cx;
-    P.p.cy[pi] = cy;
-    P.p.ctr[pi] = ctr;
-    P.p.nfac[pi] += nf;
-    P.p.ncol[pi] += nc;
+  __device__ uint32_t finish(int s, const St& v, bool alive) {
+    const int32_t pi = cpid[s];
+    if (!(isfinite(v.x) && isfinite(v.y) && isfinite(v.e) && isfinite(v.w))) cnt(SU_NONFINITE, 1u);
+    P.p.x[pi] = v.x;
+    P.p.y[pi] = v.y;
+    P.p.ox[pi] = v.ox;
+    P.p.oy[pi] = v.oy;
+    P.p.e[pi] = v.e;
+    P.p.w[pi] = v.w;
+    P.p.mfp[pi] = v.mfp;
+    P.p.dep[pi] += v.dstep;
+    P.p.cx[pi] = v.cx;
+    P.p.cy[pi] = v.cy;
+    P.p.ctr[pi] = v.ctr;
+    P.p.nfac[pi] += v.nf;
+    P.p.ncol[pi] += v.nc;
     if (alive) P.p.ncen[pi] += 1u; else P.p.status[pi] = 0u;
-    cnt(SU_FACETS, nf);
-    cnt(SU_COLLISIONS, nc);
-    fsum(SF_TALLY, dstep);
+    cnt(SU_FACETS, v.nf);
+    cnt(SU_COLLISIONS, v.nc);
+    fsum(SF_TALLY, v.dstep);
     return T_FREE;
   }
 
-  // calculate_time_to_events + determine_next_event (Listing 2) for the
-  // state in slot s (whose x, y, exn, eyn, iox, ioy, mfp, dcen, st, nd are stored): the
-  // next event's type and distance go to the slot.  The event cap (R27) ends the
-  // history here.  Same expressions as the history kernel (R28 clamps).
-  __device__ uint32_t classify(int s, uint32_t nf, uint32_t nc) {
-    if ((int64_t)(nf + nc) >= P.max_events) {
-      double acc = d(C_ACC, s), dstep = d(C_DSTEP, s);
-      const int32_t cx = i(C_CX, s), cy = i(C_CY, s);
-      const double w = d(C_W, s), e = d(C_E, s);
-      cnt(SU_EVENT_CAP, 1u);
-      flush(s, cx, cy, acc, dstep);
-      cnt(SU_KILLED, 1u);
-      fsum(SF_KILLED_E, w * e);
-      fsum(SF_KILLED_W, w);
-      return finish(s, d(C_X, s), d(C_Y, s), d(C_OX, s), d(C_OY, s), e, w, d(C_MFP, s), dstep, cx,
-                    cy, (uint32_t)i(C_CTR, s), nf, nc, false);
-    }
-    const double sig = d(C_ND, s) * d(C_ST, s);
-    const double tx = (d(C_EXN, s) - d(C_X, s)) * d(C_IOX, s);
-    const double ty = (d(C_EYN, s) - d(C_Y, s)) * d(C_IOY, s);
+  // The event cap (R27): flush, count, kill.  v.e must be loaded.
+  __device__ uint32_t cap_kill(int s, St& v) {
+    cnt(SU_EVENT_CAP, 1u);
+    flush(s, v);
+    cnt(SU_KILLED, 1u);
+    fsum(SF_KILLED_E, v.w * v.e);
+    fsum(SF_KILLED_W, v.w);
+    return finish(s, v, false);
+  }
+
+  // calculate_time_to_events + determine_next_event (Listing 2) from the
+  // state in registers: the distance goes to the slot, the type bits are returned.  Same
+  // expressions as the history kernel (R28 clamps).
+  __device__ uint32_t classify(int s, const St& v) {
+    const double sig = v.nd * v.st;
+    const double tx = (v.exn - v.x) * v.iox;
+    const double ty = (v.eyn - v.y) * v.ioy;
     const bool ax = ty > 0.0 && tx < ty;
     double df = ax ? tx : ty;
     df = df < 0.0 ? 0.0 : df;
-    const double ds = d(C_DCEN, s);
-    const double mfp = d(C_MFP, s);
+    const double ds = v.dcen;
+    const uint32_t accb = v.acc != 0.0 ? T_ACCBIT : 0u;
     // n_mfp / Sigma_t only when a collision is possible (the history kernel's screen)
     const double dmin = df < ds ? df : ds;
     const double dsig = dmin * sig;
-    const bool maybe_coll = !(mfp > dsig * 0x1.00001p+0) || dsig < 0x1p-960;
+    const bool maybe_coll = !(v.mfp > dsig * 0x1.00001p+0) || dsig < 0x1p-960;
     if (maybe_coll && sig > 0.0) {
-      const double dc = mfp / sig;
+      const double dc = v.mfp / sig;
       if (dc < df && dc < ds) {
         d(C_D, s) = dc;
-        return T_COLL;
+        return T_COLL | accb;
       }
     }
     if (df < ds) {
       d(C_D, s) = df;
-      return T_FACET | (ax ? T_AXBIT : 0u);
+      return T_FACET | (ax ? T_AXBIT : 0u) | accb;
     }
     d(C_D, s) = ds;
-    return T_CENSUS;
+    return T_CENSUS | accb;
+  }
+
+  __device__ void load_nfc(int s, St& v) {
+    const int2 a = i2(C_CXY, s), b = i2(C_NFC, s);
+    v.cx = a.x; v.cy = a.y; v.nf = (uint32_t)b.x; v.nc = (uint32_t)b.y;
   }
 
   // ---- collision ----
-  __device__ uint32_t collision(int s) {
-    double x = d(C_X, s), y = d(C_Y, s), ox = d(C_OX, s), oy = d(C_OY, s);
-    double w = d(C_W, s), e = d(C_E, s), acc = d(C_ACC, s), dstep = d(C_DSTEP, s);
-    double dcen = d(C_DCEN, s);
-    const double dd = d(C_D, s), nd = d(C_ND, s);
-    const double sig = nd * d(C_ST, s);
-    const double pa = d(C_PA, s);
-    const int32_t cx = i(C_CX, s), cy = i(C_CY, s);
-    uint32_t ctr = (uint32_t)i(C_CTR, s);
-    const uint32_t nf = (uint32_t)i(C_NF, s);
-    const uint32_t nc = (uint32_t)i(C_NC, s) + 1u;
-    acc += ((w * dd) * sig) * d(C_H, s);
-    x = x + dd * ox;
-    y = y + dd * oy;
-    dcen = dcen - dd;
-    const uint64_t pid = (uint64_t)(P.first_id + i(C_PID, s));
-    const U64x2 r = threefry2x64_20((uint64_t)ctr, 0, pid, P.seed);
-    ctr += 1u;
+  __device__ uint32_t collision(int s, uint32_t ty) {
+    St v;
+    v.x = d(C_X, s); v.y = d(C_Y, s); v.ox = d(C_OX, s); v.oy = d(C_OY, s);
+    v.mfp = d(C_MFP, s); v.dcen = d(C_DCEN, s);
+    v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
+    v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.e = d(C_E, s); v.st = d(C_ST, s); v.H = d(C_H, s);
+    v.nd = d(C_ND, s);
+    load_nfc(s, v);
+    v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
+    const double dd = d(C_D, s), pa = d(C_PA, s);
+    const double sig = v.nd * v.st;
+    v.nc += 1u;
+    v.acc += ((v.w * dd) * sig) * v.H;
+    v.x = v.x + dd * v.ox;
+    v.y = v.y + dd * v.oy;
+    v.dcen = v.dcen - dd;
+    const uint64_t pid = (uint64_t)(P.first_id + cpid[s]);
+    const U64x2 r = threefry2x64_20((uint64_t)v.ctr, 0, pid, P.seed);
+    v.ctr += 1u;
     double mfp_u = u01(r.b);
     bool absorbed = false;
     if (!ph.analog) {                           // implicit capture
-      const double w0 = w;
-      w = w * (1.0 - pa);
-      fsum(SF_ABSORBED_W, w0 - w);
+      const double w0 = v.w;
+      v.w = v.w * (1.0 - pa);
+      fsum(SF_ABSORBED_W, w0 - v.w);
     } else if (u01(r.b) < pa) {                // sampled absorption (R31)
       absorbed = true;
     } else {                                    // scatter: n_mfp from the next counter
-      const U64x2 r2 = threefry2x64_20((uint64_t)ctr, 0, pid, P.seed);
-      ctr += 1u;
+      const U64x2 r2 = threefry2x64_20((uint64_t)v.ctr, 0, pid, P.seed);
+      v.ctr += 1u;
       mfp_u = u01(r2.a);
     }
     if (absorbed) {
-      flush(s, cx, cy, acc, dstep);
-      fsum(SF_ABSORBED_W, w);
-      fsum(SF_ABSORBED_E, w * e);
+      flush(s, v);
+      fsum(SF_ABSORBED_W, v.w);
+      fsum(SF_ABSORBED_E, v.w * v.e);
       cnt(SU_ABSORBED, 1u);
-      return finish(s, x, y, ox, oy, e, w, d(C_MFP, s), dstep, cx, cy, ctr, nf, nc, false);
+      return finish(s, v, false);
     }
+    const double e = v.e;
     const double mu = 1.0 - 2.0 * u01(r.a);
     const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
     const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
     const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
     const double q = 1.0 - ct * ct;
     const double stt = sgn * sqrt(q > 0.0 ? q : 0.0);
-    const double nox = ox * ct - oy * stt;
-    const double noy = ox * stt + oy * ct;
-    ox = nox;
-    oy = noy;
-    const double tcen = dcen / speed(e, ph);
-    e = e2;
-    bool kill = e < ph.e_min || w < ph.w_min;   // termination
-    if (kill && ph.roulette && !(e < ph.e_min)) {
+    const double nox = v.ox * ct - v.oy * stt;
+    const double noy = v.ox * stt + v.oy * ct;
+    v.ox = nox;
+    v.oy = noy;
+    const double tcen = v.dcen / speed(e, ph);
+    v.e = e2;
+    bool kill = v.e < ph.e_min || v.w < ph.w_min;   // termination
+    if (kill && ph.roulette && !(v.e < ph.e_min)) {
       // Russian roulette (R32): survive with probability w / w_s at weight w_s
-      const U64x2 r3 = threefry2x64_20((uint64_t)ctr, 0, pid, P.seed);
-      ctr += 1u;
-      if (u01(r3.a) < w / ph.w_roul) {
-        fsum(SF_ROULETTE, ph.w_roul - w);
-        w = ph.w_roul;
+      const U64x2 r3 = threefry2x64_20((uint64_t)v.ctr, 0, pid, P.seed);
+      v.ctr += 1u;
+      if (u01(r3.a) < v.w / ph.w_roul) {
+        fsum(SF_ROULETTE, ph.w_roul - v.w);
+        v.w = ph.w_roul;
         kill = false;
       }
     }
     if (kill) {
-      flush(s, cx, cy, acc, dstep);
-      fsum(SF_KILLED_E, w * e);
-      fsum(SF_KILLED_W, w);
+      flush(s, v);
+      fsum(SF_KILLED_E, v.w * v.e);
+      fsum(SF_KILLED_W, v.w);
       cnt(SU_KILLED, 1u);
-      return finish(s, x, y, ox, oy, e, w, d(C_MFP, s), dstep, cx, cy, ctr, nf, nc, false);
+      return finish(s, v, false);
     }
-    double exn = __ldg(P.mesh.ex + cx + (ox > 0.0 ? 1 : 0));
-    double eyn = __ldg(P.mesh.ey + cy + (oy > 0.0 ? 1 : 0));
-    dcen = tcen * speed(e, ph);
+    v.exn = edge_x(v.cx + (v.ox > 0.0 ? 1 : 0));
+    v.eyn = edge_y(v.cy + (v.oy > 0.0 ? 1 : 0));
+    v.dcen = tcen * speed(v.e, ph);
     uint32_t nr = 0;
-    const Mat m = refresh_xs(P.xs, ph, e, nr);
+    const Mat m = refresh_xs(P.xs, ph, v.e, nr);
     if (nr) cnt(SU_XS_RANGE, nr);
-    double iox = 1.0 / ox, ioy = 1.0 / oy;
-    if (ox == 0.0) { exn = ev_inf(); iox = ev_inf(); }
-    if (oy == 0.0) { eyn = ev_inf(); ioy = ev_inf(); }
-    d(C_X, s) = x; d(C_Y, s) = y; d(C_OX, s) = ox; d(C_OY, s) = oy;
-    d(C_IOX, s) = iox; d(C_IOY, s) = ioy; d(C_EXN, s) = exn; d(C_EYN, s) = eyn;
-    d(C_MFP, s) = -log(mfp_u); d(C_DCEN, s) = dcen; d(C_ACC, s) = acc;
-    d(C_W, s) = w; d(C_E, s) = e; d(C_ST, s) = m.st; d(C_H, s) = m.H; d(C_PA, s) = m.pa;
-    i(C_NC, s) = (int32_t)nc;
-    i(C_CTR, s) = (int32_t)ctr;
-    return classify(s, nf, nc);
+    v.st = m.st;
+    v.H = m.H;
+    v.iox = 1.0 / v.ox;
+    v.ioy = 1.0 / v.oy;
+    if (v.ox == 0.0) { v.exn = ev_inf(); v.iox = ev_inf(); }
+    if (v.oy == 0.0) { v.eyn = ev_inf(); v.ioy = ev_inf(); }
+    v.mfp = -log(mfp_u);
+    i2(C_CTRSEQ, s).x = (int)v.ctr;
+    i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);
+    if ((int64_t)(v.nf + v.nc) >= P.max_events) return cap_kill(s, v);
+    d(C_X, s) = v.x; d(C_Y, s) = v.y; d(C_OX, s) = v.ox; d(C_OY, s) = v.oy;
+    d(C_IOX, s) = v.iox; d(C_IOY, s) = v.ioy; d(C_EXN, s) = v.exn; d(C_EYN, s) = v.eyn;
+    d(C_MFP, s) = v.mfp; d(C_DCEN, s) = v.dcen; d(C_ACC, s) = v.acc;
+    d(C_W, s) = v.w; d(C_E, s) = v.e; d(C_ST, s) = v.st; d(C_H, s) = v.H; d(C_PA, s) = m.pa;
+    return classify(s, v);
   }
 
   // ---- facet ----
-  __device__ uint32_t facet(int s, bool ax) {
-    double x = d(C_X, s), y = d(C_Y, s);
-    double acc = d(C_ACC, s), dstep = d(C_DSTEP, s);
-    const double dd = d(C_D, s), w = d(C_W, s);
-    const double sig = d(C_ND, s) * d(C_ST, s);
-    int32_t cx = i(C_CX, s), cy = i(C_CY, s);
-    const uint32_t nf = (uint32_t)i(C_NF, s) + 1u;
-    acc += ((w * dd) * sig) * d(C_H, s);
-    d(C_MFP, s) = clamp0(d(C_MFP, s) - dd * sig);
-    d(C_DCEN, s) = d(C_DCEN, s) - dd;
-    const double ox = d(C_OX, s), oy = d(C_OY, s);
-    const double xm = x + dd * ox, ym = y + dd * oy;
-    x = ax ? d(C_EXN, s) : xm;                  // snap the crossed coordinate
-    y = ax ? ym : d(C_EYN, s);
-    flush(s, cx, cy, acc, dstep);               // deposit of the cell being left
-    const int32_t c = ax ? cx : cy;
-    const bool pos = ax ? (ox > 0.0) : (oy > 0.0);
+  __device__ uint32_t facet(int s, uint32_t ty) {
+    const bool ax = (ty & T_AXBIT) != 0;
+    St v;
+    v.x = d(C_X, s); v.y = d(C_Y, s);
+    v.iox = d(C_IOX, s); v.ioy = d(C_IOY, s); v.exn = d(C_EXN, s); v.eyn = d(C_EYN, s);
+    // the direction cosine of the coordinate that moves (the other is snapped to the edge);
+    // the crossed axis' direction is the sign of its reciprocal
+    const double om = d(ax ? C_OY : C_OX, s);
+    v.mfp = d(C_MFP, s); v.dcen = d(C_DCEN, s);
+    v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
+    v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.st = d(C_ST, s); v.H = d(C_H, s);
+    v.nd = d(C_ND, s);
+    load_nfc(s, v);
+    const double dd = d(C_D, s);
+    const double sig = v.nd * v.st;
+    v.nf += 1u;
+    v.acc += ((v.w * dd) * sig) * v.H;
+    v.mfp = clamp0(v.mfp - dd * sig);
+    v.dcen = v.dcen - dd;
+    const double moved = (ax ? v.y : v.x) + dd * om;
+    v.x = ax ? v.exn : moved;                   // snap the crossed coordinate
+    v.y = ax ? moved : v.eyn;
+    flush(s, v);                                // deposit of the cell being left
+    const int32_t c = ax ? v.cx : v.cy;
+    const bool pos = (ax ? v.iox : v.ioy) > 0.0;
     const int32_t cs = c + (pos ? 1 : -1);
-    const bool refl = (uint32_t)cs >= (uint32_t)(ax ? P.mesh.nx : P.mesh.ny);
+    const bool refl = (uint32_t)cs >= (uint32_t)(ax ? P.mesh.gnx : P.mesh.ny);
     const int32_t c2 = refl ? c : cs;
     if (refl) {
+      v.ox = d(C_OX, s);
+      v.oy = d(C_OY, s);
       if (ph.vacuum) {                          // vacuum boundary (R30): escape
+        v.e = d(C_E, s);
+        v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
         cnt(SU_ESCAPED, 1u);
-        const double e = d(C_E, s);
-        fsum(SF_ESCAPED_E, w * e);
-        fsum(SF_ESCAPED_W, w);
-        return finish(s, x, y, ox, oy, e, w, d(C_MFP, s), dstep, cx, cy, (uint32_t)i(C_CTR, s), nf,
-                      (uint32_t)i(C_NC, s), false);
+        fsum(SF_ESCAPED_E, v.w * v.e);
+        fsum(SF_ESCAPED_W, v.w);
+        return finish(s, v, false);
       }
-      if (ax) { d(C_OX, s) = -ox; d(C_IOX, s) = -d(C_IOX, s); }
-      else    { d(C_OY, s) = -oy; d(C_IOY, s) = -d(C_IOY, s); }
+      if (ax) { v.ox = -v.ox; v.iox = -v.iox; d(C_OX, s) = v.ox; d(C_IOX, s) = v.iox; }
+      else    { v.oy = -v.oy; v.ioy = -v.ioy; d(C_OY, s) = v.oy; d(C_IOY, s) = v.ioy; }
     }
     const bool pos2 = refl ? !pos : pos;
     const int32_t ke = pos2 ? c2 + 1 : c2;
-    if (ax) { cx = c2; d(C_EXN, s) = __ldg(P.mesh.ex + ke); i(C_CX, s) = cx; }
-    else    { cy = c2; d(C_EYN, s) = __ldg(P.mesh.ey + ke); i(C_CY, s) = cy; }
-    d(C_X, s) = x;
-    d(C_Y, s) = y;
-    d(C_ACC, s) = acc;
-    d(C_DSTEP, s) = dstep;
-    d(C_ND, s) = nd_of(cx, cy);                 // the new cell's density
-    i(C_NF, s) = (int32_t)nf;
-    return classify(s, nf, (uint32_t)i(C_NC, s));
+    if (ax) { v.cx = c2; v.exn = edge_x(ke); d(C_EXN, s) = v.exn; }
+    else    { v.cy = c2; v.eyn = edge_y(ke); d(C_EYN, s) = v.eyn; }
+    v.nd = nd_of(v.cx, v.cy);                   // the new cell's density
+    i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);
+    if ((int64_t)(v.nf + v.nc) >= P.max_events) {
+      v.e = d(C_E, s);
+      v.ox = d(C_OX, s);
+      v.oy = d(C_OY, s);
+      v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
+      i2(C_CXY, s) = make_int2(v.cx, v.cy);
+      return cap_kill(s, v);
+    }
+    d(C_X, s) = v.x;
+    d(C_Y, s) = v.y;
+    d(C_MFP, s) = v.mfp;
+    d(C_DCEN, s) = v.dcen;
+    d(C_DSTEP, s) = v.dstep;
+    d(C_ND, s) = v.nd;
+    i2(C_CXY, s) = make_int2(v.cx, v.cy);
+    return classify(s, v);                      // acc == 0 after the flush
   }
 
   // ---- census ----
-  __device__ uint32_t census(int s) {
-    double acc = d(C_ACC, s), dstep = d(C_DSTEP, s);
-    const double dd = d(C_D, s), w = d(C_W, s), e = d(C_E, s);
-    const double ox = d(C_OX, s), oy = d(C_OY, s);
+  __device__ uint32_t census(int s, uint32_t ty) {
+    St v;
+    v.ox = d(C_OX, s); v.oy = d(C_OY, s);
+    v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
+    v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.e = d(C_E, s);
+    load_nfc(s, v);
+    v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
+    const double dd = d(C_D, s);
     const double sig = d(C_ND, s) * d(C_ST, s);
-    const int32_t cx = i(C_CX, s), cy = i(C_CY, s);
-    acc += ((w * dd) * sig) * d(C_H, s);
-    const double x = d(C_X, s) + dd * ox;
-    const double y = d(C_Y, s) + dd * oy;
+    v.acc += ((v.w * dd) * sig) * d(C_H, s);
+    v.x = d(C_X, s) + dd * v.ox;
+    v.y = d(C_Y, s) + dd * v.oy;
     const double nm = d(C_MFP, s) - dd * sig;
-    const double mfp = nm > 0.0 ? nm : 0.0;
-    flush(s, cx, cy, acc, dstep);
+    v.mfp = nm > 0.0 ? nm : 0.0;
+    flush(s, v);
     cnt(SU_CENSUS, 1u);
-    fsum(SF_CENSUS_E, w * e);
-    fsum(SF_CENSUS_W, w);
-    return finish(s, x, y, ox, oy, e, w, mfp, dstep, cx, cy, (uint32_t)i(C_CTR, s),
-                  (uint32_t)i(C_NF, s), (uint32_t)i(C_NC, s), true);
+    fsum(SF_CENSUS_E, v.w * v.e);
+    fsum(SF_CENSUS_W, v.w);
+    return finish(s, v, true);
   }
 
-  // ---- a new particle (local index in C_PID): its slot state and first event ----
+  // ---- a new particle (local index in cpid): its slot state and first event ----
   __device__ uint32_t birth(int s) {
-    const int32_t pi = i(C_PID, s);
+    const int32_t pi = cpid[s];
     if (P.p.status[pi] != 1u) return T_FREE;
-    const double ox = P.p.ox[pi], oy = P.p.oy[pi];
-    const double e = P.p.e[pi];
-    const int32_t cx = P.p.cx[pi], cy = P.p.cy[pi];
+    St v;
+    v.ox = P.p.ox[pi]; v.oy = P.p.oy[pi];
+    v.e = P.p.e[pi];
+    v.cx = P.p.cx[pi]; v.cy = P.p.cy[pi];
     uint32_t nr = 0;
-    const Mat m = refresh_xs(P.xs, ph, e, nr);
+    const Mat m = refresh_xs(P.xs, ph, v.e, nr);
     if (nr) cnt(SU_XS_RANGE, nr);
-    double exn = __ldg(P.mesh.ex + cx + (ox > 0.0 ? 1 : 0));
-    double eyn = __ldg(P.mesh.ey + cy + (oy > 0.0 ? 1 : 0));
-    double iox = 1.0 / ox, ioy = 1.0 / oy;
-    if (ox == 0.0) { exn = ev_inf(); iox = ev_inf(); }
-    if (oy == 0.0) { eyn = ev_inf(); ioy = ev_inf(); }
-    d(C_X, s) = P.p.x[pi]; d(C_Y, s) = P.p.y[pi]; d(C_OX, s) = ox; d(C_OY, s) = oy;
-    d(C_IOX, s) = iox; d(C_IOY, s) = ioy; d(C_EXN, s) = exn; d(C_EYN, s) = eyn;
-    d(C_MFP, s) = P.p.mfp[pi]; d(C_DCEN, s) = speed(e, ph) * P.dt;
-    d(C_ACC, s) = 0.0; d(C_DSTEP, s) = 0.0;
-    d(C_W, s) = P.p.w[pi]; d(C_E, s) = e; d(C_ST, s) = m.st; d(C_H, s) = m.H; d(C_PA, s) = m.pa;
-    d(C_ND, s) = nd_of(cx, cy);
-    i(C_CX, s) = cx; i(C_CY, s) = cy; i(C_NF, s) = 0; i(C_NC, s) = 0;
-    i(C_CTR, s) = (int32_t)P.p.ctr[pi]; i(C_SEQ, s) = 0;
+    v.exn = edge_x(v.cx + (v.ox > 0.0 ? 1 : 0));
+    v.eyn = edge_y(v.cy + (v.oy > 0.0 ? 1 : 0));
+    v.iox = 1.0 / v.ox;
+    v.ioy = 1.0 / v.oy;
+    if (v.ox == 0.0) { v.exn = ev_inf(); v.iox = ev_inf(); }
+    if (v.oy == 0.0) { v.eyn = ev_inf(); v.ioy = ev_inf(); }
+    v.x = P.p.x[pi]; v.y = P.p.y[pi];
+    v.mfp = P.p.mfp[pi]; v.dcen = speed(v.e, ph) * P.dt;
+    v.acc = 0.0; v.dstep = 0.0;
+    v.w = P.p.w[pi]; v.st = m.st; v.H = m.H;
+    v.nd = nd_of(v.cx, v.cy);
+    v.nf = 0u; v.nc = 0u;
+    v.ctr = P.p.ctr[pi];
     cnt(SU_ALIVE, 1u);
-    return classify(s, 0u, 0u);
+    d(C_X, s) = v.x; d(C_Y, s) = v.y; d(C_OX, s) = v.ox; d(C_OY, s) = v.oy;
+    d(C_IOX, s) = v.iox; d(C_IOY, s) = v.ioy; d(C_EXN, s) = v.exn; d(C_EYN, s) = v.eyn;
+    d(C_MFP, s) = v.mfp; d(C_DCEN, s) = v.dcen; d(C_DSTEP, s) = 0.0;
+    d(C_W, s) = v.w; d(C_E, s) = v.e; d(C_ST, s) = v.st; d(C_H, s) = v.H; d(C_PA, s) = m.pa;
+    d(C_ND, s) = v.nd;
+    i2(C_CXY, s) = make_int2(v.cx, v.cy);
+    i2(C_NFC, s) = make_int2(0, 0);
+    i2(C_CTRSEQ, s) = make_int2((int)v.ctr, 0);
+    if (P.max_events <= 0) return cap_kill(s, v);
+    return classify(s, v);
   }
 };
 
@@ -387,8 +458,8 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
   __shared__ unsigned long long s_u[SU_COUNT];
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
   double* c8 = reinterpret_cast<double*>(smem);
-  int32_t* c4 = reinterpret_cast<int32_t*>(c8 + (size_t)kCol8 * kSlots);
-  uint8_t* s_type = reinterpret_cast<uint8_t*>(c4 + (size_t)kCol4 * kSlots);
+  int32_t* cpid = reinterpret_cast<int32_t*>(c8 + (size_t)kCol8 * kSlots);
+  uint8_t* s_type = reinterpret_cast<uint8_t*>(cpid + kSlots);
   uint8_t* s_wq = s_type + kSlots;             // per-warp event queue (slot offsets)
   uint8_t* s_blk = s_wq + kSlots;              // block map (kBlk)
   const int t = threadIdx.x;
@@ -410,7 +481,7 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
     }
   }
   __syncthreads();
-  EvKernel<kDet, kFmt, kBlk> K{P, P.ph, s_nd, s_blk, s_u, P.slot_f + gt, sstride, l2_evict_last(), c8, c4};
+  EvKernel<kDet, kFmt, kBlk> K{P, P.ph, s_nd, s_blk, s_u, P.slot_f + gt, sstride, l2_evict_last(), c8, cpid};
   const unsigned long long span = (unsigned long long)(P.hi - P.lo);
   const int sb = wid * kWSlots;                // this warp's slots [sb, sb + 64)
   uint8_t* wq = s_wq + sb;
@@ -430,11 +501,11 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
       if (base + nfree >= span) exhausted = true;
       const unsigned ra = (unsigned)__popc(fa & lt), rb = (unsigned)(__popc(fa) + __popc(fb & lt));
       if (ta == T_FREE && ra < avail) {
-        K.i(C_PID, sb + lane) = (int32_t)(P.lo + (int64_t)(base + ra));
+        cpid[sb + lane] = (int32_t)(P.lo + (int64_t)(base + ra));
         ta = T_BIRTH;
       }
       if (tb == T_FREE && rb < avail) {
-        K.i(C_PID, sb + 32 + lane) = (int32_t)(P.lo + (int64_t)(base + rb));
+        cpid[sb + 32 + lane] = (int32_t)(P.lo + (int64_t)(base + rb));
         tb = T_BIRTH;
       }
     }
@@ -443,25 +514,36 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
       continue;
     }
     // ---- Listing 2: all collisions, then all facets, then all census, then the births ----
+    // Each type's queue is compacted per slot half (slots sb + lane, then sb + 32 + lane): a
+    // half's 32 slots lie in distinct 4-byte banks pairwise, so the handlers' 8-byte column
+    // accesses of any subset of them take the minimum two shared-memory wavefronts (a queue
+    // drawn from all 64 slots would put up to four lanes on one bank pair).
+    // the event types present in the warp's slots (one REDUX): absent types cost nothing
+    const unsigned present = __reduce_or_sync(kFull, (1u << (ta & 7u)) | (1u << (tb & 7u)));
 #pragma unroll 1
     for (uint32_t T = 0; T < 4; ++T) {
-      const bool a = (ta & 7u) == T, b = (tb & 7u) == T;
-      const unsigned ma = __ballot_sync(kFull, a), mb = __ballot_sync(kFull, b);
-      const int na = __popc(ma), n = na + __popc(mb);
-      if (n == 0) continue;
-      if (a) wq[__popc(ma & lt)] = (uint8_t)lane;
-      if (b) wq[na + __popc(mb & lt)] = (uint8_t)(32 + lane);
-      __syncwarp();
-      for (int k = lane; k < n; k += 32) {
-        const int s = sb + wq[k];
-        uint32_t nt;
-        if (T == T_COLL) nt = K.collision(s);
-        else if (T == T_FACET) nt = K.facet(s, (s_type[s] & T_AXBIT) != 0);
-        else if (T == T_CENSUS) nt = K.census(s);
-        else nt = K.birth(s);
-        s_type[s] = (uint8_t)nt;
+      if (!(present & (1u << T))) continue;
+#pragma unroll 1
+      for (int h = 0; h < 2; ++h) {
+        const uint32_t ty = h ? tb : ta;
+        const bool mine = (ty & 7u) == T;
+        const unsigned m = __ballot_sync(kFull, mine);
+        if (m == 0u) continue;
+        const int n = __popc(m);
+        if (mine) wq[__popc(m & lt)] = (uint8_t)(32 * h + lane);
+        __syncwarp();
+        if (lane < n) {
+          const int s = sb + wq[lane];
+          const uint32_t tys = s_type[s];
+          uint32_t nt;
+          if (T == T_COLL) nt = K.collision(s, tys);
+          else if (T == T_FACET) nt = K.facet(s, tys);
+          else if (T == T_CENSUS) nt = K.census(s, tys);
+          else nt = K.birth(s);
+          s_type[s] = (uint8_t)nt;
+        }
+        __syncwarp();
       }
-      __syncwarp();
     }
   }
   if (lane == 0 && iter > 0) atomicMax(&E.ctl->iter, iter);

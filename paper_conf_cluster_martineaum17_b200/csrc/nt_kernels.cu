@@ -123,16 +123,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const unsigned long long span = (unsigned long long)(P.hi - P.lo);
   const double* __restrict__ ex = P.mesh.ex;
   const double* __restrict__ ey = P.mesh.ey;
-  const int32_t nx = P.mesh.nx, ny = P.mesh.ny;
+  const int32_t nx = P.mesh.gnx, ny = P.mesh.ny;      // reflection bounds (whole mesh)
+  const int32_t snx = P.mesh.nx, x0 = P.mesh.x0;      // storage width, first stored column
   const Phys& ph = P.ph;
   const uint32_t strip = (uint32_t)P.mesh.strip;        // tiled: cells per row of tiles
   // storage index of (cx, cy): 4x4 tiles (kTiled) or row-major, as nt_device.cuh cell_index
   // (32-bit: nt_init_mesh guarantees the storage fits 2^32 cells)
   auto cidx_of = [&](int32_t cx_, int32_t cy_) -> uint32_t {
+    const uint32_t lx = kSlab ? (uint32_t)(cx_ - x0) : (uint32_t)cx_;   // x-slab storage offset
     if constexpr (kTiled)
-      return (uint32_t)(cy_ >> 2) * strip + ((uint32_t)cx_ << 2) + (uint32_t)(cy_ & 3);
+      return (uint32_t)(cy_ >> 2) * strip + (lx << 2) + (uint32_t)(cy_ & 3);
     else
-      return (uint32_t)cy_ * (uint32_t)nx + (uint32_t)cx_;
+      return (uint32_t)cy_ * (uint32_t)snx + lx;
   };
   const uint32_t max_ev = P.max_events < 0xffffffffll ? (uint32_t)P.max_events : 0xffffffffu;
   const uint64_t pol_keep = l2_evict_last();     // tally REDs, density gathers
@@ -144,7 +146,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   };
   // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather
   auto dload = [&](int32_t cx_, int32_t cy_, uint32_t ci_) {
-    if constexpr (kBlk) return dens_load_blk(P.mesh, s_blk, cx_, cy_, ci_, pol_keep);
+    if constexpr (kBlk) return dens_load_blk<kSlab>(P.mesh, s_blk, cx_, cy_, ci_, pol_keep);
     else return dens_load<kFmt>(P.mesh, ci_, pol_keep);
   };
 
@@ -238,8 +240,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
             cx = ld_stream(P.p.cx + i, pol_stream);
             cy = ld_stream(P.p.cy + i, pol_stream);
             ctr = ld_stream(P.p.ctr + i, pol_stream);
-            cidx = cidx_of(cx, cy);
-            draw = dload(cx, cy, cidx);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             iox = 1.0 / ox;
@@ -269,9 +269,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
               nc = P.p.nc_s[i];
               if constexpr (kDet) seq = P.p.seq_s[i];
             }
+            // born (or resumed) outside this rank's slab: hand over before any event (and
+            // before touching the density, which this rank holds for its columns only)
+            bool stay = true;
             if constexpr (kSlab) {
-              // born (or resumed) outside this rank's slab: hand over before any event
-              if (outside_slab(cx)) park_to(4u, P.out_q, P.out_count);
+              if (outside_slab(cx)) {
+                park_to(4u, P.out_q, P.out_count);
+                stay = false;
+              }
+            }
+            if (stay) {
+              cidx = cidx_of(cx, cy);
+              draw = dload(cx, cy, cidx);
             }
           }
         }

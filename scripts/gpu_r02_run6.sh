@@ -1,0 +1,9 @@
+OUT=gpurun_out/r02_t6; mkdir -p $OUT
+python -c "import __graft_entry__ as g; g.build()"
+NT_PARITY_REPORT=$OUT/parity timeout 2400 python -m pytest tests -m gpu -q -p no:cacheprovider -x > $OUT/pytest_gpu.log 2>&1
+echo "PYTEST $(tail -1 $OUT/pytest_gpu.log)"; grep -E "^FAILED|Error" $OUT/pytest_gpu.log | head -10
+for c in csp stream split scatter; do
+  timeout 300 python bench.py --config $c --no-cpu-baseline --no-e2e --no-extras --steps 5 --json-out $OUT/b_$c.json > /dev/null 2>&1
+  python -c "import json; d=json.load(open('$OUT/b_$c.json')); print('$c history', '%.2f ms' % d['roofline']['kernel_ms'], 'frac %.3f' % d['roofline']['frac'], d['clocks']['sm_mhz'])" 2>&1 | tail -1
+done
+bash scripts/dev/ab_variants.sh r02_ab3_evedge "evdiv evldg" "csp:event stream:event split:event scatter:event" 2 2>&1 | grep -v pytest

@@ -28,6 +28,10 @@ KEYS = [
     "launch__block_size", "smsp__thread_inst_executed_per_inst_executed.ratio",
     "sm__pipe_fp64_cycles_active.avg.pct_of_peak_sustained_active", "smsp__inst_executed.sum",
     "smsp__issue_active.avg.pct_of_peak_sustained_active", "sm__throughput.avg.pct_of_peak_sustained_elapsed",
+    # shared memory (the event variant's slot state)
+    "smsp__inst_executed_op_shared_ld.sum", "smsp__inst_executed_op_shared_st.sum",
+    "l1tex__data_pipe_lsu_wavefronts_mem_shared_op_ld.sum", "l1tex__data_pipe_lsu_wavefronts_mem_shared_op_st.sum",
+    "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_ld.sum", "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_st.sum",
 ]
 STALL = re.compile(r"^smsp__pcsamp_warps_issue_stalled_([a-z_]+)$")
 
@@ -128,6 +132,53 @@ def main():
                                 sorted(mix.items(), key=lambda kv: -kv[1])[:24])]
     except Exception as e:  # noqa: BLE001
         lines.append(f"(source page unavailable: {e})")
+    # CUDA source lines (needs -lineinfo and --import-source on): stall samples and executed
+    # instructions of the SASS under each line of our .cu/.cuh files ("cuda,sass" listing:
+    # a "File Path" row per file, a "Function Name" row per kernel, then each source line
+    # followed by its SASS rows)
+    try:
+        src = list(csv.reader(io.StringIO(ncu(["-i", a.rep, "--page", "source", "--csv",
+                                                "--print-source", "cuda,sass"]))))
+        agg: dict[str, dict] = {}
+        fname, func, line, h = "", "", None, None
+        seen_pairs: dict = {}
+        for row in src:
+            if not row:
+                continue
+            if row[0] == "File Path":
+                fname = Path(row[1]).name if len(row) > 1 else ""
+            elif row[0] == "Function Name":
+                # a (file, function) block repeats for every captured launch of the kernel
+                fn = row[1] if len(row) > 1 else ""
+                n_seen = seen_pairs.get((fname, fn), 0)
+                seen_pairs[(fname, fn)] = n_seen + 1
+                func = f"launch {n_seen}: {fn}"
+                line = None
+            elif row[0] == "Line No":
+                h = row
+            elif h is not None:
+                if row[0]:
+                    line = (row[0], row[1].strip())
+                    continue
+                if line is None:
+                    continue
+                iW = h.index("Warp Stall Sampling (All Samples)")
+                iE = h.index("Instructions Executed")
+                iT = h.index("Thread Instructions Executed")
+                f = lambda v: float(v) if v.replace(".", "", 1).isdigit() else 0.0  # noqa: E731
+                k = agg.setdefault(func, {}).setdefault((fname, line[0]), {"src": line[1], "w": 0.0, "e": 0.0, "t": 0.0})
+                k["w"] += f(row[iW])
+                k["e"] += f(row[iE])
+                k["t"] += f(row[iT])
+        for nb, (func, d) in enumerate(agg.items()):
+            tot = sum(v["w"] for v in d.values()) or 1.0
+            lines += ["", f"### {func[:70]}...: top {a.top} stall-sampled CUDA source lines", "",
+                      "| file:line | stall share | warp instr executed | avg threads | source |", "|---|---|---|---|---|"]
+            for (fn, ln), v in sorted(d.items(), key=lambda kv: -kv[1]["w"])[:a.top]:
+                thr = v["t"] / v["e"] if v["e"] else 0.0
+                lines.append(f"| {fn}:{ln} | {100 * v['w'] / tot:.1f}% | {v['e']:.4g} | {thr:.1f} | `{v['src'][:80]}` |")
+    except Exception as e:  # noqa: BLE001
+        lines.append(f"(CUDA source page unavailable: {e})")
     Path(a.out).write_text("\n".join(lines) + "\n")
     if a.traffic_key and traffic:
         p = Path(a.out).parent / "ncu_traffic.json"

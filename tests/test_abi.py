@@ -40,7 +40,7 @@ def test_exports_every_declared_symbol(L):
 
 def test_identity_calls(L):
     from paper_conf_cluster_martineaum17_b200 import binding
-    assert L.nt_abi_version() == 4
+    assert L.nt_abi_version() == 5
     assert b"sm_100a" in L.nt_build_info()
     assert b"-fmad=false" in L.nt_build_info()
     for k, v in binding.STATUS.items():

@@ -419,6 +419,27 @@ def test_slab_decomposition_matches_oracle(nt, orc, cfgname, nslabs):
     assert rounds >= 2 if cfg.density != "uniform_hi" else True
 
 
+def test_slab_storage_scales_with_ranks(nt, orc):
+    """x-slab ranks store only their columns plus a one-column halo (§IX: a
+    decomposition is what lets a mesh exceed one node's memory): the mesh bytes of a
+    4-slab rank are about a quarter of the replicated context's, and the slabs' tallies
+    still add up to the oracle's."""
+    cfg = wl.CONFIGS["tiny_csp"].with_(nx=1024, ny=1024, n_particles=2000, name="slab_mem")
+    rep = nt.setup(cfg)
+    full = rep.mesh_bytes()
+    rep.close()
+    ranks = [nt.setup(cfg, first_id=lo, n_local=n, rank=r, nranks=4, decomposition=1)
+             for r, (lo, n) in enumerate(wl.shard(cfg.n_particles, r, 4) for r in range(4))]
+    for t in ranks:
+        assert t.mesh_bytes() <= 0.27 * full, (t.mesh_bytes(), full)
+    for t in ranks:
+        t.close()
+    gt, gp, gs, rounds = _run_slabs(nt, cfg, 4)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)
+    compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+
+
 @pytest.mark.parametrize("mode", ["history", "event"])
 @pytest.mark.parametrize("cap", [1, 255, 256, 257, 300, 600])
 @pytest.mark.parametrize("det", [True, False])
