@@ -185,19 +185,33 @@ def parse():
     ap.add_argument("--layout", type=int, default=0, help="0 tiled 4x4 (default), 1 row-major")
     ap.add_argument("--density-format", type=int, default=0,
                     help="0 u8/u16 codes + block map (default), 1 f64 map, 2 codes without block map")
-    ap.add_argument("--tally-mode", type=int, default=0, help="0 one RED per flush, 1 warp-aggregated")
+    ap.add_argument("--tally-mode", type=int, default=0,
+                    help="0 one RED per flush, 1 warp-aggregated, 2 CAS-emulated fp64 add, "
+                         "3 shared-memory hot window around the source")
     ap.add_argument("--defer-below", type=int, default=0,
                     help="collision deferral threshold (0 default 8, 1 off, 33 park every collision)")
     ap.add_argument("--xs-search", type=int, default=0,
                     help="0 bucketed binary search, 1 plain binary search, 2 cached-bin linear walk")
     ap.add_argument("--table-size", type=int, default=0,
                     help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
+    ap.add_argument("--particle-layout", type=int, default=0,
+                    help="0 structure of arrays (default), 1 AoS records while tracking (ablation)")
     ap.add_argument("--json-out", default=None)
     ap.add_argument("--no-extras", action="store_true",
                     help="skip the short runs of the other configs / modes added to the JSON line")
     ap.add_argument("--mesh", type=int, default=0, help="experiment: override nx = ny")
     ap.add_argument("--particles", type=int, default=0, help="experiment: override the particle count")
     return ap.parse_args()
+
+
+def hot_window(cfg, margin=2, cells=2048):
+    """tally_mode 3's privatised window: the cells around the source rectangle (<= 2048)."""
+    sx, sy, sw, sh = cfg.source
+    x0 = max(0, int(sx / cfg.width * cfg.nx) - margin)
+    y0 = max(0, int(sy / cfg.height * cfg.ny) - margin)
+    nx = max(1, min(cfg.nx - x0, int(math.ceil(sw / cfg.width * cfg.nx)) + 2 * margin, cells))
+    ny = max(1, min(cfg.ny - y0, int(math.ceil(sh / cfg.height * cfg.ny)) + 2 * margin, cells // nx))
+    return (x0, y0, nx, ny)
 
 
 def dist_env():
@@ -324,7 +338,8 @@ def main():
                          e_min=cfg.e_min, w_min=cfg.w_min, ctas_per_sm=a.ctas_per_sm,
                          refill_min=a.refill_min, layout=a.layout, density_format=a.density_format,
                          tally_mode=a.tally_mode, defer_below=a.defer_below,
-                         xs_search=a.xs_search)
+                         xs_search=a.xs_search, hot_window=hot_window(cfg),
+                         particle_layout=a.particle_layout)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -429,8 +444,10 @@ def main():
             "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
             "config": {"workload": cfg.name, "mode": a.mode, "nx": cfg.nx, "ny": cfg.ny,
                        "layout": "tiled4x4" if a.layout == 0 else "row-major",
+                       "particle_store": ["SoA", "AoS (ablation)"][a.particle_layout],
                        "density_format": ["codes+block map", "f64", "codes"][a.density_format],
-                       "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED"][a.tally_mode],
+                       "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED", "CAS-emulated fp64 add",
+                                 "shared-memory hot window %s + RED" % (hot_window(cfg),)][a.tally_mode],
                        "defer_below": a.defer_below or 8,
                        "xs_search": ["bucketed binary", "binary", "cached-bin walk"][a.xs_search],
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,

@@ -90,8 +90,12 @@ typedef struct {
     int32_t tally_mode;        /* production tally flushes: 0: one fp64
                                   atomic add per flush; 1: warp-aggregated -- lanes flushing
                                   into the same cell at the same time are summed with warp
-                                  shuffles and one lane issues the atomic (history mode,
-                                  u8 block-map meshes; others fall back to 0)              */
+                                  shuffles and one lane issues the atomic; 2: the fp64 add
+                                  emulated by a 64-bit compare-and-swap loop;
+                                  3: a per-CTA shared-memory copy of the hot window
+                                  hot_* (privatisation), merged with one atomic
+                                  per cell when the CTA ends.  Ablations: history mode,
+                                  production, u8 block-map meshes; others use 0.          */
     int32_t defer_below;       /* history mode, collision deferral: a lane whose next event
                                   is a collision while fewer than this many lanes of its
                                   warp collide is parked (state to the particle store) and
@@ -125,6 +129,12 @@ typedef struct {
                                   neighbour (nt_run_timestep exchanges them over NCCL, or
                                   the caller drives nt_slab_*).  Production tally only.   */
     double roulette_weight;    /* survivor weight (0 -> 2 w_min)                           */
+    int32_t hot_x0, hot_y0;    /* tally_mode 3: first column and row of the hot window     */
+    int32_t hot_nx, hot_ny;    /* its size in cells, hot_nx * hot_ny <= 2048 (16 KB)       */
+    int32_t particle_layout;   /* 0: structure of arrays; 1: array of 128 B
+                                  records while the history kernel runs (ablation, P:526-551;
+                                  production tally, default kernel; others use 0)          */
+    int32_t reserved1;
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

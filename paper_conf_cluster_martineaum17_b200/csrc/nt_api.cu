@@ -104,6 +104,7 @@ struct nt_ctx {
   int64_t n_total = 0, first_id = 0, n_local = 0;
   uint64_t seed = 0;
   DevBuf soa;
+  DevBuf aos;                            // particle_layout 1: AoS records during the step
   Soa p{};
   int32_t* defer_q = nullptr;            // regime-parking queue (in soa)
   // x-slab decomposition (decomposition 1)
@@ -280,7 +281,11 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
       !(opt.e_min > 0.0) || !(opt.w_min >= 0.0) || opt.mode < 0 || opt.mode > 1 ||
       opt.rank < 0 || opt.rank >= opt.nranks || opt.density_format < 0 ||
       opt.density_format > 2 || opt.layout < 0 || opt.layout > 1 || opt.tally_mode < 0 ||
-      opt.tally_mode > 1)
+      opt.tally_mode > 3)
+    return NT_ERR_ARG;
+  if (opt.particle_layout < 0 || opt.particle_layout > 1) return NT_ERR_ARG;
+  if (opt.tally_mode == 3 && (opt.hot_x0 < 0 || opt.hot_y0 < 0 || opt.hot_nx < 1 || opt.hot_ny < 1 ||
+                              (int64_t)opt.hot_nx * opt.hot_ny > kHotCells))
     return NT_ERR_ARG;
   // nranks > 1 needs a communicator, except for x-slabs driven by the caller (nt_slab_*)
   if (opt.nranks > 1 && !opt.nccl_unique_id && opt.decomposition != 1) return NT_ERR_ARG;
@@ -332,7 +337,7 @@ nt_status nt_destroy(nt_ctx* c) {
   if (c->evs) event_state_destroy(c->evs);
   for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->tally_full, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
-                    &c->sort_tmp, &c->backup, &c->stats_d})
+                    &c->sort_tmp, &c->backup, &c->stats_d, &c->aos})
     b->release();
   if (c->stats_h) cudaFreeHost(c->stats_h);
   for (auto& ev : c->ev)
@@ -724,6 +729,12 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.seed = c->seed;
   tp.dt = dt;
   tp.max_events = c->opt.max_events_per_history;
+  if (c->opt.tally_mode == 3) {       // the hot window, clipped to the mesh
+    tp.hot_x0 = c->opt.hot_x0 < c->nx ? c->opt.hot_x0 : c->nx - 1;
+    tp.hot_y0 = c->opt.hot_y0 < c->ny ? c->opt.hot_y0 : c->ny - 1;
+    tp.hot_nx = c->opt.hot_nx < c->nx - tp.hot_x0 ? c->opt.hot_nx : c->nx - tp.hot_x0;
+    tp.hot_ny = c->opt.hot_ny < c->ny - tp.hot_y0 ? c->opt.hot_ny : c->ny - tp.hot_y0;
+  }
   tp.refill_min = c->opt.refill_min > 0 ? c->opt.refill_min : 4;
 
   char* s = c->scratch.as<char>();
@@ -737,7 +748,7 @@ static TrackParams make_params(nt_ctx* c, double dt) {
 // Persistent grid of the history kernel: SMs x resident CTAs (ctas_per_sm caps it).
 static int history_grid(nt_ctx* c, bool det) {
   int per_sm = history_max_ctas_per_sm(det, c->dens_fmt, c->tiled != 0, c->blk_n > 0,
-                                       c->opt.ctas_per_sm);
+                                       c->opt.ctas_per_sm, c->opt.tally_mode);
   if (per_sm < 1) per_sm = 1;
   if (c->opt.ctas_per_sm > 0 && c->opt.ctas_per_sm < per_sm) per_sm = c->opt.ctas_per_sm;
   return c->sm_count * per_sm;
@@ -778,10 +789,20 @@ static nt_status det_snapshot(nt_ctx* c, int64_t lo, int64_t nb, bool restore) {
 // to fill the GPU, so the third launch is one long latency-bound tail; profiles/ab.)
 // scratch [0, 8): phase-1 counter, [16, 24): parking queue length, [32, 40): phase-2
 // counter, [40, 48): emigrant count, [64, 72): arrivals count.
-static nt_status track_phases(nt_ctx* c, const TrackParams& bp, bool det, uint32_t& launches,
+static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uint32_t& launches,
                               const unsigned long long* src_count, bool slab) {
   NvtxRange nvtx_("history phases");
   char* s = c->scratch.as<char>();
+  TrackParams bp = bp_in;
+  // particle_layout 1 (AoS ablation): the kernels work on 128 B records, copied from and back
+  // to the structure-of-arrays store around the phases (production, default kernel only)
+  const bool aos = c->opt.particle_layout == 1 && !det && !slab;
+  if (aos) {
+    NT_CUDA(c, c->aos.ensure((size_t)(c->n_local > 0 ? c->n_local : 1) * sizeof(ParticleAoS)));
+    bp.aos = c->aos.as<ParticleAoS>();
+    launch_aos_copy(c->p, bp.aos, c->n_local, true, c->stream);
+    ++launches;
+  }
   unsigned long long* qlen = reinterpret_cast<unsigned long long*>(s + 16);
   NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 24, c->stream));
   const int grid = history_grid(c, det);
@@ -809,6 +830,10 @@ static nt_status track_phases(nt_ctx* c, const TrackParams& bp, bool det, uint32
     }
     launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, slab,
                    c->stream);
+    ++launches;
+  }
+  if (aos) {
+    launch_aos_copy(c->p, bp.aos, c->n_local, false, c->stream);
     ++launches;
   }
   NT_CUDA(c, cudaGetLastError());

@@ -31,6 +31,18 @@ struct Soa {
   int64_t *gid;                // global id (RNG key); = first_id + local index unless slabs
 };
 
+// Array-of-structures particle record (the particle_layout 1 ablation, §VI-D: the
+// paper measured SoA vs AoS on CPUs only; on its GPU it used SoA).  Same fields as Soa
+// (without the global id), 128 B per particle.
+struct ParticleAoS {
+  double x, y, ox, oy, e, w, mfp, dep, dcen, acc, dstep;
+  int32_t cx, cy;
+  uint32_t ctr, nfac, ncol, ncen, nf_s, nc_s, seq_s;
+  uint8_t status;
+  uint8_t pad[3];
+};
+static_assert(sizeof(ParticleAoS) == 128, "AoS record size");
+
 // A particle migrating between x-slabs (decomposition 1): its store fields plus the
 // mid-step state of a parked particle.
 struct SlabRec {

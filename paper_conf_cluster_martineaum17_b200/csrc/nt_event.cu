@@ -45,17 +45,27 @@ constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many sl
 #ifndef NT_EV_EDGE_DIV
 #define NT_EV_EDGE_DIV 0
 #endif
+// Per-type queue of a warp (A/B option): 0 lane-paired -- lane k owns slots k and k+32 and
+// the events of a type run in at most two rounds (round 1: one event of every lane that has
+// one, round 2: the second of lanes that have two), so a round touches slots k or k+32 only
+// and its 8-byte column accesses are bank-conflict free; 1 compacted per slot half with
+// ballot + popc ranks (any lane may handle any slot of the half).
+#ifndef NT_EV_COMPACT
+#define NT_EV_COMPACT 0
+#endif
 
 // Type byte of a slot: bits 0-2 the next event (or free / birth), bit 3 the facet crosses
 // an X edge, bit 4 the slot's deposit accumulator is non-zero (it is zero after every
 // flush, so most events neither load nor store it).
+// bit 5: the current cell's block (of the block map) is uniform, so a facet that stays in
+// the block keeps the stored number density (every cell of the block has it).
 enum : uint32_t { T_COLL = 0, T_FACET = 1, T_CENSUS = 2, T_BIRTH = 3, T_FREE = 4, T_AXBIT = 8,
-                  T_ACCBIT = 16 };
+                  T_ACCBIT = 16, T_UNIBIT = 32 };
 
 // 8-byte slot columns (three of them pack two i32 fields) and one 4-byte column
 enum Col8 : int {
   C_X = 0, C_Y, C_OX, C_OY, C_IOX, C_IOY, C_EXN, C_EYN, C_MFP, C_DCEN, C_ACC, C_DSTEP,
-  C_W, C_E, C_ST, C_H, C_PA, C_ND, C_D, C_CXY, C_NFC, C_CTRSEQ, kCol8
+  C_W, C_E, C_ST, C_H, C_PA, C_ND, C_CXY, C_NFC, C_CTRSEQ, kCol8
 };
 
 constexpr size_t kSmemCols = (size_t)kSlots * (kCol8 * 8 + 4);
@@ -87,6 +97,7 @@ struct St {
   double x, y, ox, oy, iox, ioy, exn, eyn, mfp, dcen, acc, dstep, w, e, st, H, nd;
   int32_t cx, cy;
   uint32_t nf, nc, ctr;
+  uint32_t uni;             // T_UNIBIT when the cell's block is uniform
 };
 
 template <bool kDet, int kFmt, bool kBlk>
@@ -128,12 +139,20 @@ struct EvKernel {
 #endif
   }
 
-  // number density of cell (cx, cy)
-  __device__ double nd_of(int32_t cx, int32_t cy) {
+  // number density of cell (cx, cy); uni: its block is uniform (block map)
+  __device__ double nd_of(int32_t cx, int32_t cy, bool& uni) {
     const uint32_t ci = cidx(cx, cy);
-    if constexpr (kBlk) return s_nd[dens_load_blk(P.mesh, s_blk, cx, cy, ci, pol)];
-    else if constexpr (kFmt == kDensU8) return s_nd[ldg_u8_hint(P.mesh.rho8 + ci, pol)];
-    else return number_density<kFmt>(P.mesh, P.mesh.nd_tab, ci, ph.cn);
+    uni = false;
+    if constexpr (kBlk) {
+      uint32_t code = s_blk[(cy >> P.mesh.bshift) * P.mesh.nbx + (cx >> P.mesh.bshift)];
+      uni = code != kBlkMixed;
+      if (!uni) code = ldg_u8_hint(P.mesh.rho8 + ci, pol);
+      return s_nd[code];
+    } else if constexpr (kFmt == kDensU8) {
+      return s_nd[ldg_u8_hint(P.mesh.rho8 + ci, pol)];
+    } else {
+      return number_density<kFmt>(P.mesh, P.mesh.nd_tab, ci, ph.cn);
+    }
   }
 
   // the flush of DESIGN.md §3: production RED or deterministic record
@@ -195,8 +214,10 @@ struct EvKernel {
   }
 
   // calculate_time_to_events + determine_next_event (Listing 2) from the
-  // state in registers: the distance goes to the slot, the type bits are returned.  Same
-  // expressions as the history kernel (R28 clamps).
+  // state in registers: the type bits are returned (the handler re-derives the event's
+  // distance from the state it loads anyway -- the same expressions, so the same value --
+  // instead of a stored distance column).  Same expressions as the history kernel
+  // (R28 clamps).
   __device__ uint32_t classify(int s, const St& v) {
     const double sig = v.nd * v.st;
     const double tx = (v.exn - v.x) * v.iox;
@@ -205,23 +226,16 @@ struct EvKernel {
     double df = ax ? tx : ty;
     df = df < 0.0 ? 0.0 : df;
     const double ds = v.dcen;
-    const uint32_t accb = v.acc != 0.0 ? T_ACCBIT : 0u;
+    const uint32_t accb = (v.acc != 0.0 ? T_ACCBIT : 0u) | v.uni;
     // n_mfp / Sigma_t only when a collision is possible (the history kernel's screen)
     const double dmin = df < ds ? df : ds;
     const double dsig = dmin * sig;
     const bool maybe_coll = !(v.mfp > dsig * 0x1.00001p+0) || dsig < 0x1p-960;
     if (maybe_coll && sig > 0.0) {
       const double dc = v.mfp / sig;
-      if (dc < df && dc < ds) {
-        d(C_D, s) = dc;
-        return T_COLL | accb;
-      }
+      if (dc < df && dc < ds) return T_COLL | accb;
     }
-    if (df < ds) {
-      d(C_D, s) = df;
-      return T_FACET | (ax ? T_AXBIT : 0u) | accb;
-    }
-    d(C_D, s) = ds;
+    if (df < ds) return T_FACET | (ax ? T_AXBIT : 0u) | accb;
     return T_CENSUS | accb;
   }
 
@@ -238,10 +252,12 @@ struct EvKernel {
     v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
     v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.e = d(C_E, s); v.st = d(C_ST, s); v.H = d(C_H, s);
     v.nd = d(C_ND, s);
+    v.uni = ty & T_UNIBIT;
     load_nfc(s, v);
     v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
-    const double dd = d(C_D, s), pa = d(C_PA, s);
+    const double pa = d(C_PA, s);
     const double sig = v.nd * v.st;
+    const double dd = v.mfp / sig;               // the collision distance classify compared
     v.nc += 1u;
     v.acc += ((v.w * dd) * sig) * v.H;
     v.x = v.x + dd * v.ox;
@@ -338,8 +354,10 @@ struct EvKernel {
     v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.st = d(C_ST, s); v.H = d(C_H, s);
     v.nd = d(C_ND, s);
     load_nfc(s, v);
-    const double dd = d(C_D, s);
     const double sig = v.nd * v.st;
+    // the facet distance classify chose (axis from the type byte), clamped at 0 (R28)
+    double dd = ax ? (v.exn - v.x) * v.iox : (v.eyn - v.y) * v.ioy;
+    dd = dd < 0.0 ? 0.0 : dd;
     v.nf += 1u;
     v.acc += ((v.w * dd) * sig) * v.H;
     v.mfp = clamp0(v.mfp - dd * sig);
@@ -371,7 +389,17 @@ struct EvKernel {
     const int32_t ke = pos2 ? c2 + 1 : c2;
     if (ax) { v.cx = c2; v.exn = edge_x(ke); d(C_EXN, s) = v.exn; }
     else    { v.cy = c2; v.eyn = edge_y(ke); d(C_EYN, s) = v.eyn; }
-    v.nd = nd_of(v.cx, v.cy);                   // the new cell's density
+    // the new cell's density: unchanged when the facet stays inside a uniform
+    // block of the block map (a reflection keeps the cell)
+    v.uni = ty & T_UNIBIT;
+    bool keep = false;
+    if constexpr (kBlk) keep = v.uni && ((c2 >> P.mesh.bshift) == (c >> P.mesh.bshift));
+    if (!keep) {
+      bool u;
+      v.nd = nd_of(v.cx, v.cy, u);
+      v.uni = u ? T_UNIBIT : 0u;
+      d(C_ND, s) = v.nd;
+    }
     i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);
     if ((int64_t)(v.nf + v.nc) >= P.max_events) {
       v.e = d(C_E, s);
@@ -386,7 +414,6 @@ struct EvKernel {
     d(C_MFP, s) = v.mfp;
     d(C_DCEN, s) = v.dcen;
     d(C_DSTEP, s) = v.dstep;
-    d(C_ND, s) = v.nd;
     i2(C_CXY, s) = make_int2(v.cx, v.cy);
     return classify(s, v);                      // acc == 0 after the flush
   }
@@ -399,7 +426,7 @@ struct EvKernel {
     v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.e = d(C_E, s);
     load_nfc(s, v);
     v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
-    const double dd = d(C_D, s);
+    const double dd = d(C_DCEN, s);              // census: the remaining census distance
     const double sig = d(C_ND, s) * d(C_ST, s);
     v.acc += ((v.w * dd) * sig) * d(C_H, s);
     v.x = d(C_X, s) + dd * v.ox;
@@ -434,7 +461,9 @@ struct EvKernel {
     v.mfp = P.p.mfp[pi]; v.dcen = speed(v.e, ph) * P.dt;
     v.acc = 0.0; v.dstep = 0.0;
     v.w = P.p.w[pi]; v.st = m.st; v.H = m.H;
-    v.nd = nd_of(v.cx, v.cy);
+    bool u;
+    v.nd = nd_of(v.cx, v.cy, u);
+    v.uni = u ? T_UNIBIT : 0u;
     v.nf = 0u; v.nc = 0u;
     v.ctr = P.p.ctr[pi];
     cnt(SU_ALIVE, 1u);
@@ -514,12 +543,10 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
       continue;
     }
     // ---- Listing 2: all collisions, then all facets, then all census, then the births ----
-    // Each type's queue is compacted per slot half (slots sb + lane, then sb + 32 + lane): a
-    // half's 32 slots lie in distinct 4-byte banks pairwise, so the handlers' 8-byte column
-    // accesses of any subset of them take the minimum two shared-memory wavefronts (a queue
-    // drawn from all 64 slots would put up to four lanes on one bank pair).
     // the event types present in the warp's slots (one REDUX): absent types cost nothing
     const unsigned present = __reduce_or_sync(kFull, (1u << (ta & 7u)) | (1u << (tb & 7u)));
+#if NT_EV_COMPACT
+    // queues compacted per slot half: ballot + popc ranks, any lane may take any slot
 #pragma unroll 1
     for (uint32_t T = 0; T < 4; ++T) {
       if (!(present & (1u << T))) continue;
@@ -545,6 +572,31 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
         __syncwarp();
       }
     }
+#else
+    // lane-paired queues: lane k owns slots k and k + 32; a type's events run in at most two
+    // rounds, the second only for lanes holding two of them
+#pragma unroll 1
+    for (uint32_t T = 0; T < 4; ++T) {
+      if (!(present & (1u << T))) continue;
+      bool pa = (ta & 7u) == T, pb = (tb & 7u) == T;
+#pragma unroll 1
+      while (__any_sync(kFull, pa || pb)) {
+        if (pa || pb) {
+          const bool first = pa;
+          const int s = sb + (first ? lane : 32 + lane);
+          const uint32_t ty = first ? ta : tb;
+          uint32_t nt;
+          if (T == T_COLL) nt = K.collision(s, ty);
+          else if (T == T_FACET) nt = K.facet(s, ty);
+          else if (T == T_CENSUS) nt = K.census(s, ty);
+          else nt = K.birth(s);
+          if (first) { ta = nt; pa = false; } else { tb = nt; pb = false; }
+        }
+      }
+    }
+    s_type[sb + lane] = (uint8_t)ta;
+    s_type[sb + 32 + lane] = (uint8_t)tb;
+#endif
   }
   if (lane == 0 && iter > 0) atomicMax(&E.ctl->iter, iter);
 

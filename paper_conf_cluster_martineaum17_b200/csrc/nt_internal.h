@@ -13,6 +13,7 @@ struct TrackParams {
   Tables xs;
   Phys ph;
   Soa p;
+  ParticleAoS* aos;           // particle_layout 1: the AoS copy the history kernel works on
   int64_t n;                  // local particles
   int64_t lo, hi;             // local index range processed by this launch
   int64_t first_id;           // global id of local index 0
@@ -31,6 +32,8 @@ struct TrackParams {
   int32_t slab_lo, slab_hi;
   int32_t* out_q;             // emigrant local indices
   unsigned long long* out_count;
+  // tally_mode 3: the hot window of cells privatised in shared memory (whole-mesh columns)
+  int32_t hot_x0, hot_y0, hot_nx, hot_ny;
   unsigned long long* counter;      // dynamic work counter (particles claimed)
   unsigned long long* stats_u;      // [SU_COUNT]
   double* stats_f;                  // [SF_COUNT]
@@ -61,11 +64,14 @@ void launch_inject(const InjectParams& ip, cudaStream_t s);
 // The density format (tp.mesh.fmt) and the storage layout (tp.mesh.tiled) select the
 // instantiation; 128-thread CTAs with <= 80 registers (6 resident per SM), or -- minb = 7,
 // production u8 + block map only -- <= 72 registers (7 per SM).
-// tally_mode 1 (production u8 + block map only): warp-aggregated tally flushes.
+// tally_mode 1/2/3 (production u8 + block map only): warp-aggregated flushes / CAS-emulated
+// fp64 add / shared-memory hot window (tp.hot_*).
 // xs_search 2 (u8 + block map only): the cached-bin linear walk; 1 is a data change (the
 // caller passes tables without bucket index, nb = 0).
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
                     int xs_search, bool slab, cudaStream_t s);
+// particle_layout 1: copy the particle store SoA -> AoS (to_aos) or back, particles [0, n)
+void launch_aos_copy(const Soa& p, ParticleAoS* aos, int64_t n, bool to_aos, cudaStream_t s);
 // Slab decomposition: pack the emigrants (out_q[0, n)) into records, those left of slab_lo
 // first (counter cnt[0]), the others from the end (cnt[1]); unpack n records into the slots
 // free_slots[0, n_free) and then [base, ...), status 2, and queue them in arr_q.
@@ -73,7 +79,7 @@ void launch_slab_pack(const TrackParams& tp, const int32_t* out_q, int64_t n, Sl
                       unsigned long long* cnt, cudaStream_t s);
 void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32_t* free_slots,
                         int64_t n_free, int64_t base, int32_t* arr_q, cudaStream_t s);
-int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb);
+int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);
 void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s);
@@ -93,6 +99,7 @@ void launch_stats_to_f64(const unsigned long long* su, const double* sf, double*
                          cudaStream_t s);
 
 constexpr int kHistoryBlock = 128;
+constexpr int kHotCells = 2048;     // tally_mode 3: cells of the shared-memory hot window (16 KB)
 // history kernel: events a lane may run between two warp votes (refill checks); the A/B
 // sweep in profiles/ab/r01_ab4_history_variants.md chose 256
 constexpr int kInnerEvents = 256;   // (also best for the parked-particle phase: ab9, ab10)

@@ -80,13 +80,22 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 //
 // kDet = true: instead of the RED, every flush is written as a (cell, particle, sequence)
 // keyed record; the host sorts the records and applies them in the oracle's order.
-template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, bool kAgg, bool kXsWalk,
-          bool kVar, bool kSlab>
+// kTally (production flushes, tally_mode): 0 one fp64 RED per flush; 1 warp-aggregated;
+// 2 the fp64 add emulated with a 64-bit compare-and-swap loop (how fp64 atomics were done
+// before native ones); 3 a per-CTA shared-memory copy of a hot window of cells
+// (privatisation), merged into the tally with one RED per cell at the end.
+template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, int kTally, bool kXsWalk,
+          bool kVar, bool kSlab, bool kAoS = false>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
+  // particle-store field f of local particle idx: structure of arrays, or -- the
+  // AoS ablation (particle_layout 1) -- one 128 B record per particle
+#define PP(f, idx) (kAoS ? &P.aos[idx].f : P.p.f + (idx))
   static_assert(!(kSlab && kDet), "slab decomposition: production tally only");
   static_assert(!kBlk || kFmt == kDensU8, "the block map indexes u8 material codes");
-  static_assert(!(kAgg && kDet), "aggregation reorders the sum: production tally only");
+  static_assert(!(kTally && kDet), "tally modes reorder the sum: production tally only");
+  static_assert(!(kTally == 3 && kSlab), "hot window: replicated meshes only");
+  static_assert(!(kAoS && kSlab), "AoS particle store: replicated meshes only");
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
   // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
   // almost no shared memory and the L1 stays free for the density / edge gathers.
@@ -95,6 +104,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
   __shared__ __align__(16) uint8_t s_blk[kBlk ? kBlkMax : 1];
   __shared__ double s_wabs[kHistoryBlock];   // weight absorbed by implicit capture, per thread
+  __shared__ double s_hot[kTally == 3 ? kHotCells : 1];   // privatised hot window (kTally 3)
   const int t = threadIdx.x;
   const int64_t gt = (int64_t)blockIdx.x * kHistoryBlock + t;
   const int64_t sstride = (int64_t)gridDim.x * kHistoryBlock;
@@ -102,6 +112,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
 #pragma unroll
   for (int k = 0; k < SF_COUNT; ++k) sf[k * sstride] = 0.0;
   if (t < kWarps * SU_COUNT) (&s_u[0][0])[t] = 0u;
+  if constexpr (kTally == 3)
+    for (int k = t; k < kHotCells; k += kHistoryBlock) s_hot[k] = 0.0;
   __syncthreads();
   if constexpr (kFmt == kDensU8) {
     for (int k = t; k < 256; k += kHistoryBlock) s_nd[k] = k < P.mesh.ncodes ? P.mesh.nd_tab[k] : 0.0;
@@ -144,10 +156,21 @@ history_kernel(const __grid_constant__ TrackParams P) {
     if constexpr (kSlab) return (uint64_t)__ldg(P.p.gid + i_);
     else return (uint64_t)(P.first_id + i_);
   };
-  // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather
+  // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather.  With the block
+  // map, uni_ records whether the cell's block is uniform: a facet that stays inside a
+  // uniform block (31 of 32 crossings for 32-cell blocks) keeps the code it has -- every cell
+  // of the block has it -- and needs no lookup at all.
+  bool buni = false;             // the current cell's block is uniform (kBlk)
   auto dload = [&](int32_t cx_, int32_t cy_, uint32_t ci_) {
-    if constexpr (kBlk) return dens_load_blk<kSlab>(P.mesh, s_blk, cx_, cy_, ci_, pol_keep);
-    else return dens_load<kFmt>(P.mesh, ci_, pol_keep);
+    if constexpr (kBlk) {
+      const int32_t lx = kSlab ? cx_ - P.mesh.x0 : cx_;
+      uint32_t code = s_blk[(cy_ >> P.mesh.bshift) * P.mesh.nbx + (lx >> P.mesh.bshift)];
+      buni = code != kBlkMixed;
+      if (!buni) code = ldg_u8_hint(P.mesh.rho8 + ci_, pol_keep);
+      return code;
+    } else {
+      return dens_load<kFmt>(P.mesh, ci_, pol_keep);
+    }
   };
 
   bool active = false, exhausted = false;
@@ -186,23 +209,23 @@ history_kernel(const __grid_constant__ TrackParams P) {
   // takes a new particle.  Used for regime parking (status 2, park_q) and, with x-slabs,
   // for emigrants (status 4, out_q).
   auto park_to = [&](uint8_t st, int32_t* q, unsigned long long* qn) {
-    P.p.x[i] = x;
-    P.p.y[i] = y;
-    P.p.ox[i] = ox;
-    P.p.oy[i] = oy;
-    P.p.e[i] = e;
-    P.p.w[i] = w;
-    P.p.mfp[i] = mfp;
-    P.p.cx[i] = cx;
-    P.p.cy[i] = cy;
-    P.p.ctr[i] = ctr;
-    P.p.dcen[i] = dcen;
-    P.p.acc[i] = acc;
-    P.p.dstep[i] = dstep;
-    P.p.nf_s[i] = nf;
-    P.p.nc_s[i] = nc;
-    if constexpr (kDet) P.p.seq_s[i] = seq;
-    P.p.status[i] = st;
+    (*PP(x, i)) = x;
+    (*PP(y, i)) = y;
+    (*PP(ox, i)) = ox;
+    (*PP(oy, i)) = oy;
+    (*PP(e, i)) = e;
+    (*PP(w, i)) = w;
+    (*PP(mfp, i)) = mfp;
+    (*PP(cx, i)) = cx;
+    (*PP(cy, i)) = cy;
+    (*PP(ctr, i)) = ctr;
+    (*PP(dcen, i)) = dcen;
+    (*PP(acc, i)) = acc;
+    (*PP(dstep, i)) = dstep;
+    (*PP(nf_s, i)) = nf;
+    (*PP(nc_s, i)) = nc;
+    if constexpr (kDet) (*PP(seq_s, i)) = seq;
+    (*PP(status, i)) = st;
     const unsigned am = __activemask();
     const int ld = __ffs(am) - 1;
     unsigned long long k = 0;
@@ -228,18 +251,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
         if (my < span2) {
           i = resume ? P.resume_q[my] : (int32_t)(P.lo + (int64_t)my);
-          if (P.p.status[i] == (resume ? 2u : 1u)) {
+          if ((*PP(status, i)) == (resume ? 2u : 1u)) {
             active = true;
-            x = ld_stream(P.p.x + i, pol_stream);
-            y = ld_stream(P.p.y + i, pol_stream);
-            ox = ld_stream(P.p.ox + i, pol_stream);
-            oy = ld_stream(P.p.oy + i, pol_stream);
-            e = ld_stream(P.p.e + i, pol_stream);
-            w = ld_stream(P.p.w + i, pol_stream);
-            mfp = ld_stream(P.p.mfp + i, pol_stream);
-            cx = ld_stream(P.p.cx + i, pol_stream);
-            cy = ld_stream(P.p.cy + i, pol_stream);
-            ctr = ld_stream(P.p.ctr + i, pol_stream);
+            x = ld_stream(PP(x, i), pol_stream);
+            y = ld_stream(PP(y, i), pol_stream);
+            ox = ld_stream(PP(ox, i), pol_stream);
+            oy = ld_stream(PP(oy, i), pol_stream);
+            e = ld_stream(PP(e, i), pol_stream);
+            w = ld_stream(PP(w, i), pol_stream);
+            mfp = ld_stream(PP(mfp, i), pol_stream);
+            cx = ld_stream(PP(cx, i), pol_stream);
+            cy = ld_stream(PP(cy, i), pol_stream);
+            ctr = ld_stream(PP(ctr, i), pol_stream);
             exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
             eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
             iox = 1.0 / ox;
@@ -262,12 +285,12 @@ history_kernel(const __grid_constant__ TrackParams P) {
             } else {                 // the parked state (phase 1 counted the XS clamps)
               uint32_t nr_dummy = 0;
               m = refresh_xs(P.xs, ph, e, nr_dummy);
-              dcen = P.p.dcen[i];
-              acc = P.p.acc[i];
-              dstep = P.p.dstep[i];
-              nf = P.p.nf_s[i];
-              nc = P.p.nc_s[i];
-              if constexpr (kDet) seq = P.p.seq_s[i];
+              dcen = (*PP(dcen, i));
+              acc = (*PP(acc, i));
+              dstep = (*PP(dstep, i));
+              nf = (*PP(nf_s, i));
+              nc = (*PP(nc_s, i));
+              if constexpr (kDet) seq = (*PP(seq_s, i));
             }
             // born (or resumed) outside this rank's slab: hand over before any event (and
             // before touching the density, which this rank holds for its columns only)
@@ -339,8 +362,24 @@ history_kernel(const __grid_constant__ TrackParams P) {
             }
             if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
             ++seq;
-          } else if constexpr (kAgg) {
+          } else if constexpr (kTally == 1) {
             red_add_warp(P.mesh.tally, cell, acc, pol_keep);
+          } else if constexpr (kTally == 2) {
+            // fp64 add by compare-and-swap on the 64-bit word (retried while another thread
+            // changed the cell in between)
+            unsigned long long* a = reinterpret_cast<unsigned long long*>(P.mesh.tally + cell);
+            unsigned long long old = *a, assumed;
+            do {
+              assumed = old;
+              old = atomicCAS(a, assumed,
+                              (unsigned long long)__double_as_longlong(__longlong_as_double((long long)assumed) + acc));
+            } while (assumed != old);
+          } else if constexpr (kTally == 3) {
+            const uint32_t hx = (uint32_t)(cx - P.hot_x0), hy = (uint32_t)(cy - P.hot_y0);
+            if (hx < (uint32_t)P.hot_nx && hy < (uint32_t)P.hot_ny)
+              atomicAdd(&s_hot[hy * (uint32_t)P.hot_nx + hx], acc);     // shared-memory atomic
+            else
+              red_add_hint(P.mesh.tally + cell, acc, pol_keep);
           } else {
             red_add_hint(P.mesh.tally + cell, acc, pol_keep);   // fire-and-forget fp64 RED at L2
           }
@@ -471,7 +510,18 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const int32_t ke = pos2 ? c2 + 1 : c2;
           if (ax) exn = __ldg(ex + ke); else eyn = __ldg(ey + ke);
           cidx = cidx_of(cx, cy);
-          draw = dload(cx, cy, cidx);                 // new cell's density
+          // new cell's density; unchanged inside a uniform block (a reflection
+          // keeps the cell, c2 == c)
+#ifndef NT_BLK_SKIP
+#define NT_BLK_SKIP 0
+#endif
+          if constexpr (kBlk && NT_BLK_SKIP) {
+            const int32_t o = (kSlab && ax) ? x0 : 0;
+            const bool same = ((c2 - o) >> P.mesh.bshift) == ((c - o) >> P.mesh.bshift);
+            if (!(same && buni)) draw = dload(cx, cy, cidx);
+          } else {
+            draw = dload(cx, cy, cidx);
+          }
           nf += 1u;
           if constexpr (kSlab) {
             // entered the neighbour's slab: the facet is done, the neighbour continues
@@ -494,24 +544,24 @@ history_kernel(const __grid_constant__ TrackParams P) {
         if (outcome != 0) {
           if (!(isfinite(x) && isfinite(y) && isfinite(e) && isfinite(w)))
             cnt(SU_NONFINITE, 1u);
-          st_stream(P.p.x + i, x, pol_stream);
-          st_stream(P.p.y + i, y, pol_stream);
-          st_stream(P.p.ox + i, ox, pol_stream);
-          st_stream(P.p.oy + i, oy, pol_stream);
-          st_stream(P.p.e + i, e, pol_stream);
-          st_stream(P.p.w + i, w, pol_stream);
-          st_stream(P.p.mfp + i, mfp, pol_stream);
-          st_stream(P.p.dep + i, ld_stream(P.p.dep + i, pol_stream) + dstep, pol_stream);
-          st_stream(P.p.cx + i, cx, pol_stream);
-          st_stream(P.p.cy + i, cy, pol_stream);
-          st_stream(P.p.ctr + i, ctr, pol_stream);
-          st_stream(P.p.nfac + i, ld_stream(P.p.nfac + i, pol_stream) + nf, pol_stream);
-          st_stream(P.p.ncol + i, ld_stream(P.p.ncol + i, pol_stream) + nc, pol_stream);
+          st_stream(PP(x, i), x, pol_stream);
+          st_stream(PP(y, i), y, pol_stream);
+          st_stream(PP(ox, i), ox, pol_stream);
+          st_stream(PP(oy, i), oy, pol_stream);
+          st_stream(PP(e, i), e, pol_stream);
+          st_stream(PP(w, i), w, pol_stream);
+          st_stream(PP(mfp, i), mfp, pol_stream);
+          st_stream(PP(dep, i), ld_stream(PP(dep, i), pol_stream) + dstep, pol_stream);
+          st_stream(PP(cx, i), cx, pol_stream);
+          st_stream(PP(cy, i), cy, pol_stream);
+          st_stream(PP(ctr, i), ctr, pol_stream);
+          st_stream(PP(nfac, i), ld_stream(PP(nfac, i), pol_stream) + nf, pol_stream);
+          st_stream(PP(ncol, i), ld_stream(PP(ncol, i), pol_stream) + nc, pol_stream);
           if (outcome == 1) {
-            P.p.ncen[i] += 1u;
-            if (resume) P.p.status[i] = 1u;           // was parked (2)
+            (*PP(ncen, i)) += 1u;
+            if (resume) (*PP(status, i)) = 1u;           // was parked (2)
           } else {
-            P.p.status[i] = 0u;
+            (*PP(status, i)) = 0u;
           }
           cnt(SU_FACETS, nf);
           cnt(SU_COLLISIONS, nc);
@@ -550,6 +600,15 @@ history_kernel(const __grid_constant__ TrackParams P) {
   // ---- CTA reduction of the statistics, one atomic per statistic per CTA ----
   fsum(SF_ABSORBED_W, s_wabs[t]);
   __syncthreads();
+  if constexpr (kTally == 3) {        // merge the privatised window: one RED per touched cell
+    for (int k = t; k < P.hot_nx * P.hot_ny; k += kHistoryBlock) {
+      const double v = s_hot[k];
+      if (v != 0.0) {
+        const int32_t hx = k % P.hot_nx, hy = k / P.hot_nx;
+        red_add_hint(P.mesh.tally + cidx_of(P.hot_x0 + hx, P.hot_y0 + hy), v, pol_keep);
+      }
+    }
+  }
   const int lane2 = t & 31;
   for (int k = wid; k < SU_COUNT + SF_COUNT; k += kWarps) {
     if (k < SU_COUNT) {
@@ -569,6 +628,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
   }
 }
 
+#undef PP
+
 // Instantiations: deterministic/production x density format x layout x block map x physics
 // variants (kVar: the code paths of DESIGN.md R30-R32, compiled only into the kernels used
 // when a variant is switched on, so the default kernels carry none of it); the u8 +
@@ -579,59 +640,63 @@ history_kernel(const __grid_constant__ TrackParams P) {
 #define NT_HIST_MINB 6   // resident CTAs per SM the default kernel is compiled for (A/B ab11)
 #endif
 template <bool kDet, bool kTiled, bool kVar>
-static void* history_fn(int fmt, bool blk, int minb, int agg, int xs) {
+static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos) {
   if (fmt == kDensU8) {
-    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, false, false, kVar, false>;
+    if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, 0, false, kVar, false>;
     if constexpr (!kVar) {
-      if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, false, true, false, false>;
+      if (aos) return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, 0, false, false, false, true>;
+      if (xs == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 0, true, false, false>;
       if constexpr (!kDet) {
-        if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, false, false, false, false>;
-        if (agg) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, true, false, false, false>;
+        if (minb >= 7) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 7, 0, false, false, false>;
+        if (tally == 1) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 1, false, false, false>;
+        if (tally == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 2, false, false, false>;
+        if (tally == 3) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 3, false, false, false>;
       }
     }
-    return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, false, false, kVar, false>;
+    return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, 0, false, kVar, false>;
   }
-  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, false, false, kVar, false>;
-  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, false, false, kVar, false>;
+  if (fmt == kDensU16) return (void*)history_kernel<kDet, kDensU16, kTiled, false, 6, 0, false, kVar, false>;
+  return (void*)history_kernel<kDet, kDensF64, kTiled, false, 6, 0, false, kVar, false>;
 }
 
 // x-slab decomposition kernels: production tally, physics variants compiled in.
 template <bool kTiled>
 static void* history_slab_fn(int fmt, bool blk) {
   if (fmt == kDensU8)
-    return blk ? (void*)history_kernel<false, kDensU8, kTiled, true, 6, false, false, true, true>
-               : (void*)history_kernel<false, kDensU8, kTiled, false, 6, false, false, true, true>;
-  if (fmt == kDensU16) return (void*)history_kernel<false, kDensU16, kTiled, false, 6, false, false, true, true>;
-  return (void*)history_kernel<false, kDensF64, kTiled, false, 6, false, false, true, true>;
+    return blk ? (void*)history_kernel<false, kDensU8, kTiled, true, 6, 0, false, true, true>
+               : (void*)history_kernel<false, kDensU8, kTiled, false, 6, 0, false, true, true>;
+  if (fmt == kDensU16) return (void*)history_kernel<false, kDensU16, kTiled, false, 6, 0, false, true, true>;
+  return (void*)history_kernel<false, kDensF64, kTiled, false, 6, 0, false, true, true>;
 }
 
 template <bool kVar>
-static void* history_select_v(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs) {
-  if (det) return tiled ? history_fn<true, true, kVar>(fmt, blk, minb, agg, xs)
-                        : history_fn<true, false, kVar>(fmt, blk, minb, agg, xs);
-  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, agg, xs)
-               : history_fn<false, false, kVar>(fmt, blk, minb, agg, xs);
+static void* history_select_v(bool det, int fmt, bool tiled, bool blk, int minb, int tally, int xs,
+                              bool aos) {
+  if (det) return tiled ? history_fn<true, true, kVar>(fmt, blk, minb, tally, xs, aos)
+                        : history_fn<true, false, kVar>(fmt, blk, minb, tally, xs, aos);
+  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, tally, xs, aos)
+               : history_fn<false, false, kVar>(fmt, blk, minb, tally, xs, aos);
 }
 
-static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int agg, int xs,
-                            bool var, bool slab = false) {
+static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int tally, int xs,
+                            bool var, bool slab = false, bool aos = false) {
   if (slab) return tiled ? history_slab_fn<true>(fmt, blk) : history_slab_fn<false>(fmt, blk);
-  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, agg, xs)
-             : history_select_v<false>(det, fmt, tiled, blk, minb, agg, xs);
+  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, tally, xs, false)
+             : history_select_v<false>(det, fmt, tiled, blk, minb, tally, xs, aos);
 }
 
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
                     int xs_search, bool slab, cudaStream_t s) {
   const bool var = tp.ph.vacuum || tp.ph.analog || tp.ph.roulette;
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode, xs_search, var, slab);
+                            tally_mode, xs_search, var, slab, tp.aos != nullptr);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }
 
-int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb) {
+int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally) {
   int n = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, 0, 0, false),
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&n, history_select(det, fmt, tiled, blk, minb, tally, 0, false),
                                                 kHistoryBlock, 0);
   return n;
 }
@@ -682,7 +747,9 @@ __global__ void slab_pack_kernel(const __grid_constant__ TrackParams P, const in
   r.e = P.p.e[i]; r.w = P.p.w[i]; r.mfp = P.p.mfp[i];
   r.dcen = P.p.dcen[i]; r.acc = P.p.acc[i]; r.dstep = P.p.dstep[i]; r.dep = P.p.dep[i];
   r.cx = P.p.cx[i]; r.cy = P.p.cy[i]; r.ctr = P.p.ctr[i];
-  r.nf = P.p.nf_s[i]; r.nc = P.p.nc_s[i]; r.seq = P.p.seq_s[i];
+  // (x-slabs run the production tally only: the flush sequence is not kept -- compute-
+  // sanitizer initcheck flagged the read of the never-written column)
+  r.nf = P.p.nf_s[i]; r.nc = P.p.nc_s[i]; r.seq = 0u;
   r.nfac = P.p.nfac[i]; r.ncol = P.p.ncol[i]; r.ncen = P.p.ncen[i]; r.pad = 0u;
 }
 
@@ -715,6 +782,28 @@ void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32
   if (n <= 0) return;
   slab_unpack_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(p, src, n, free_slots, n_free,
                                                                   base, arr_q);
+}
+
+// ---------------------------------------------------------------------------------------
+// particle_layout 1 (AoS ablation): the particle store into 128 B records and back.
+__global__ void aos_copy_kernel(const Soa p, ParticleAoS* __restrict__ a, int64_t n, int to_aos) {
+  const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (i >= n) return;
+  ParticleAoS& r = a[i];
+  if (to_aos) {
+    r.x = p.x[i]; r.y = p.y[i]; r.ox = p.ox[i]; r.oy = p.oy[i]; r.e = p.e[i]; r.w = p.w[i];
+    r.mfp = p.mfp[i]; r.dep = p.dep[i]; r.cx = p.cx[i]; r.cy = p.cy[i]; r.ctr = p.ctr[i];
+    r.nfac = p.nfac[i]; r.ncol = p.ncol[i]; r.ncen = p.ncen[i]; r.status = p.status[i];
+  } else {
+    p.x[i] = r.x; p.y[i] = r.y; p.ox[i] = r.ox; p.oy[i] = r.oy; p.e[i] = r.e; p.w[i] = r.w;
+    p.mfp[i] = r.mfp; p.dep[i] = r.dep; p.cx[i] = r.cx; p.cy[i] = r.cy; p.ctr[i] = r.ctr;
+    p.nfac[i] = r.nfac; p.ncol[i] = r.ncol; p.ncen[i] = r.ncen; p.status[i] = r.status;
+  }
+}
+
+void launch_aos_copy(const Soa& p, ParticleAoS* aos, int64_t n, bool to_aos, cudaStream_t s) {
+  if (n <= 0) return;
+  aos_copy_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(p, aos, n, to_aos ? 1 : 0);
 }
 
 // ---------------------------------------------------------------------------------------

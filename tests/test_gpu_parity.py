@@ -138,12 +138,38 @@ def test_parity_production_atomic(nt, orc, cfgname, mode, density_format, layout
     compare_stats(gs, os_, rtol=1e-9)
 
 
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "small_csp", "small_scatter", "tiny_split", "tiny_mosaic"])
+def test_parity_aos_particle_layout(nt, orc, cfgname):
+    """particle_layout 1 (AoS records while the history kernel runs): same
+    per-particle results, tally within the production bar."""
+    cfg = wl.CONFIGS[cfgname]
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, particle_layout=1)
+    ot, op, (os_,) = orc.run(cfg)
+    compare_particles(gp, op)
+    compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+    compare_stats(gs, os_, rtol=1e-9)
+
+
+def hot_window(cfg, margin=2, cells=2048):
+    """The cells around the source rectangle (tally_mode 3's privatised window)."""
+    sx, sy, sw, sh = cfg.source
+    x0 = max(0, int(sx / cfg.width * cfg.nx) - margin)
+    y0 = max(0, int(sy / cfg.height * cfg.ny) - margin)
+    nx = min(cfg.nx - x0, int(math.ceil(sw / cfg.width * cfg.nx)) + 2 * margin)
+    ny = min(cfg.ny - y0, max(1, min(int(math.ceil(sh / cfg.height * cfg.ny)) + 2 * margin, cells // max(nx, 1))))
+    return (x0, y0, max(1, min(nx, cells)), ny)
+
+
+@pytest.mark.parametrize("tally_mode", [1, 2, 3])
 @pytest.mark.parametrize("mode", MODES)
 @pytest.mark.parametrize("cfgname", ["tiny_hotspot", "tiny_scatter_1g", "tiny_mosaic", "tiny_csp"])
-def test_parity_warp_aggregated_tally(nt, orc, cfgname, mode):
-    """tally_mode 1: same-cell flushes of a warp summed with shuffles, one atomic per cell."""
+def test_parity_tally_modes(nt, orc, cfgname, mode, tally_mode):
+    """Production tally ablations (history mode; event mode uses one RED per flush):
+    1 same-cell flushes of a warp summed with shuffles, one atomic per cell; 2 fp64 add by
+    compare-and-swap; 3 shared-memory privatised hot window."""
     cfg = wl.CONFIGS[cfgname]
-    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, tally_mode=1)
+    gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, mode=mode, tally_mode=tally_mode,
+                             hot_window=hot_window(cfg))
     ot, op, (os_,) = orc.run(cfg)
     compare_particles(gp, op)
     compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
