@@ -540,18 +540,14 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     while ((range >> s) >= (uint64_t)target) ++s;
     const int64_t nb = (int64_t)(range >> s) + 1;
     idx[t].resize((size_t)nb + 1);
+    // bin of each bucket's first value, max{i in [0, n-2] : k[i] <= v}: the values increase
+    // with b, so one merge-like sweep over the keys (O(nb + n)) instead of a search each
+    int64_t lo = 0;
     for (int64_t b = 0; b <= nb; ++b) {
       const uint64_t bits = b0 + ((uint64_t)b << s);
       double v;
       if (bits >= 0x7ff0000000000000ull) v = INFINITY; else std::memcpy(&v, &bits, 8);
-      // bin of v: max{i in [0, n-2] : k[i] <= v}
-      int64_t lo = 0, hi = n - 1;
-      if (v >= k[n - 1]) lo = n - 2;
-      else
-        while (hi - lo > 1) {
-          const int64_t mid = (lo + hi) / 2;
-          if (k[mid] <= v) lo = mid; else hi = mid;
-        }
+      while (lo < n - 2 && k[lo + 1] <= v) ++lo;
       idx[t][(size_t)b] = (uint32_t)lo;
     }
     base[t] = b0;

@@ -344,16 +344,37 @@ struct EvKernel {
   __device__ uint32_t facet(int s, uint32_t ty) {
     const bool ax = (ty & T_AXBIT) != 0;
     St v;
+    load_nfc(s, v);
+    v.iox = d(C_IOX, s); v.ioy = d(C_IOY, s);
+    // the cell this facet leads into, its heading edge and its density depend only on the
+    // cell and the direction: issue those loads first, so they overlap the deposit arithmetic
+    const int32_t c = ax ? v.cx : v.cy;
+    const bool pos = (ax ? v.iox : v.ioy) > 0.0;  // the crossed axis' direction (sign of 1/omega)
+    const int32_t cs = c + (pos ? 1 : -1);
+    const bool refl = (uint32_t)cs >= (uint32_t)(ax ? P.mesh.gnx : P.mesh.ny);   // (P:240-242)
+    const int32_t c2 = refl ? c : cs;
+    const int32_t ke = (refl ? !pos : pos) ? c2 + 1 : c2;
+    const double enew = ax ? edge_x(ke) : edge_y(ke);
+    const int32_t ncx = ax ? c2 : v.cx, ncy = ax ? v.cy : c2;
+    // the new cell's density (P:163-164): unchanged when the facet stays inside a uniform
+    // block of the block map (a reflection keeps the cell)
+    uint32_t uni = ty & T_UNIBIT;
+    bool keep = false;
+    if constexpr (kBlk) keep = uni && ((c2 >> P.mesh.bshift) == (c >> P.mesh.bshift));
+    double ndn = 0.0;
+    if (!keep) {
+      bool u;
+      ndn = nd_of(ncx, ncy, u);
+      uni = u ? T_UNIBIT : 0u;
+    }
     v.x = d(C_X, s); v.y = d(C_Y, s);
-    v.iox = d(C_IOX, s); v.ioy = d(C_IOY, s); v.exn = d(C_EXN, s); v.eyn = d(C_EYN, s);
-    // the direction cosine of the coordinate that moves (the other is snapped to the edge);
-    // the crossed axis' direction is the sign of its reciprocal
+    v.exn = d(C_EXN, s); v.eyn = d(C_EYN, s);
+    // the direction cosine of the coordinate that moves (the other is snapped to the edge)
     const double om = d(ax ? C_OY : C_OX, s);
     v.mfp = d(C_MFP, s); v.dcen = d(C_DCEN, s);
     v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
     v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.st = d(C_ST, s); v.H = d(C_H, s);
     v.nd = d(C_ND, s);
-    load_nfc(s, v);
     const double sig = v.nd * v.st;
     // the facet distance classify chose (axis from the type byte), clamped at 0 (R28)
     double dd = ax ? (v.exn - v.x) * v.iox : (v.eyn - v.y) * v.ioy;
@@ -366,11 +387,6 @@ struct EvKernel {
     v.x = ax ? v.exn : moved;                   // snap the crossed coordinate
     v.y = ax ? moved : v.eyn;
     flush(s, v);                                // deposit of the cell being left
-    const int32_t c = ax ? v.cx : v.cy;
-    const bool pos = (ax ? v.iox : v.ioy) > 0.0;
-    const int32_t cs = c + (pos ? 1 : -1);
-    const bool refl = (uint32_t)cs >= (uint32_t)(ax ? P.mesh.gnx : P.mesh.ny);   // (P:240-242)
-    const int32_t c2 = refl ? c : cs;
     if (refl) {
       v.ox = d(C_OX, s);
       v.oy = d(C_OY, s);
@@ -385,19 +401,13 @@ struct EvKernel {
       if (ax) { v.ox = -v.ox; v.iox = -v.iox; d(C_OX, s) = v.ox; d(C_IOX, s) = v.iox; }
       else    { v.oy = -v.oy; v.ioy = -v.ioy; d(C_OY, s) = v.oy; d(C_IOY, s) = v.ioy; }
     }
-    const bool pos2 = refl ? !pos : pos;
-    const int32_t ke = pos2 ? c2 + 1 : c2;
-    if (ax) { v.cx = c2; v.exn = edge_x(ke); d(C_EXN, s) = v.exn; }
-    else    { v.cy = c2; v.eyn = edge_y(ke); d(C_EYN, s) = v.eyn; }
-    // the new cell's density (P:163-164): unchanged when the facet stays inside a uniform
-    // block of the block map (a reflection keeps the cell)
-    v.uni = ty & T_UNIBIT;
-    bool keep = false;
-    if constexpr (kBlk) keep = v.uni && ((c2 >> P.mesh.bshift) == (c >> P.mesh.bshift));
+    v.cx = ncx;
+    v.cy = ncy;
+    if (ax) { v.exn = enew; d(C_EXN, s) = v.exn; }
+    else    { v.eyn = enew; d(C_EYN, s) = v.eyn; }
+    v.uni = uni;
     if (!keep) {
-      bool u;
-      v.nd = nd_of(v.cx, v.cy, u);
-      v.uni = u ? T_UNIBIT : 0u;
+      v.nd = ndn;
       d(C_ND, s) = v.nd;
     }
     i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);

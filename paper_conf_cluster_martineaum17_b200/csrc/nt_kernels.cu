@@ -156,17 +156,16 @@ history_kernel(const __grid_constant__ TrackParams P) {
     if constexpr (kSlab) return (uint64_t)__ldg(P.p.gid + i_);
     else return (uint64_t)(P.first_id + i_);
   };
-  // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather.  With the block
-  // map, uni_ records whether the cell's block is uniform: a facet that stays inside a
-  // uniform block (31 of 32 crossings for 32-cell blocks) keeps the code it has -- every cell
-  // of the block has it -- and needs no lookup at all.
-  bool buni = false;             // the current cell's block is uniform (kBlk)
+  // density (code) of cell (cx_, cy_) at storage index ci_: issue the gather (with the block
+  // map: the block's code from shared memory, the cell's own only in mixed blocks).  Measured
+  // and rejected in round 2 (profiles/ab/r02_ab4, r02_ab8): keeping the code while a facet
+  // stays inside a uniform block (more spills), and issuing the facet's edge and density
+  // loads before its deposit arithmetic (csp +0.5%, split +2%).
   auto dload = [&](int32_t cx_, int32_t cy_, uint32_t ci_) {
     if constexpr (kBlk) {
       const int32_t lx = kSlab ? cx_ - P.mesh.x0 : cx_;
       uint32_t code = s_blk[(cy_ >> P.mesh.bshift) * P.mesh.nbx + (lx >> P.mesh.bshift)];
-      buni = code != kBlkMixed;
-      if (!buni) code = ldg_u8_hint(P.mesh.rho8 + ci_, pol_keep);
+      if (code == kBlkMixed) code = ldg_u8_hint(P.mesh.rho8 + ci_, pol_keep);
       return code;
     } else {
       return dens_load<kFmt>(P.mesh, ci_, pol_keep);
@@ -510,18 +509,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const int32_t ke = pos2 ? c2 + 1 : c2;
           if (ax) exn = __ldg(ex + ke); else eyn = __ldg(ey + ke);
           cidx = cidx_of(cx, cy);
-          // new cell's density; unchanged inside a uniform block (a reflection
-          // keeps the cell, c2 == c)
-#ifndef NT_BLK_SKIP
-#define NT_BLK_SKIP 0
-#endif
-          if constexpr (kBlk && NT_BLK_SKIP) {
-            const int32_t o = (kSlab && ax) ? x0 : 0;
-            const bool same = ((c2 - o) >> P.mesh.bshift) == ((c - o) >> P.mesh.bshift);
-            if (!(same && buni)) draw = dload(cx, cy, cidx);
-          } else {
-            draw = dload(cx, cy, cidx);
-          }
+          draw = dload(cx, cy, cidx);                 // new cell's density
           nf += 1u;
           if constexpr (kSlab) {
             // entered the neighbour's slab: the facet is done, the neighbour continues

@@ -20,5 +20,5 @@ for spec in "$@"; do
   nvcc -gencode arch=compute_100a,code=sm_100a -shared -o $PKG/lib/variants/libneutral_b200_$name.so \
        $objs $ROOT/build/variants/nt_kernels_$name.o $ROOT/build/variants/nt_event_$name.o \
        -L$NCCL/lib -l:libnccl.so.2 -Xlinker -rpath,$NCCL/lib
-  echo "$name: $(grep -A2 'history_kernelILb0ELi2ELb1ELb1ELi6ELb0ELb0ELb0ELb0E' $ROOT/build/variants/ptxas_$name.log | sed -n 3p)"
+  echo "$name: $(grep -A2 'history_kernelILb0ELi2ELb1ELb1ELi6ELi0ELb0ELb0ELb0ELb0E' $ROOT/build/variants/ptxas_$name.log | sed -n 3p)"
 done
