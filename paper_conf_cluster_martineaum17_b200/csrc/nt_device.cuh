@@ -228,9 +228,19 @@ __device__ __forceinline__ uint64_t l2_evict_first() {
   asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));
   return p;
 }
+// The tally is never read by the tracking kernels, so the RED needs no "memory" clobber:
+// without it the compiler may schedule the particle's other loads and stores across the
+// flush (NT_RED_CLOBBER=1 restores the compiler barrier; A/B option).
+#ifndef NT_RED_CLOBBER
+#define NT_RED_CLOBBER 0
+#endif
 __device__ __forceinline__ void red_add_hint(double* a, double v, uint64_t pol) {
+#if NT_RED_CLOBBER
   asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol)
                : "memory");
+#else
+  asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol));
+#endif
 }
 // Warp-aggregated flush (tally_mode 1): the lanes executing this call that flush into the
 // same cell are grouped with __match_any_sync; the group's lowest lane adds the group's

@@ -54,6 +54,7 @@ constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many sl
 #define NT_EV_COMPACT 0
 #endif
 
+
 // Type byte of a slot: bits 0-2 the next event (or free / birth), bit 3 the facet crosses
 // an X edge, bit 4 the slot's deposit accumulator is non-zero (it is zero after every
 // flush, so most events neither load nor store it).
@@ -341,53 +342,73 @@ struct EvKernel {
   }
 
   // ---- facet ----
-  __device__ uint32_t facet(int s, uint32_t ty) {
-    const bool ax = (ty & T_AXBIT) != 0;
+  // Three stages: pre (state loads; the next cell, its heading edge and its density depend
+  // only on the cell and the direction, so those loads go first), math (deposit, timers,
+  // snap, flush -- no branch), post (reflection, stores, event cap, classification).  (A
+  // lane holding two facets handling both interleaved, for twice the ILP, was measured and
+  // rejected: csp 70.5 -> 91.2 ms, profiles/ab/r02_ab9.)
+  struct Fct {
     St v;
+    double om, enew, ndn, dd;
+    int32_t c, c2, ncx, ncy;
+    uint32_t uni;
+    bool ax, refl, keep;
+  };
+
+  __device__ void facet_pre(int s, uint32_t ty, Fct& f) {
+    St& v = f.v;
+    f.ax = (ty & T_AXBIT) != 0;
     load_nfc(s, v);
     v.iox = d(C_IOX, s); v.ioy = d(C_IOY, s);
-    // the cell this facet leads into, its heading edge and its density depend only on the
-    // cell and the direction: issue those loads first, so they overlap the deposit arithmetic
-    const int32_t c = ax ? v.cx : v.cy;
-    const bool pos = (ax ? v.iox : v.ioy) > 0.0;  // the crossed axis' direction (sign of 1/omega)
-    const int32_t cs = c + (pos ? 1 : -1);
-    const bool refl = (uint32_t)cs >= (uint32_t)(ax ? P.mesh.gnx : P.mesh.ny);
-    const int32_t c2 = refl ? c : cs;
-    const int32_t ke = (refl ? !pos : pos) ? c2 + 1 : c2;
-    const double enew = ax ? edge_x(ke) : edge_y(ke);
-    const int32_t ncx = ax ? c2 : v.cx, ncy = ax ? v.cy : c2;
+    f.c = f.ax ? v.cx : v.cy;
+    const bool pos = (f.ax ? v.iox : v.ioy) > 0.0;  // crossed axis' direction: sign of 1/omega
+    const int32_t cs = f.c + (pos ? 1 : -1);
+    f.refl = (uint32_t)cs >= (uint32_t)(f.ax ? P.mesh.gnx : P.mesh.ny);
+    f.c2 = f.refl ? f.c : cs;
+    const int32_t ke = (f.refl ? !pos : pos) ? f.c2 + 1 : f.c2;
+    f.enew = f.ax ? edge_x(ke) : edge_y(ke);
+    f.ncx = f.ax ? f.c2 : v.cx;
+    f.ncy = f.ax ? v.cy : f.c2;
     // the new cell's density: unchanged when the facet stays inside a uniform
     // block of the block map (a reflection keeps the cell)
-    uint32_t uni = ty & T_UNIBIT;
-    bool keep = false;
-    if constexpr (kBlk) keep = uni && ((c2 >> P.mesh.bshift) == (c >> P.mesh.bshift));
-    double ndn = 0.0;
-    if (!keep) {
+    f.uni = ty & T_UNIBIT;
+    f.keep = false;
+    if constexpr (kBlk) f.keep = f.uni && ((f.c2 >> P.mesh.bshift) == (f.c >> P.mesh.bshift));
+    f.ndn = 0.0;
+    if (!f.keep) {
       bool u;
-      ndn = nd_of(ncx, ncy, u);
-      uni = u ? T_UNIBIT : 0u;
+      f.ndn = nd_of(f.ncx, f.ncy, u);
+      f.uni = u ? T_UNIBIT : 0u;
     }
     v.x = d(C_X, s); v.y = d(C_Y, s);
     v.exn = d(C_EXN, s); v.eyn = d(C_EYN, s);
     // the direction cosine of the coordinate that moves (the other is snapped to the edge)
-    const double om = d(ax ? C_OY : C_OX, s);
+    f.om = d(f.ax ? C_OY : C_OX, s);
     v.mfp = d(C_MFP, s); v.dcen = d(C_DCEN, s);
     v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
     v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.st = d(C_ST, s); v.H = d(C_H, s);
     v.nd = d(C_ND, s);
+  }
+
+  __device__ void facet_math(int s, Fct& f) {
+    St& v = f.v;
     const double sig = v.nd * v.st;
     // the facet distance classify chose (axis from the type byte), clamped at 0 (R28)
-    double dd = ax ? (v.exn - v.x) * v.iox : (v.eyn - v.y) * v.ioy;
+    double dd = f.ax ? (v.exn - v.x) * v.iox : (v.eyn - v.y) * v.ioy;
     dd = dd < 0.0 ? 0.0 : dd;
     v.nf += 1u;
     v.acc += ((v.w * dd) * sig) * v.H;
     v.mfp = clamp0(v.mfp - dd * sig);
     v.dcen = v.dcen - dd;
-    const double moved = (ax ? v.y : v.x) + dd * om;
-    v.x = ax ? v.exn : moved;                   // snap the crossed coordinate
-    v.y = ax ? moved : v.eyn;
+    const double moved = (f.ax ? v.y : v.x) + dd * f.om;
+    v.x = f.ax ? v.exn : moved;                 // snap the crossed coordinate
+    v.y = f.ax ? moved : v.eyn;
     flush(s, v);                                // deposit of the cell being left
-    if (refl) {
+  }
+
+  __device__ uint32_t facet_post(int s, Fct& f) {
+    St& v = f.v;
+    if (f.refl) {
       v.ox = d(C_OX, s);
       v.oy = d(C_OY, s);
       if (ph.vacuum) {                          // vacuum boundary (R30): escape
@@ -398,16 +419,16 @@ struct EvKernel {
         fsum(SF_ESCAPED_W, v.w);
         return finish(s, v, false);
       }
-      if (ax) { v.ox = -v.ox; v.iox = -v.iox; d(C_OX, s) = v.ox; d(C_IOX, s) = v.iox; }
-      else    { v.oy = -v.oy; v.ioy = -v.ioy; d(C_OY, s) = v.oy; d(C_IOY, s) = v.ioy; }
+      if (f.ax) { v.ox = -v.ox; v.iox = -v.iox; d(C_OX, s) = v.ox; d(C_IOX, s) = v.iox; }
+      else      { v.oy = -v.oy; v.ioy = -v.ioy; d(C_OY, s) = v.oy; d(C_IOY, s) = v.ioy; }
     }
-    v.cx = ncx;
-    v.cy = ncy;
-    if (ax) { v.exn = enew; d(C_EXN, s) = v.exn; }
-    else    { v.eyn = enew; d(C_EYN, s) = v.eyn; }
-    v.uni = uni;
-    if (!keep) {
-      v.nd = ndn;
+    v.cx = f.ncx;
+    v.cy = f.ncy;
+    if (f.ax) { v.exn = f.enew; d(C_EXN, s) = v.exn; }
+    else      { v.eyn = f.enew; d(C_EYN, s) = v.eyn; }
+    v.uni = f.uni;
+    if (!f.keep) {
+      v.nd = f.ndn;
       d(C_ND, s) = v.nd;
     }
     i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);
@@ -426,6 +447,13 @@ struct EvKernel {
     d(C_DSTEP, s) = v.dstep;
     i2(C_CXY, s) = make_int2(v.cx, v.cy);
     return classify(s, v);                      // acc == 0 after the flush
+  }
+
+  __device__ uint32_t facet(int s, uint32_t ty) {
+    Fct f;
+    facet_pre(s, ty, f);
+    facet_math(s, f);
+    return facet_post(s, f);
   }
 
   // ---- census ----
@@ -589,6 +617,7 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
     for (uint32_t T = 0; T < 4; ++T) {
       if (!(present & (1u << T))) continue;
       bool pa = (ta & 7u) == T, pb = (tb & 7u) == T;
+
 #pragma unroll 1
       while (__any_sync(kFull, pa || pb)) {
         if (pa || pb) {
