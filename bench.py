@@ -194,6 +194,8 @@ def parse():
                     help="0 bucketed binary search, 1 plain binary search, 2 cached-bin linear walk")
     ap.add_argument("--table-size", type=int, default=0,
                     help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
+    ap.add_argument("--fused-consumers", type=int, default=0,
+                    help="history mode: fuse the parking phases, k consumer CTAs per SM (0: two launches)")
     ap.add_argument("--particle-layout", type=int, default=0,
                     help="0 structure of arrays (default), 1 AoS records while tracking (ablation)")
     ap.add_argument("--json-out", default=None)
@@ -339,7 +341,7 @@ def main():
                          refill_min=a.refill_min, layout=a.layout, density_format=a.density_format,
                          tally_mode=a.tally_mode, defer_below=a.defer_below,
                          xs_search=a.xs_search, hot_window=hot_window(cfg),
-                         particle_layout=a.particle_layout)
+                         particle_layout=a.particle_layout, fused_consumers=a.fused_consumers)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -445,6 +447,8 @@ def main():
             "config": {"workload": cfg.name, "mode": a.mode, "nx": cfg.nx, "ny": cfg.ny,
                        "layout": "tiled4x4" if a.layout == 0 else "row-major",
                        "particle_store": ["SoA", "AoS (ablation)"][a.particle_layout],
+                       "phases": (f"fused, {a.fused_consumers} consumer CTA(s)/SM" if a.fused_consumers
+                                  else "two launches (park, resume)"),
                        "density_format": ["codes+block map", "f64", "codes"][a.density_format],
                        "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED", "CAS-emulated fp64 add",
                                  "shared-memory hot window %s + RED" % (hot_window(cfg),)][a.tally_mode],

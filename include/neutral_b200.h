@@ -134,7 +134,12 @@ typedef struct {
     int32_t particle_layout;   /* 0: structure of arrays; 1: array of 128 B
                                   records while the history kernel runs (ablation, P:526-551;
                                   production tally, default kernel; others use 0)          */
-    int32_t reserved1;
+    int32_t fused_consumers;   /* history mode, production: 0 runs the parked collisions in
+                                  a second launch after phase 1 (the default); k > 0 fuses
+                                  both phases into one launch in which k CTAs per SM resume
+                                  parked particles while the others still run phase 1
+                                  (they join when their range is exhausted).  Results are
+                                  unchanged.  u8 block-map meshes, default kernel options */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

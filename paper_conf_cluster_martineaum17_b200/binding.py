@@ -55,7 +55,7 @@ class Options(C.Structure):
                 ("roulette", C.c_int32), ("decomposition", C.c_int32),
                 ("roulette_weight", C.c_double), ("hot_x0", C.c_int32), ("hot_y0", C.c_int32),
                 ("hot_nx", C.c_int32), ("hot_ny", C.c_int32), ("particle_layout", C.c_int32),
-                ("reserved1", C.c_int32)]
+                ("fused_consumers", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -188,7 +188,8 @@ class Tracker:
                  density_format: int = 0, layout: int = 0, tally_mode: int = 0,
                  defer_below: int = 0, xs_search: int = 0, boundary: int = 0,
                  analog: int = 0, roulette: int = 0, roulette_weight: float = 0.0,
-                 decomposition: int = 0, hot_window=(0, 0, 0, 0), particle_layout: int = 0):
+                 decomposition: int = 0, hot_window=(0, 0, 0, 0), particle_layout: int = 0,
+                 fused_consumers: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -216,6 +217,7 @@ class Tracker:
         o.decomposition = decomposition
         o.hot_x0, o.hot_y0, o.hot_nx, o.hot_ny = hot_window
         o.particle_layout = particle_layout
+        o.fused_consumers = fused_consumers
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:

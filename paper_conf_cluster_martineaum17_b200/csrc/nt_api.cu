@@ -284,6 +284,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
       opt.tally_mode > 3)
     return NT_ERR_ARG;
   if (opt.particle_layout < 0 || opt.particle_layout > 1) return NT_ERR_ARG;
+  if (opt.fused_consumers < 0 || opt.fused_consumers > 8) return NT_ERR_ARG;
   if (opt.tally_mode == 3 && (opt.hot_x0 < 0 || opt.hot_y0 < 0 || opt.hot_nx < 1 || opt.hot_ny < 1 ||
                               (int64_t)opt.hot_nx * opt.hot_ny > kHotCells))
     return NT_ERR_ARG;
@@ -784,7 +785,8 @@ static nt_status det_snapshot(nt_ctx* c, int64_t lo, int64_t nb, bool restore) {
 // particles scattered back out of dense matter -- csp 27.1 -> 27.8-29.6 ms: too few of them
 // to fill the GPU, so the third launch is one long latency-bound tail; profiles/ab.)
 // scratch [0, 8): phase-1 counter, [16, 24): parking queue length, [32, 40): phase-2
-// counter, [40, 48): emigrant count, [64, 72): arrivals count.
+// counter, [40, 48): emigrant count, [64, 72): arrivals count, [88, 96): fused-phase queue
+// positions claimed, [96, 100): fused-phase producer warps done.
 static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uint32_t& launches,
                               const unsigned long long* src_count, bool slab) {
   NvtxRange nvtx_("history phases");
@@ -802,6 +804,33 @@ static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uin
   unsigned long long* qlen = reinterpret_cast<unsigned long long*>(s + 16);
   NT_CUDA(c, cudaMemsetAsync(s + 16, 0, 24, c->stream));
   const int grid = history_grid(c, det);
+  // fused phases: one launch, consumers resume parked particles during phase 1 (the
+  // conditions mirror the kernel selection in nt_kernels.cu history_fn)
+  const bool var = c->ph.vacuum || c->ph.analog || c->ph.roulette;
+  const bool fused = c->opt.fused_consumers > 0 && !det && !slab && !src_count && !var && !aos &&
+                     c->dens_fmt == kDensU8 && c->blk_n > 0 && c->opt.tally_mode == 0 &&
+                     c->opt.xs_search != 2 && c->opt.ctas_per_sm < 7;
+  if (fused) {
+    NvtxRange nvtx2_("fused phases");
+    NT_CUDA(c, cudaMemsetAsync(c->defer_q, 0, (size_t)(c->n_local > 0 ? c->n_local : 1) * 4, c->stream));
+    NT_CUDA(c, cudaMemsetAsync(s + 88, 0, 16, c->stream));
+    TrackParams p = bp;
+    p.phase = 1;
+    p.park_q = c->defer_q;
+    p.park_count = qlen;
+    p.park_coll_below = c->opt.defer_below;
+    int coll = c->opt.fused_consumers * c->sm_count;
+    if (coll >= grid) coll = grid - 1;
+    p.coll_ctas = coll;
+    p.n_prod = (uint32_t)(grid - coll) * (uint32_t)(kHistoryBlock / 32);
+    p.park_taken = reinterpret_cast<unsigned long long*>(s + 88);
+    p.prod_done = reinterpret_cast<unsigned int*>(s + 96);
+    launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, slab,
+                   c->stream);
+    ++launches;
+    NT_CUDA(c, cudaGetLastError());
+    return NT_OK;
+  }
   for (int ph = 1; ph <= 2; ++ph) {
     TrackParams p = bp;
     p.phase = ph;

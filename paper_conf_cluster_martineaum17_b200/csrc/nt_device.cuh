@@ -330,6 +330,20 @@ __device__ __forceinline__ uint32_t dens_load_blk(const Mesh& M, const uint8_t* 
   return code;
 }
 
+// Cross-CTA hand-over within one launch (fused phases): volatile / L2-only accesses.
+__device__ __forceinline__ int32_t ld_volatile(const int32_t* p) {
+  return *reinterpret_cast<const volatile int32_t*>(p);
+}
+__device__ __forceinline__ uint32_t ld_volatile(const unsigned int* p) {
+  return *reinterpret_cast<const volatile unsigned int*>(p);
+}
+__device__ __forceinline__ unsigned long long ld_volatile(const unsigned long long* p) {
+  return *reinterpret_cast<const volatile unsigned long long*>(p);
+}
+__device__ __forceinline__ void st_volatile(int32_t* p, int32_t v) {
+  *reinterpret_cast<volatile int32_t*>(p) = v;
+}
+
 __device__ __forceinline__ void prefetch_l1(const void* p) {
   asm volatile("prefetch.global.L1 [%0];" ::"l"(p));
 }
@@ -385,19 +399,32 @@ __device__ __forceinline__ uint32_t xs_ldu(const uint32_t* p) {
 // table -- two dependent loads per lookup (the index pair, then the run).  A bucket holding
 // more keys falls back to a binary search inside it.  Same bin as a full binary search by
 // construction.
-__device__ __forceinline__ double xs_lookup(const Table& T, double e) {
+// Split in two so a caller can issue the first dependent load (the bucket's index pair)
+// early and finish the lookup later: xs_begin (bin bounds) and xs_end (pairs + lerp).
+struct XsPre {
+  double e;
   int32_t lo, hi;                             // k[lo] <= e < k[hi]
+};
+__device__ __forceinline__ XsPre xs_begin(const Table& T, double e) {
+  XsPre r;
+  r.e = e;
   if (e >= T.klast) {
-    lo = T.n - 2;
-    hi = T.n - 1;
+    r.lo = T.n - 2;
+    r.hi = T.n - 1;
   } else if (T.nb > 0) {
     const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
-    lo = (int32_t)xs_ldu(T.idx + b);
-    hi = (int32_t)xs_ldu(T.idx + b + 1) + 1;
+    r.lo = (int32_t)xs_ldu(T.idx + b);
+    r.hi = (int32_t)xs_ldu(T.idx + b + 1) + 1;
   } else {
-    lo = 0;
-    hi = T.n - 1;
+    r.lo = 0;
+    r.hi = T.n - 1;
   }
+  return r;
+}
+
+__device__ __forceinline__ double xs_end(const Table& T, XsPre r) {
+  const double e = r.e;
+  int32_t lo = r.lo, hi = r.hi;
   double k0, k1, v0, v1;
   if (hi - lo <= 2) {
     const double2 a = xs_ld2(T.kv + lo), b = xs_ld2(T.kv + lo + 1), c = xs_ld2(T.kv + lo + 2);
@@ -421,6 +448,10 @@ __device__ __forceinline__ double xs_lookup(const Table& T, double e) {
   return v0 + t * (v1 - v0);
 }
 
+__device__ __forceinline__ double xs_lookup(const Table& T, double e) {
+  return xs_end(T, xs_begin(T, e));
+}
+
 struct Mat {
   double st;   // (sigma_s + sigma_a) * barn, m^2
   double pa;   // sigma_a / sigma_t
@@ -433,6 +464,22 @@ __device__ __forceinline__ double clamp_count(double e, const Table& T, uint32_t
   return e;
 }
 
+// refresh_xs in two halves (the XS-range count of the clamps is returned by the first and
+// committed by the caller only if the refresh is used)
+struct MatPre {
+  XsPre s, c;
+  double e;
+  uint32_t nr;
+};
+__device__ __forceinline__ MatPre refresh_begin(const Tables& T, double e) {
+  MatPre p;
+  p.nr = 0;
+  p.e = e;
+  p.s = xs_begin(T.s, clamp_count(e, T.s, p.nr));
+  p.c = xs_begin(T.c, clamp_count(e, T.c, p.nr));
+  return p;
+}
+
 __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, double e,
                                           uint32_t& nrange) {
   const double es = clamp_count(e, T.s, nrange);
@@ -440,6 +487,19 @@ __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, doubl
   const double ss = xs_lookup(T.s, es);
   const double sa = xs_lookup(T.c, ea);
   const double t = ss + sa;
+  Mat m;
+  m.st = t * kBarn;
+  m.pa = t > 0.0 ? sa / t : 0.0;
+  const double rs = t > 0.0 ? ss / t : 0.0;
+  m.H = e - rs * (e * ph.f);
+  return m;
+}
+
+__device__ __forceinline__ Mat refresh_end(const Tables& T, const Phys& ph, const MatPre& p) {
+  const double ss = xs_end(T.s, p.s);
+  const double sa = xs_end(T.c, p.c);
+  const double t = ss + sa;
+  const double e = p.e;
   Mat m;
   m.st = t * kBarn;
   m.pa = t > 0.0 ? sa / t : 0.0;

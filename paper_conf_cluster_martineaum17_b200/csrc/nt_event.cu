@@ -3,15 +3,16 @@
 // Listing 2 advances every particle by one event per iteration: compute the time to each
 // event and determine the next one, then handle all collisions, all facets and all census
 // events in separate loops.  Here the particle set is split into per-warp sets
-// of kWSlots slots, and each warp runs Listing 2 on its own set with warp-level event
-// queues: per iteration the warp snapshots its slots' next-event types, and for each type
-// in turn (collisions, facets, census, new particles) compacts the slots of that type into
-// a queue with one __ballot_sync per slot half and __popc(mask & lanemask_lt) ranks, then
-// handles the queue with all lanes on the same event type (converged code, the Over Events
-// advantage).  No CTA-wide barrier runs inside the loop: warps proceed
-// independently, and a warp refills its free slots from a global counter (one atomicAdd
-// per refill) whenever enough are free, so every warp stays busy until the id range is
-// exhausted (the load balancing of P:344-348).
+// of 64 slots, and each warp runs Listing 2 on its own set with warp-level per-type
+// queues: lane k owns slots k and k + 32 and keeps their next-event types in registers; per
+// iteration one REDUX finds the types present, and each present type (collisions, facets,
+// census, new particles) is handled in at most two rounds -- round 1 one event of every lane
+// holding one, round 2 the second event of lanes holding two (one vote) -- so every round
+// runs one event type across the warp (converged code, the Over Events advantage,
+// P:384-390) and touches one slot per bank pair per half-warp (bank-conflict free).  No
+// CTA-wide barrier runs inside the loop: warps proceed independently, and a warp refills its
+// free slots from a global counter (one atomicAdd per refill) whenever enough are free, so
+// every warp stays busy until the id range is exhausted (the load balancing of P:344-348).
 //
 // State.  Over Events cannot keep a history's cached state in registers across events
 // (P:377-383): every handler loads the particle's state, updates it and stores it back.
@@ -52,6 +53,10 @@ constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many sl
 // ballot + popc ranks (any lane may handle any slot of the half).
 #ifndef NT_EV_COMPACT
 #define NT_EV_COMPACT 0
+#endif
+// A/B option: lane-paired types kept in registers across iterations (no type bytes in smem)
+#ifndef NT_EV_REGTYPES
+#define NT_EV_REGTYPES 0
 #endif
 
 
@@ -554,9 +559,14 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
   uint8_t* wq = s_wq + sb;
   bool exhausted = false;
   unsigned iter = 0;
+#if NT_EV_REGTYPES && !NT_EV_COMPACT
+  uint32_t ta = T_FREE, tb = T_FREE;      // lane k's slots' types stay in its registers
+#endif
   for (;; ++iter) {
+#if !(NT_EV_REGTYPES && !NT_EV_COMPACT)
     __syncwarp();
     uint32_t ta = s_type[sb + lane], tb = s_type[sb + 32 + lane];
+#endif
     // ---- refill: new particles for the free slots (one atomicAdd per warp) ----
     const unsigned fa = __ballot_sync(kFull, ta == T_FREE), fb = __ballot_sync(kFull, tb == T_FREE);
     const unsigned nfree = (unsigned)(__popc(fa) + __popc(fb));
@@ -633,8 +643,10 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
         }
       }
     }
+#if !NT_EV_REGTYPES
     s_type[sb + lane] = (uint8_t)ta;
     s_type[sb + 32 + lane] = (uint8_t)tb;
+#endif
 #endif
   }
   if (lane == 0 && iter > 0) atomicMax(&E.ctl->iter, iter);

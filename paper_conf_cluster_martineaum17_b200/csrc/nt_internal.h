@@ -28,6 +28,13 @@ struct TrackParams {
   const unsigned long long* resume_count;
   int32_t* park_q;            // out-queue of parked local indices
   unsigned long long* park_count;
+  // fused phases (fused_consumers > 0): one launch; CTAs [0, coll_ctas) start as consumers
+  // of park_q (entries published as index + 1 after a fence), the others produce (phase 1)
+  // and turn consumer when their range is exhausted
+  int32_t coll_ctas;
+  uint32_t n_prod;                  // producer warps
+  unsigned long long* park_taken;   // park_q entries claimed by consumers
+  unsigned int* prod_done;          // producer warps finished producing
   // x-slab decomposition (decomposition 1): particles leaving columns [slab_lo, slab_hi)
   int32_t slab_lo, slab_hi;
   int32_t* out_q;             // emigrant local indices

@@ -14,6 +14,13 @@
 
 namespace nt {
 
+#ifndef NT_SMEM_FSUM
+#define NT_SMEM_FSUM 0   // A/B option: per-thread f64 statistic sums in shared memory
+#endif
+#ifndef NT_XS_EARLY
+#define NT_XS_EARLY 0    // A/B option: a collision issues the new energy's XS index loads early
+#endif
+
 __device__ __forceinline__ double d_inf() { return __longlong_as_double(0x7ff0000000000000ll); }
 
 // ---------------------------------------------------------------------------------------
@@ -85,7 +92,7 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 // before native ones); 3 a per-CTA shared-memory copy of a hot window of cells
 // (privatisation), merged into the tally with one RED per cell at the end.
 template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, int kTally, bool kXsWalk,
-          bool kVar, bool kSlab, bool kAoS = false>
+          bool kVar, bool kSlab, bool kAoS = false, bool kFused = false>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
   // particle-store field f of local particle idx: structure of arrays, or -- the
@@ -96,6 +103,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   static_assert(!(kTally && kDet), "tally modes reorder the sum: production tally only");
   static_assert(!(kTally == 3 && kSlab), "hot window: replicated meshes only");
   static_assert(!(kAoS && kSlab), "AoS particle store: replicated meshes only");
+  static_assert(!(kFused && (kSlab || kDet || kAoS)), "fused phases: production, replicated, SoA");
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
   // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
   // almost no shared memory and the L1 stays free for the density / edge gathers.
@@ -104,13 +112,23 @@ history_kernel(const __grid_constant__ TrackParams P) {
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
   __shared__ __align__(16) uint8_t s_blk[kBlk ? kBlkMax : 1];
   __shared__ double s_wabs[kHistoryBlock];   // weight absorbed by implicit capture, per thread
+#if NT_SMEM_FSUM
+  // f64 statistic sums per thread in shared memory (a history's end adds 2-3 of them: a
+  // shared-memory RMW instead of a global one on the critical path of short histories)
+  __shared__ double s_f[SF_COUNT][kHistoryBlock];
+#endif
   __shared__ double s_hot[kTally == 3 ? kHotCells : 1];   // privatised hot window (kTally 3)
   const int t = threadIdx.x;
   const int64_t gt = (int64_t)blockIdx.x * kHistoryBlock + t;
   const int64_t sstride = (int64_t)gridDim.x * kHistoryBlock;
   double* __restrict__ sf = P.slot_f + gt;          // sf[k * sstride]: statistic k
+#if NT_SMEM_FSUM
+#pragma unroll
+  for (int k = 0; k < SF_COUNT; ++k) s_f[k][t] = 0.0;
+#else
 #pragma unroll
   for (int k = 0; k < SF_COUNT; ++k) sf[k * sstride] = 0.0;
+#endif
   if (t < kWarps * SU_COUNT) (&s_u[0][0])[t] = 0u;
   if constexpr (kTally == 3)
     for (int k = t; k < kHotCells; k += kHistoryBlock) s_hot[k] = 0.0;
@@ -126,7 +144,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
   }
   const int wid = t >> 5;
   auto cnt = [&](int k, uint32_t v) { atomicAdd(&s_u[wid][k], v); };
+#if NT_SMEM_FSUM
+  auto fsum = [&](int k, double v) { s_f[k][t] += v; };
+#else
   auto fsum = [&](int k, double v) { sf[k * sstride] += v; };
+#endif
   s_wabs[t] = 0.0;
   const double* __restrict__ ndtab = (kFmt == kDensU8) ? s_nd : P.mesh.nd_tab;
 
@@ -203,6 +225,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
   const bool resume = P.resume_q != nullptr;
   const unsigned long long span2 = resume ? *P.resume_count : span;
   const int park_coll_below = P.park_coll_below;
+  // Fused phases (kFused): one launch; consumer warps resume parked particles while the
+  // producers still run phase 1, so the parked collisions' ALU work fills the issue slots
+  // the RED-bound streaming leaves free.  Per lane: res = the particle is a resumed one;
+  // a consumer lane holds at most one claimed queue position (pend, qpos) and is done (fin)
+  // once every producer has finished and its claim lies beyond the final queue length.
+  bool consumer = kFused && (int)blockIdx.x < P.coll_ctas;
+  bool res = resume, pend = false, fin = false;
+  uint32_t qpos = 0;
   // Park this lane: the state before its next event to the particle store (status st), the
   // index to queue q (one atomicAdd per group of converged lanes); the lane goes idle and
   // takes a new particle.  Used for regime parking (status 2, park_q) and, with x-slabs,
@@ -230,15 +260,91 @@ history_kernel(const __grid_constant__ TrackParams P) {
     unsigned long long k = 0;
     if (lane == ld) k = atomicAdd(qn, (unsigned long long)__popc(am));
     k = __shfl_sync(am, k, ld) + (unsigned long long)__popc(am & lt_mask);
-    q[k] = i;
+    if constexpr (kFused) {
+      // publish to consumers running in this launch: the state, then the entry (index + 1)
+      __threadfence();
+      st_volatile(q + k, i + 1);
+    } else {
+      q[k] = i;
+    }
     active = false;
   };
   auto outside_slab = [&](int32_t cx_) { return cx_ < P.slab_lo || cx_ >= P.slab_hi; };
 
+  // set up the per-history registers of the particle just loaded (x .. ctr, e known)
+  auto setup_loaded = [&]() __attribute__((always_inline)) {
+    exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
+    eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
+    iox = 1.0 / ox;
+    ioy = 1.0 / oy;
+    if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
+    if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
+  };
+
   for (;;) {
+    if constexpr (kFused) {
+      if (consumer) {
+        // ---- consumer refill: claim queue positions for idle lanes, take published ones ----
+        const unsigned want = __ballot_sync(kFull, !active && !pend && !fin);
+        if (want) {
+          const int leader = __ffs(want) - 1;
+          unsigned long long base = 0;
+          if (lane == leader) base = atomicAdd(P.park_taken, (unsigned long long)__popc(want));
+          base = __shfl_sync(kFull, base, leader);
+          if (!active && !pend && !fin) {
+            const unsigned long long q = base + (unsigned long long)__popc(want & lt_mask);
+            // a particle is parked at most once, so positions past the store are never filled
+            if (q >= (unsigned long long)P.n) fin = true;
+            else { qpos = (uint32_t)q; pend = true; }
+          }
+        }
+        if (pend) {
+          int32_t v = ld_volatile(P.park_q + qpos);
+          if (v == 0 && ld_volatile(P.prod_done) >= P.n_prod) {
+            // every producer is done: the queue is final
+            if ((unsigned long long)qpos >= ld_volatile(P.park_count)) { fin = true; pend = false; }
+            else v = ld_volatile(P.park_q + qpos);
+          }
+          if (v != 0) {
+            // a parked particle (status 2): its state from L2 (written by another CTA before
+            // the fence that precedes the entry)
+            __threadfence();
+            pend = false;
+            i = v - 1;
+            active = true;
+            res = true;
+            x = __ldcg(P.p.x + i);
+            y = __ldcg(P.p.y + i);
+            ox = __ldcg(P.p.ox + i);
+            oy = __ldcg(P.p.oy + i);
+            e = __ldcg(P.p.e + i);
+            w = __ldcg(P.p.w + i);
+            mfp = __ldcg(P.p.mfp + i);
+            cx = __ldcg(P.p.cx + i);
+            cy = __ldcg(P.p.cy + i);
+            ctr = __ldcg(P.p.ctr + i);
+            dcen = __ldcg(P.p.dcen + i);
+            acc = __ldcg(P.p.acc + i);
+            dstep = __ldcg(P.p.dstep + i);
+            nf = __ldcg(P.p.nf_s + i);
+            nc = __ldcg(P.p.nc_s + i);
+            setup_loaded();
+            uint32_t nr_dummy = 0;              // (the producer counted the XS clamps)
+            m = refresh_xs(P.xs, ph, e, nr_dummy);
+            cidx = cidx_of(cx, cy);
+            draw = dload(cx, cy, cidx);
+          }
+        }
+        if (!__any_sync(kFull, active)) {
+          if (__all_sync(kFull, fin)) break;
+          __nanosleep(256);
+          continue;
+        }
+      }
+    }
     // ---- refill idle lanes with new particles: one atomic per warp ----
     const unsigned idle = __ballot_sync(kFull, !active);
-    if (!exhausted && idle != 0u && (__popc(idle) >= P.refill_min || idle == kFull)) {
+    if (!consumer && !exhausted && idle != 0u && (__popc(idle) >= P.refill_min || idle == kFull)) {
       const int leader = __ffs(idle) - 1;
       unsigned long long base = 0;
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
@@ -262,12 +368,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
             cx = ld_stream(PP(cx, i), pol_stream);
             cy = ld_stream(PP(cy, i), pol_stream);
             ctr = ld_stream(PP(ctr, i), pol_stream);
-            exn = __ldg(ex + cx + (ox > 0.0 ? 1 : 0));
-            eyn = __ldg(ey + cy + (oy > 0.0 ? 1 : 0));
-            iox = 1.0 / ox;
-            ioy = 1.0 / oy;
-            if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
-            if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
+            res = resume;
+            setup_loaded();
             if constexpr (kXsWalk) {
               bin_s = xs_bin(P.xs.s, clamp_only(e, P.xs.s));
               bin_a = xs_bin(P.xs.c, clamp_only(e, P.xs.c));
@@ -309,6 +411,13 @@ history_kernel(const __grid_constant__ TrackParams P) {
       }
     }
     if (!__any_sync(kFull, active)) {
+      if (kFused && !consumer && exhausted) {
+        // this producer warp is done: count it, then resume parked particles too
+        __threadfence();
+        if (lane == 0) atomicAdd(P.prod_done, 1u);
+        consumer = true;
+        continue;
+      }
       if (exhausted) break;
       continue;
     }
@@ -394,7 +503,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_KILLED_E, w * e);
           fsum(SF_KILLED_W, w);
           outcome = 2;
-        } else if (coll && __popc(__activemask()) < park_coll_below) {
+        } else if (coll && !(kFused && consumer) && __popc(__activemask()) < park_coll_below) {
           park_to(2u, P.park_q, P.park_count);
         } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
@@ -427,6 +536,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
           } else {
             const double mu = 1.0 - 2.0 * u01(r.a);
             const double e2 = e * (((ph.AA + ph.twoA * mu) + 1.0) / ph.Ap1sq);
+#if NT_XS_EARLY
+            // the new energy's table bins: issue the index loads now, so their latency
+            // overlaps the scatter arithmetic (used only if the particle survives)
+            const MatPre mpre = refresh_begin(P.xs, e2);
+#endif
             const double ct = 0.5 * (ph.Ap1 * sqrt(e2 / e) - ph.Am1 * sqrt(e / e2));
             const double sgn = (r.a & 1ull) ? -1.0 : 1.0;
             const double q = 1.0 - ct * ct;
@@ -463,7 +577,12 @@ history_kernel(const __grid_constant__ TrackParams P) {
                 m = refresh_xs_walk(P.xs, ph, e, nr, bin_s, bin_a);
                 if (nr) cnt(SU_XS_RANGE, nr);
               } else {
+#if NT_XS_EARLY
+                if (mpre.nr) cnt(SU_XS_RANGE, mpre.nr);
+                m = refresh_end(P.xs, ph, mpre);
+#else
                 m = xs_refresh(e);
+#endif
               }
               iox = 1.0 / ox;
               ioy = 1.0 / oy;
@@ -547,7 +666,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           st_stream(PP(ncol, i), ld_stream(PP(ncol, i), pol_stream) + nc, pol_stream);
           if (outcome == 1) {
             (*PP(ncen, i)) += 1u;
-            if (resume) (*PP(status, i)) = 1u;           // was parked (2)
+            if (res) (*PP(status, i)) = 1u;              // was parked (2)
           } else {
             (*PP(status, i)) = 0u;
           }
@@ -573,7 +692,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
         if (active && nf + nc >= max_ev) event(true);
       }
     };
-    if (!exhausted) {
+    if (kFused && consumer) {
+      // refill as soon as enough lanes can take a parked particle
+      for (;;) {
+        run_lane();
+        if (__popc(__ballot_sync(kFull, !active && !fin)) >= P.refill_min || !__any_sync(kFull, active))
+          break;
+      }
+    } else if (!exhausted) {
       for (;;) {
         run_lane();
         if (__popc(__ballot_sync(kFull, !active)) >= P.refill_min) break;
@@ -608,7 +734,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
       const int kf = k - SU_COUNT;
       double v = 0.0;
       for (int j = lane2; j < kHistoryBlock; j += 32)
+#if NT_SMEM_FSUM
+        v += s_f[kf][j];
+#else
         v += P.slot_f[(int64_t)blockIdx.x * kHistoryBlock + j + kf * sstride];
+#endif
 #pragma unroll
       for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(kFull, v, o);
       if (lane2 == 0 && v != 0.0) atomicAdd(P.stats_f + kf, v);
@@ -628,7 +758,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
 #define NT_HIST_MINB 6   // resident CTAs per SM the default kernel is compiled for (A/B ab11)
 #endif
 template <bool kDet, bool kTiled, bool kVar>
-static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos) {
+static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos, bool fused) {
   if (fmt == kDensU8) {
     if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, 0, false, kVar, false>;
     if constexpr (!kVar) {
@@ -639,6 +769,8 @@ static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos
         if (tally == 1) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 1, false, false, false>;
         if (tally == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 2, false, false, false>;
         if (tally == 3) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 3, false, false, false>;
+        // fused phases: the default kernel otherwise (nt_api.cu history_fused mirrors this)
+        if (fused) return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, 0, false, false, false, false, true>;
       }
     }
     return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, 0, false, kVar, false>;
@@ -659,25 +791,25 @@ static void* history_slab_fn(int fmt, bool blk) {
 
 template <bool kVar>
 static void* history_select_v(bool det, int fmt, bool tiled, bool blk, int minb, int tally, int xs,
-                              bool aos) {
-  if (det) return tiled ? history_fn<true, true, kVar>(fmt, blk, minb, tally, xs, aos)
-                        : history_fn<true, false, kVar>(fmt, blk, minb, tally, xs, aos);
-  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, tally, xs, aos)
-               : history_fn<false, false, kVar>(fmt, blk, minb, tally, xs, aos);
+                              bool aos, bool fused) {
+  if (det) return tiled ? history_fn<true, true, kVar>(fmt, blk, minb, tally, xs, aos, false)
+                        : history_fn<true, false, kVar>(fmt, blk, minb, tally, xs, aos, false);
+  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, tally, xs, aos, fused)
+               : history_fn<false, false, kVar>(fmt, blk, minb, tally, xs, aos, fused);
 }
 
 static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int tally, int xs,
-                            bool var, bool slab = false, bool aos = false) {
+                            bool var, bool slab = false, bool aos = false, bool fused = false) {
   if (slab) return tiled ? history_slab_fn<true>(fmt, blk) : history_slab_fn<false>(fmt, blk);
-  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, tally, xs, false)
-             : history_select_v<false>(det, fmt, tiled, blk, minb, tally, xs, aos);
+  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, tally, xs, false, false)
+             : history_select_v<false>(det, fmt, tiled, blk, minb, tally, xs, aos, fused);
 }
 
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
                     int xs_search, bool slab, cudaStream_t s) {
   const bool var = tp.ph.vacuum || tp.ph.analog || tp.ph.roulette;
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode, xs_search, var, slab, tp.aos != nullptr);
+                            tally_mode, xs_search, var, slab, tp.aos != nullptr, tp.coll_ctas > 0);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
 }

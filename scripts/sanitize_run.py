@@ -39,6 +39,15 @@ def main():
                 t.close()
                 n += 1
                 print(f"{name} {mode} det={det}: ok", flush=True)
+        # fused phases (one launch, cross-CTA hand-over of parked particles)
+        for fused in (1, 2):
+            t = binding.setup(cfg, mode="history", fused_consumers=fused, defer_below=33)
+            t.run_timestep(cfg.dt)
+            compare_particles(t.read_particles(), op)
+            compare_tally(t.read_tally(), ot, rtol=1e-6, floor=1e-12)
+            t.close()
+            n += 1
+            print(f"{name} history fused={fused}: ok", flush=True)
     # x-slabs (caller-driven exchange, 2 contexts)
     cfg = wl.CONFIGS["tiny_csp"].with_(n_particles=300)
     ts = [binding.setup(cfg, first_id=lo, n_local=k, rank=r, nranks=2, decomposition=1)

@@ -24,9 +24,10 @@ CASES = [
     ("csp", "history", {"density_format": 1}), ("csp", "event", {"density_format": 1}),
     ("csp", "history", {"layout": 1}), ("csp", "event", {"layout": 1}),
     ("csp", "history", {"deterministic": True}),
+    ("csp", "history", {"fused_consumers": 1}),
     ("stream", "history", {}), ("stream", "event", {}),
     ("scatter", "history", {}), ("scatter", "event", {}),
-    ("split", "history", {}), ("split", "event", {}),
+    ("split", "history", {}), ("split", "event", {}), ("split", "history", {"fused_consumers": 1}),
 ]
 
 _CACHE = {}

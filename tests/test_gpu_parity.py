@@ -138,6 +138,24 @@ def test_parity_production_atomic(nt, orc, cfgname, mode, density_format, layout
     compare_stats(gs, os_, rtol=1e-9)
 
 
+@pytest.mark.parametrize("fused", [1, 2])
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "small_csp", "small_scatter", "tiny_split", "tiny_mosaic",
+                                     "tiny_mid", "tiny_hotspot"])
+def test_parity_fused_phases(nt, orc, cfgname, fused):
+    """fused_consumers k: one launch in which k CTAs per SM resume the parked collisions
+    while the others run phase 1 (hand-over through a published queue): same per-particle
+    results, tally within the production bar, every particle tracked once."""
+    cfg = wl.CONFIGS[cfgname]
+    for defer_below in (8, 33):                     # 33: every collision is parked
+        gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, fused_consumers=fused,
+                                 defer_below=defer_below)
+        ot, op, (os_,) = orc.run(cfg)
+        compare_particles(gp, op)
+        compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+        compare_stats(gs, os_, rtol=1e-9)
+        assert np.all(gp["status"] <= 1)
+
+
 @pytest.mark.parametrize("cfgname", ["tiny_csp", "small_csp", "small_scatter", "tiny_split", "tiny_mosaic"])
 def test_parity_aos_particle_layout(nt, orc, cfgname):
     """particle_layout 1 (AoS records while the history kernel runs): same
