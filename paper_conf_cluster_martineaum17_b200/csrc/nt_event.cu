@@ -36,7 +36,7 @@ namespace nt {
 #define NT_EV_WARPS 16
 #endif
 #ifndef NT_EV_REFILL
-#define NT_EV_REFILL 16
+#define NT_EV_REFILL 4
 #endif
 constexpr int kEvWarps = NT_EV_WARPS;        // warps per CTA (one CTA per SM)
 constexpr int kEvBlock = kEvWarps * 32;
@@ -56,7 +56,7 @@ constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many sl
 #endif
 // A/B option: lane-paired types kept in registers across iterations (no type bytes in smem)
 #ifndef NT_EV_REGTYPES
-#define NT_EV_REGTYPES 0
+#define NT_EV_REGTYPES 1
 #endif
 
 

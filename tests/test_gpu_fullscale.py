@@ -23,11 +23,12 @@ CASES = [
     ("csp", "history", {}), ("csp", "event", {}),
     ("csp", "history", {"density_format": 1}), ("csp", "event", {"density_format": 1}),
     ("csp", "history", {"layout": 1}), ("csp", "event", {"layout": 1}),
-    ("csp", "history", {"deterministic": True}),
+    ("csp", "history", {"deterministic": True}), ("csp", "event", {"deterministic": True}),
     ("csp", "history", {"fused_consumers": 1}),
-    ("stream", "history", {}), ("stream", "event", {}),
-    ("scatter", "history", {}), ("scatter", "event", {}),
+    ("stream", "history", {}), ("stream", "event", {}), ("stream", "history", {"deterministic": True}),
+    ("scatter", "history", {}), ("scatter", "event", {}), ("scatter", "history", {"deterministic": True}),
     ("split", "history", {}), ("split", "event", {}), ("split", "history", {"fused_consumers": 1}),
+    ("split", "history", {"deterministic": True}),
 ]
 
 _CACHE = {}
