@@ -199,7 +199,10 @@ const char *nt_last_error(const nt_ctx *ctx); /* never NULL                     
 
 /* The structured 2D mesh of cell-centred mass densities:
  * nx x ny uniform cells over [0,width] x [0,height], density[ny][nx] row-major, kg/m^3,
- * finite and >= 0.  Cell edges are edge(i) = (i*width)/nx. */
+ * finite and >= 0.  Cell edges are edge(i) = (i*width)/nx.  With x-slabs
+ * (decomposition 1) every rank passes the whole map but stores -- and validates -- only
+ * its columns [floor(r nx/P), floor((r+1) nx/P)) plus one halo column on each side; its
+ * tally holds those columns too (nt_read_tally assembles the whole map). */
 nt_status nt_init_mesh(nt_ctx *ctx, int32_t nx, int32_t ny, double width, double height,
                        const double *density);
 
