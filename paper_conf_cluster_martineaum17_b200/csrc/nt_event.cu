@@ -55,6 +55,13 @@ constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many sl
 #define NT_EV_COMPACT 0
 #endif
 // A/B option: lane-paired types kept in registers across iterations (no type bytes in smem)
+// A/B option: iterate over the present event types only (find-first-set), not all four
+#ifndef NT_EV_DOWHILE
+#define NT_EV_DOWHILE 1
+#endif
+#ifndef NT_EV_FFS
+#define NT_EV_FFS 1
+#endif
 #ifndef NT_EV_REGTYPES
 #define NT_EV_REGTYPES 1
 #endif
@@ -623,13 +630,24 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
 #else
     // lane-paired queues: lane k owns slots k and k + 32; a type's events run in at most two
     // rounds, the second only for lanes holding two of them
+#if NT_EV_FFS
+#pragma unroll 1
+    for (unsigned pm = present & 0xfu; pm != 0u; pm &= pm - 1u) {   // present types, in order
+      const uint32_t T = (uint32_t)(__ffs(pm) - 1);
+#else
 #pragma unroll 1
     for (uint32_t T = 0; T < 4; ++T) {
       if (!(present & (1u << T))) continue;
+#endif
       bool pa = (ta & 7u) == T, pb = (tb & 7u) == T;
-
+#if NT_EV_DOWHILE
+      // (the type is present, so round 1 always runs: test for another round at the end)
+#pragma unroll 1
+      do {
+#else
 #pragma unroll 1
       while (__any_sync(kFull, pa || pb)) {
+#endif
         if (pa || pb) {
           const bool first = pa;
           const int s = sb + (first ? lane : 32 + lane);
@@ -641,7 +659,11 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
           else nt = K.birth(s);
           if (first) { ta = nt; pa = false; } else { tb = nt; pb = false; }
         }
+#if NT_EV_DOWHILE
+      } while (__any_sync(kFull, pa || pb));
+#else
       }
+#endif
     }
 #if !NT_EV_REGTYPES
     s_type[sb + lane] = (uint8_t)ta;
