@@ -43,47 +43,35 @@ constexpr int kEvBlock = kEvWarps * 32;
 constexpr int kWSlots = 64;                  // slots per warp: two per lane
 constexpr int kSlots = kEvWarps * kWSlots;   // slots per CTA
 constexpr int kEvRefill = NT_EV_REFILL;      // a warp refills once this many slots are free
-#ifndef NT_EV_EDGE_DIV
-#define NT_EV_EDGE_DIV 0
-#endif
-// Per-type queue of a warp (A/B option): 0 lane-paired -- lane k owns slots k and k+32 and
-// the events of a type run in at most two rounds (round 1: one event of every lane that has
-// one, round 2: the second of lanes that have two), so a round touches slots k or k+32 only
-// and its 8-byte column accesses are bank-conflict free; 1 compacted per slot half with
-// ballot + popc ranks (any lane may handle any slot of the half).
-#ifndef NT_EV_COMPACT
-#define NT_EV_COMPACT 0
-#endif
-// A/B option: lane-paired types kept in registers across iterations (no type bytes in smem)
-// A/B option: iterate over the present event types only (find-first-set), not all four
-#ifndef NT_EV_DOWHILE
-#define NT_EV_DOWHILE 1
-#endif
-#ifndef NT_EV_FFS
-#define NT_EV_FFS 1
-#endif
-#ifndef NT_EV_REGTYPES
-#define NT_EV_REGTYPES 1
-#endif
 
-
-// Type byte of a slot: bits 0-2 the next event (or free / birth), bit 3 the facet crosses
-// an X edge, bit 4 the slot's deposit accumulator is non-zero (it is zero after every
-// flush, so most events neither load nor store it).
-// bit 5: the current cell's block (of the block map) is uniform, so a facet that stays in
-// the block keeps the stored number density (every cell of the block has it).
+// Type byte of a slot (kept in the owning lane's registers): bits 0-2 the next event (or
+// free / birth), bit 3 the facet crosses an X edge, bit 4 the slot's deposit accumulator is
+// non-zero (it is zero after every flush, so most events neither load nor store it), bit 5
+// the current cell's block (of the block map) is uniform, so a facet that stays in the
+// block keeps the stored number density (every cell of the block has it).
 enum : uint32_t { T_COLL = 0, T_FACET = 1, T_CENSUS = 2, T_BIRTH = 3, T_FREE = 4, T_AXBIT = 8,
                   T_ACCBIT = 16, T_UNIBIT = 32 };
 
-// 8-byte slot columns (three of them pack two i32 fields) and one 4-byte column
-enum Col8 : int {
-  C_X = 0, C_Y, C_OX, C_OY, C_IOX, C_IOY, C_EXN, C_EYN, C_MFP, C_DCEN, C_ACC, C_DSTEP,
-  C_W, C_E, C_ST, C_H, C_PA, C_ND, C_CXY, C_NFC, C_CTRSEQ, kCol8
+// Slot columns, 16 bytes each: fields that are read (and mostly written) together share a
+// column, so one LDS.128 / STS.128 moves both (a lane touches slot k or k + 32 only, so a
+// quarter-warp's 16-byte accesses never share a bank group).
+enum Col : int {
+  P_XY = 0,   // x, y
+  P_O,        // omega_x, omega_y
+  P_IO,       // 1/omega_x, 1/omega_y
+  P_EN,       // heading edges x, y
+  P_MD,       // n_mfp, census distance
+  P_AD,       // deposit accumulator, deposits flushed this step
+  P_WH,       // weight, heating response H
+  P_SN,       // sigma_t (m^2), number density of the cell
+  P_EP,       // energy, p_a
+  P_CN,       // int4: cx, cy, facets, collisions (this step)
+  P_CS,       // int4: RNG counter, flush sequence, local particle index, -
+  kCols
 };
 
-constexpr size_t kSmemCols = (size_t)kSlots * (kCol8 * 8 + 4);
 constexpr size_t ev_smem_bytes(bool blk) {
-  return kSmemCols + 2 * (size_t)kSlots /* types, per-warp queues */ + (blk ? (size_t)kBlkMax : 0);
+  return (size_t)kSlots * kCols * 16 + (blk ? (size_t)kBlkMax : 0);
 }
 
 struct EvCtl {
@@ -107,7 +95,7 @@ __device__ __forceinline__ double ev_inf() { return __longlong_as_double(0x7ff00
 
 // A particle's state in registers while one of its events is handled.
 struct St {
-  double x, y, ox, oy, iox, ioy, exn, eyn, mfp, dcen, acc, dstep, w, e, st, H, nd;
+  double x, y, ox, oy, iox, ioy, exn, eyn, mfp, dcen, acc, dstep, w, e, st, H, nd, pa;
   int32_t cx, cy;
   uint32_t nf, nc, ctr;
   uint32_t uni;             // T_UNIBIT when the cell's block is uniform
@@ -123,48 +111,35 @@ struct EvKernel {
   double* sf;               // this thread's f64 statistic slots, stride sstride
   int64_t sstride;
   uint64_t pol;             // L2 evict_last: tally REDs and density gathers
-  double* c8;               // [kCol8][kSlots]
-  int32_t* cpid;            // [kSlots] local particle index
+  double2* cols;            // [kCols][kSlots] 16-byte entries
 
-  __device__ double& d(int f, int s) { return c8[f * kSlots + s]; }
-  __device__ int2& i2(int f, int s) { return reinterpret_cast<int2*>(c8 + f * kSlots)[s]; }
+  __device__ double2& c(int f, int s) { return cols[f * kSlots + s]; }
+  __device__ int4& ci(int f, int s) { return reinterpret_cast<int4*>(cols + f * kSlots)[s]; }
+  // one 8-byte half of a 16-byte entry
+  __device__ double& h(int f, int s, int k) { return reinterpret_cast<double*>(cols + f * kSlots + s)[k]; }
+  __device__ int32_t pid(int s) { return ci(P_CS, s).z; }
 
   __device__ void cnt(int k, uint32_t v) { atomicAdd(s_u + k, (unsigned long long)v); }
   __device__ void fsum(int k, double v) { sf[k * sstride] += v; }
 
   __device__ uint32_t cidx(int32_t cx, int32_t cy) { return (uint32_t)cell_index(P.mesh, cx, cy); }
 
-  // Mesh edges (DESIGN.md §3 MESH): edge(i) = (i*W)/n.  NT_EV_EDGE_DIV evaluates the
-  // expression in place -- the same IEEE operations as the edge tables, so bit-identical --
-  // instead of a dependent global load on every facet (16 warps per SM hide little latency).
-  __device__ double edge_x(int32_t k) {
-#if NT_EV_EDGE_DIV
-    return ((double)k * P.mesh.wx) / (double)P.mesh.gnx;
-#else
-    return __ldg(P.mesh.ex + k);
-#endif
-  }
-  __device__ double edge_y(int32_t k) {
-#if NT_EV_EDGE_DIV
-    return ((double)k * P.mesh.wy) / (double)P.mesh.ny;
-#else
-    return __ldg(P.mesh.ey + k);
-#endif
-  }
+  __device__ double edge_x(int32_t k) { return __ldg(P.mesh.ex + k); }
+  __device__ double edge_y(int32_t k) { return __ldg(P.mesh.ey + k); }
 
   // number density of cell (cx, cy); uni: its block is uniform (block map)
   __device__ double nd_of(int32_t cx, int32_t cy, bool& uni) {
-    const uint32_t ci = cidx(cx, cy);
+    const uint32_t ci_ = cidx(cx, cy);
     uni = false;
     if constexpr (kBlk) {
       uint32_t code = s_blk[(cy >> P.mesh.bshift) * P.mesh.nbx + (cx >> P.mesh.bshift)];
       uni = code != kBlkMixed;
-      if (!uni) code = ldg_u8_hint(P.mesh.rho8 + ci, pol);
+      if (!uni) code = ldg_u8_hint(P.mesh.rho8 + ci_, pol);
       return s_nd[code];
     } else if constexpr (kFmt == kDensU8) {
-      return s_nd[ldg_u8_hint(P.mesh.rho8 + ci, pol)];
+      return s_nd[ldg_u8_hint(P.mesh.rho8 + ci_, pol)];
     } else {
-      return number_density<kFmt>(P.mesh, P.mesh.nd_tab, ci, ph.cn);
+      return number_density<kFmt>(P.mesh, P.mesh.nd_tab, ci_, ph.cn);
     }
   }
 
@@ -172,19 +147,18 @@ struct EvKernel {
   __device__ void flush(int s, St& v) {
     const uint32_t cell = cidx(v.cx, v.cy);
     if constexpr (kDet) {
-      const int32_t pi = cpid[s];
-      int2 cs = i2(C_CTRSEQ, s);
+      int4 cs = ci(P_CS, s);
       const uint32_t seq = (uint32_t)cs.y;
       const unsigned long long rs = atomicAdd(P.rec_count, 1ull);
       if (rs < P.rec_cap) {
         P.rec_key[rs] = ((unsigned long long)cell << 40) |
-                        ((unsigned long long)((int64_t)pi - P.lo) << 24) |
+                        ((unsigned long long)((int64_t)cs.z - P.lo) << 24) |
                         (unsigned long long)(seq & 0xffffffu);
         P.rec_val[rs] = v.acc;
       }
       if (seq >= (1u << 24)) cnt(SU_REC_OVERFLOW, 1u);
       cs.y = (int)(seq + 1u);
-      i2(C_CTRSEQ, s) = cs;
+      ci(P_CS, s) = cs;
     } else {
       red_add_hint(P.mesh.tally + cell, v.acc, pol);
     }
@@ -194,7 +168,7 @@ struct EvKernel {
 
   // A history ended in slot s: write the particle store (census: alive; otherwise dead).
   __device__ uint32_t finish(int s, const St& v, bool alive) {
-    const int32_t pi = cpid[s];
+    const int32_t pi = pid(s);
     if (!(isfinite(v.x) && isfinite(v.y) && isfinite(v.e) && isfinite(v.w))) cnt(SU_NONFINITE, 1u);
     P.p.x[pi] = v.x;
     P.p.y[pi] = v.y;
@@ -216,7 +190,7 @@ struct EvKernel {
     return T_FREE;
   }
 
-  // The event cap (R27): flush, count, kill.  v.e must be loaded.
+  // The event cap (R27): flush, count, kill.  v.e, v.ox, v.oy, v.ctr must be loaded.
   __device__ uint32_t cap_kill(int s, St& v) {
     cnt(SU_EVENT_CAP, 1u);
     flush(s, v);
@@ -231,7 +205,7 @@ struct EvKernel {
   // distance from the state it loads anyway -- the same expressions, so the same value --
   // instead of a stored distance column).  Same expressions as the history kernel
   // (R28 clamps).
-  __device__ uint32_t classify(int s, const St& v) {
+  __device__ uint32_t classify(const St& v) {
     const double sig = v.nd * v.st;
     const double tx = (v.exn - v.x) * v.iox;
     const double ty = (v.eyn - v.y) * v.ioy;
@@ -252,23 +226,37 @@ struct EvKernel {
     return T_CENSUS | accb;
   }
 
-  __device__ void load_nfc(int s, St& v) {
-    const int2 a = i2(C_CXY, s), b = i2(C_NFC, s);
-    v.cx = a.x; v.cy = a.y; v.nf = (uint32_t)b.x; v.nc = (uint32_t)b.y;
+  __device__ void load_cn(int s, St& v) {
+    const int4 a = ci(P_CN, s);
+    v.cx = a.x; v.cy = a.y; v.nf = (uint32_t)a.z; v.nc = (uint32_t)a.w;
+  }
+  __device__ void store_cn(int s, const St& v) {
+    ci(P_CN, s) = make_int4(v.cx, v.cy, (int)v.nf, (int)v.nc);
+  }
+  // acc (only while its type bit says it is non-zero) and dstep
+  __device__ void load_ad(int s, uint32_t ty, St& v) {
+    if (ty & T_ACCBIT) {
+      const double2 a = c(P_AD, s);
+      v.acc = a.x; v.dstep = a.y;
+    } else {
+      v.acc = 0.0; v.dstep = h(P_AD, s, 1);
+    }
   }
 
   // ---- collision ----
   __device__ uint32_t collision(int s, uint32_t ty) {
     St v;
-    v.x = d(C_X, s); v.y = d(C_Y, s); v.ox = d(C_OX, s); v.oy = d(C_OY, s);
-    v.mfp = d(C_MFP, s); v.dcen = d(C_DCEN, s);
-    v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
-    v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.e = d(C_E, s); v.st = d(C_ST, s); v.H = d(C_H, s);
-    v.nd = d(C_ND, s);
+    { const double2 a = c(P_XY, s); v.x = a.x; v.y = a.y; }
+    { const double2 a = c(P_O, s); v.ox = a.x; v.oy = a.y; }
+    { const double2 a = c(P_MD, s); v.mfp = a.x; v.dcen = a.y; }
+    load_ad(s, ty, v);
+    { const double2 a = c(P_WH, s); v.w = a.x; v.H = a.y; }
+    { const double2 a = c(P_EP, s); v.e = a.x; v.pa = a.y; }
+    { const double2 a = c(P_SN, s); v.st = a.x; v.nd = a.y; }
     v.uni = ty & T_UNIBIT;
-    load_nfc(s, v);
-    v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
-    const double pa = d(C_PA, s);
+    load_cn(s, v);
+    int4 cs = ci(P_CS, s);
+    v.ctr = (uint32_t)cs.x;
     const double sig = v.nd * v.st;
     const double dd = v.mfp / sig;               // the collision distance classify compared
     v.nc += 1u;
@@ -276,19 +264,19 @@ struct EvKernel {
     v.x = v.x + dd * v.ox;
     v.y = v.y + dd * v.oy;
     v.dcen = v.dcen - dd;
-    const uint64_t pid = (uint64_t)(P.first_id + cpid[s]);
-    const U64x2 r = threefry2x64_20((uint64_t)v.ctr, 0, pid, P.seed);
+    const uint64_t pidg = (uint64_t)(P.first_id + cs.z);
+    const U64x2 r = threefry2x64_20((uint64_t)v.ctr, 0, pidg, P.seed);
     v.ctr += 1u;
     double mfp_u = u01(r.b);
     bool absorbed = false;
     if (!ph.analog) {                           // implicit capture
       const double w0 = v.w;
-      v.w = v.w * (1.0 - pa);
+      v.w = v.w * (1.0 - v.pa);
       fsum(SF_ABSORBED_W, w0 - v.w);
-    } else if (u01(r.b) < pa) {                // sampled absorption (R31)
+    } else if (u01(r.b) < v.pa) {              // sampled absorption (R31)
       absorbed = true;
     } else {                                    // scatter: n_mfp from the next counter
-      const U64x2 r2 = threefry2x64_20((uint64_t)v.ctr, 0, pid, P.seed);
+      const U64x2 r2 = threefry2x64_20((uint64_t)v.ctr, 0, pidg, P.seed);
       v.ctr += 1u;
       mfp_u = u01(r2.a);
     }
@@ -315,7 +303,7 @@ struct EvKernel {
     bool kill = v.e < ph.e_min || v.w < ph.w_min;   // termination
     if (kill && ph.roulette && !(v.e < ph.e_min)) {
       // Russian roulette (R32): survive with probability w / w_s at weight w_s
-      const U64x2 r3 = threefry2x64_20((uint64_t)v.ctr, 0, pid, P.seed);
+      const U64x2 r3 = threefry2x64_20((uint64_t)v.ctr, 0, pidg, P.seed);
       v.ctr += 1u;
       if (u01(r3.a) < v.w / ph.w_roul) {
         fsum(SF_ROULETTE, ph.w_roul - v.w);
@@ -338,19 +326,26 @@ struct EvKernel {
     if (nr) cnt(SU_XS_RANGE, nr);
     v.st = m.st;
     v.H = m.H;
+    v.pa = m.pa;
     v.iox = 1.0 / v.ox;
     v.ioy = 1.0 / v.oy;
     if (v.ox == 0.0) { v.exn = ev_inf(); v.iox = ev_inf(); }
     if (v.oy == 0.0) { v.eyn = ev_inf(); v.ioy = ev_inf(); }
     v.mfp = -log(mfp_u);
-    i2(C_CTRSEQ, s).x = (int)v.ctr;
-    i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);
+    cs.x = (int)v.ctr;
+    ci(P_CS, s) = cs;
+    store_cn(s, v);
     if ((int64_t)(v.nf + v.nc) >= P.max_events) return cap_kill(s, v);
-    d(C_X, s) = v.x; d(C_Y, s) = v.y; d(C_OX, s) = v.ox; d(C_OY, s) = v.oy;
-    d(C_IOX, s) = v.iox; d(C_IOY, s) = v.ioy; d(C_EXN, s) = v.exn; d(C_EYN, s) = v.eyn;
-    d(C_MFP, s) = v.mfp; d(C_DCEN, s) = v.dcen; d(C_ACC, s) = v.acc;
-    d(C_W, s) = v.w; d(C_E, s) = v.e; d(C_ST, s) = v.st; d(C_H, s) = v.H; d(C_PA, s) = m.pa;
-    return classify(s, v);
+    c(P_XY, s) = make_double2(v.x, v.y);
+    c(P_O, s) = make_double2(v.ox, v.oy);
+    c(P_IO, s) = make_double2(v.iox, v.ioy);
+    c(P_EN, s) = make_double2(v.exn, v.eyn);
+    c(P_MD, s) = make_double2(v.mfp, v.dcen);
+    c(P_AD, s) = make_double2(v.acc, v.dstep);
+    c(P_WH, s) = make_double2(v.w, v.H);
+    c(P_EP, s) = make_double2(v.e, v.pa);
+    c(P_SN, s) = make_double2(v.st, v.nd);
+    return classify(v);
   }
 
   // ---- facet ----
@@ -361,7 +356,7 @@ struct EvKernel {
   // rejected: csp 70.5 -> 91.2 ms, profiles/ab/r02_ab9.)
   struct Fct {
     St v;
-    double om, enew, ndn, dd;
+    double om, enew, ndn;
     int32_t c, c2, ncx, ncy;
     uint32_t uni;
     bool ax, refl, keep;
@@ -370,8 +365,8 @@ struct EvKernel {
   __device__ void facet_pre(int s, uint32_t ty, Fct& f) {
     St& v = f.v;
     f.ax = (ty & T_AXBIT) != 0;
-    load_nfc(s, v);
-    v.iox = d(C_IOX, s); v.ioy = d(C_IOY, s);
+    load_cn(s, v);
+    { const double2 a = c(P_IO, s); v.iox = a.x; v.ioy = a.y; }
     f.c = f.ax ? v.cx : v.cy;
     const bool pos = (f.ax ? v.iox : v.ioy) > 0.0;  // crossed axis' direction: sign of 1/omega
     const int32_t cs = f.c + (pos ? 1 : -1);
@@ -392,14 +387,14 @@ struct EvKernel {
       f.ndn = nd_of(f.ncx, f.ncy, u);
       f.uni = u ? T_UNIBIT : 0u;
     }
-    v.x = d(C_X, s); v.y = d(C_Y, s);
-    v.exn = d(C_EXN, s); v.eyn = d(C_EYN, s);
+    { const double2 a = c(P_XY, s); v.x = a.x; v.y = a.y; }
+    { const double2 a = c(P_EN, s); v.exn = a.x; v.eyn = a.y; }
     // the direction cosine of the coordinate that moves (the other is snapped to the edge)
-    f.om = d(f.ax ? C_OY : C_OX, s);
-    v.mfp = d(C_MFP, s); v.dcen = d(C_DCEN, s);
-    v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
-    v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.st = d(C_ST, s); v.H = d(C_H, s);
-    v.nd = d(C_ND, s);
+    f.om = h(P_O, s, f.ax ? 1 : 0);
+    { const double2 a = c(P_MD, s); v.mfp = a.x; v.dcen = a.y; }
+    load_ad(s, ty, v);
+    { const double2 a = c(P_WH, s); v.w = a.x; v.H = a.y; }
+    { const double2 a = c(P_SN, s); v.st = a.x; v.nd = a.y; }
   }
 
   __device__ void facet_math(int s, Fct& f) {
@@ -421,44 +416,40 @@ struct EvKernel {
   __device__ uint32_t facet_post(int s, Fct& f) {
     St& v = f.v;
     if (f.refl) {
-      v.ox = d(C_OX, s);
-      v.oy = d(C_OY, s);
+      { const double2 a = c(P_O, s); v.ox = a.x; v.oy = a.y; }
       if (ph.vacuum) {                          // vacuum boundary (R30): escape
-        v.e = d(C_E, s);
-        v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
+        v.e = h(P_EP, s, 0);
+        v.ctr = (uint32_t)ci(P_CS, s).x;
         cnt(SU_ESCAPED, 1u);
         fsum(SF_ESCAPED_E, v.w * v.e);
         fsum(SF_ESCAPED_W, v.w);
         return finish(s, v, false);
       }
-      if (f.ax) { v.ox = -v.ox; v.iox = -v.iox; d(C_OX, s) = v.ox; d(C_IOX, s) = v.iox; }
-      else      { v.oy = -v.oy; v.ioy = -v.ioy; d(C_OY, s) = v.oy; d(C_IOY, s) = v.ioy; }
+      if (f.ax) { v.ox = -v.ox; v.iox = -v.iox; }
+      else      { v.oy = -v.oy; v.ioy = -v.ioy; }
+      c(P_O, s) = make_double2(v.ox, v.oy);
+      c(P_IO, s) = make_double2(v.iox, v.ioy);
     }
     v.cx = f.ncx;
     v.cy = f.ncy;
-    if (f.ax) { v.exn = f.enew; d(C_EXN, s) = v.exn; }
-    else      { v.eyn = f.enew; d(C_EYN, s) = v.eyn; }
+    if (f.ax) v.exn = f.enew; else v.eyn = f.enew;
+    c(P_EN, s) = make_double2(v.exn, v.eyn);
     v.uni = f.uni;
     if (!f.keep) {
       v.nd = f.ndn;
-      d(C_ND, s) = v.nd;
+      h(P_SN, s, 1) = v.nd;
     }
-    i2(C_NFC, s) = make_int2((int)v.nf, (int)v.nc);
+    store_cn(s, v);
     if ((int64_t)(v.nf + v.nc) >= P.max_events) {
-      v.e = d(C_E, s);
-      v.ox = d(C_OX, s);
-      v.oy = d(C_OY, s);
-      v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
-      i2(C_CXY, s) = make_int2(v.cx, v.cy);
+      v.e = h(P_EP, s, 0);
+      { const double2 a = c(P_O, s); v.ox = a.x; v.oy = a.y; }
+      v.ctr = (uint32_t)ci(P_CS, s).x;
       return cap_kill(s, v);
     }
-    d(C_X, s) = v.x;
-    d(C_Y, s) = v.y;
-    d(C_MFP, s) = v.mfp;
-    d(C_DCEN, s) = v.dcen;
-    d(C_DSTEP, s) = v.dstep;
-    i2(C_CXY, s) = make_int2(v.cx, v.cy);
-    return classify(s, v);                      // acc == 0 after the flush
+    c(P_XY, s) = make_double2(v.x, v.y);
+    c(P_MD, s) = make_double2(v.mfp, v.dcen);
+    h(P_AD, s, 1) = v.dstep;                    // acc == 0 after the flush
+    return classify(v);
   }
 
   __device__ uint32_t facet(int s, uint32_t ty) {
@@ -471,17 +462,21 @@ struct EvKernel {
   // ---- census ----
   __device__ uint32_t census(int s, uint32_t ty) {
     St v;
-    v.ox = d(C_OX, s); v.oy = d(C_OY, s);
-    v.acc = (ty & T_ACCBIT) ? d(C_ACC, s) : 0.0;
-    v.dstep = d(C_DSTEP, s); v.w = d(C_W, s); v.e = d(C_E, s);
-    load_nfc(s, v);
-    v.ctr = (uint32_t)i2(C_CTRSEQ, s).x;
-    const double dd = d(C_DCEN, s);              // census: the remaining census distance
-    const double sig = d(C_ND, s) * d(C_ST, s);
-    v.acc += ((v.w * dd) * sig) * d(C_H, s);
-    v.x = d(C_X, s) + dd * v.ox;
-    v.y = d(C_Y, s) + dd * v.oy;
-    const double nm = d(C_MFP, s) - dd * sig;
+    { const double2 a = c(P_O, s); v.ox = a.x; v.oy = a.y; }
+    load_ad(s, ty, v);
+    { const double2 a = c(P_WH, s); v.w = a.x; v.H = a.y; }
+    v.e = h(P_EP, s, 0);
+    load_cn(s, v);
+    v.ctr = (uint32_t)ci(P_CS, s).x;
+    const double2 md = c(P_MD, s);
+    const double dd = md.y;                     // census: the remaining census distance
+    const double2 sn = c(P_SN, s);
+    const double sig = sn.y * sn.x;
+    v.acc += ((v.w * dd) * sig) * v.H;
+    const double2 xy = c(P_XY, s);
+    v.x = xy.x + dd * v.ox;
+    v.y = xy.y + dd * v.oy;
+    const double nm = md.x - dd * sig;
     v.mfp = nm > 0.0 ? nm : 0.0;
     flush(s, v);
     cnt(SU_CENSUS, 1u);
@@ -490,9 +485,9 @@ struct EvKernel {
     return finish(s, v, true);
   }
 
-  // ---- a new particle (local index in cpid): its slot state and first event ----
+  // ---- a new particle (local index in P_CS.z): its slot state and first event ----
   __device__ uint32_t birth(int s) {
-    const int32_t pi = cpid[s];
+    const int32_t pi = pid(s);
     if (P.p.status[pi] != 1u) return T_FREE;
     St v;
     v.ox = P.p.ox[pi]; v.oy = P.p.oy[pi];
@@ -510,23 +505,26 @@ struct EvKernel {
     v.x = P.p.x[pi]; v.y = P.p.y[pi];
     v.mfp = P.p.mfp[pi]; v.dcen = speed(v.e, ph) * P.dt;
     v.acc = 0.0; v.dstep = 0.0;
-    v.w = P.p.w[pi]; v.st = m.st; v.H = m.H;
+    v.w = P.p.w[pi]; v.st = m.st; v.H = m.H; v.pa = m.pa;
     bool u;
     v.nd = nd_of(v.cx, v.cy, u);
     v.uni = u ? T_UNIBIT : 0u;
     v.nf = 0u; v.nc = 0u;
     v.ctr = P.p.ctr[pi];
     cnt(SU_ALIVE, 1u);
-    d(C_X, s) = v.x; d(C_Y, s) = v.y; d(C_OX, s) = v.ox; d(C_OY, s) = v.oy;
-    d(C_IOX, s) = v.iox; d(C_IOY, s) = v.ioy; d(C_EXN, s) = v.exn; d(C_EYN, s) = v.eyn;
-    d(C_MFP, s) = v.mfp; d(C_DCEN, s) = v.dcen; d(C_DSTEP, s) = 0.0;
-    d(C_W, s) = v.w; d(C_E, s) = v.e; d(C_ST, s) = v.st; d(C_H, s) = v.H; d(C_PA, s) = m.pa;
-    d(C_ND, s) = v.nd;
-    i2(C_CXY, s) = make_int2(v.cx, v.cy);
-    i2(C_NFC, s) = make_int2(0, 0);
-    i2(C_CTRSEQ, s) = make_int2((int)v.ctr, 0);
+    c(P_XY, s) = make_double2(v.x, v.y);
+    c(P_O, s) = make_double2(v.ox, v.oy);
+    c(P_IO, s) = make_double2(v.iox, v.ioy);
+    c(P_EN, s) = make_double2(v.exn, v.eyn);
+    c(P_MD, s) = make_double2(v.mfp, v.dcen);
+    c(P_AD, s) = make_double2(0.0, 0.0);
+    c(P_WH, s) = make_double2(v.w, v.H);
+    c(P_EP, s) = make_double2(v.e, v.pa);
+    c(P_SN, s) = make_double2(v.st, v.nd);
+    store_cn(s, v);
+    ci(P_CS, s) = make_int4((int)v.ctr, 0, pi, 0);
     if (P.max_events <= 0) return cap_kill(s, v);
-    return classify(s, v);
+    return classify(v);
   }
 };
 
@@ -536,11 +534,8 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
   extern __shared__ __align__(16) unsigned char smem[];
   __shared__ unsigned long long s_u[SU_COUNT];
   __shared__ double s_nd[kFmt == kDensU8 ? 256 : 1];
-  double* c8 = reinterpret_cast<double*>(smem);
-  int32_t* cpid = reinterpret_cast<int32_t*>(c8 + (size_t)kCol8 * kSlots);
-  uint8_t* s_type = reinterpret_cast<uint8_t*>(cpid + kSlots);
-  uint8_t* s_wq = s_type + kSlots;             // per-warp event queue (slot offsets)
-  uint8_t* s_blk = s_wq + kSlots;              // block map (kBlk)
+  double2* cols = reinterpret_cast<double2*>(smem);
+  uint8_t* s_blk = reinterpret_cast<uint8_t*>(cols + (size_t)kCols * kSlots);   // block map (kBlk)
   const int t = threadIdx.x;
   const int lane = t & 31, wid = t >> 5;
   const unsigned lt = (1u << lane) - 1u;
@@ -548,7 +543,6 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
   const int64_t gt = (int64_t)bidx * kEvBlock + t;
   const int64_t sstride = (int64_t)gridDim.x * kEvBlock;
   if (t < SU_COUNT) s_u[t] = 0u;
-  for (int k = t; k < kSlots; k += kEvBlock) s_type[k] = (uint8_t)T_FREE;
 #pragma unroll
   for (int k = 0; k < SF_COUNT; ++k) P.slot_f[gt + k * sstride] = 0.0;
   if constexpr (kFmt == kDensU8) {
@@ -560,94 +554,54 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
     }
   }
   __syncthreads();
-  EvKernel<kDet, kFmt, kBlk> K{P, P.ph, s_nd, s_blk, s_u, P.slot_f + gt, sstride, l2_evict_last(), c8, cpid};
+  EvKernel<kDet, kFmt, kBlk> K{P, P.ph, s_nd, s_blk, s_u, P.slot_f + gt, sstride, l2_evict_last(), cols};
   const unsigned long long span = (unsigned long long)(P.hi - P.lo);
   const int sb = wid * kWSlots;                // this warp's slots [sb, sb + 64)
-  uint8_t* wq = s_wq + sb;
   bool exhausted = false;
   unsigned iter = 0;
-#if NT_EV_REGTYPES && !NT_EV_COMPACT
-  uint32_t ta = T_FREE, tb = T_FREE;      // lane k's slots' types stay in its registers
-#endif
+  // Lane k owns slots sb + k and sb + 32 + k; their type bytes live in its registers.
+  uint32_t ta = T_FREE, tb = T_FREE;
   for (;; ++iter) {
-#if !(NT_EV_REGTYPES && !NT_EV_COMPACT)
-    __syncwarp();
-    uint32_t ta = s_type[sb + lane], tb = s_type[sb + 32 + lane];
-#endif
-    // ---- refill: new particles for the free slots (one atomicAdd per warp) ----
-    const unsigned fa = __ballot_sync(kFull, ta == T_FREE), fb = __ballot_sync(kFull, tb == T_FREE);
-    const unsigned nfree = (unsigned)(__popc(fa) + __popc(fb));
-    if (!exhausted && nfree >= (unsigned)kEvRefill) {
-      unsigned long long base = 0;
-      if (lane == 0) base = atomicAdd(&E.ctl->counter, (unsigned long long)nfree);
-      base = __shfl_sync(kFull, base, 0);
-      const unsigned long long avail = base < span ? (span - base < nfree ? span - base : nfree) : 0ull;
-      if (base + nfree >= span) exhausted = true;
-      const unsigned ra = (unsigned)__popc(fa & lt), rb = (unsigned)(__popc(fa) + __popc(fb & lt));
-      if (ta == T_FREE && ra < avail) {
-        cpid[sb + lane] = (int32_t)(P.lo + (int64_t)(base + ra));
-        ta = T_BIRTH;
-      }
-      if (tb == T_FREE && rb < avail) {
-        cpid[sb + 32 + lane] = (int32_t)(P.lo + (int64_t)(base + rb));
-        tb = T_BIRTH;
+    // the event types present in the warp's slots (one REDUX): absent types cost nothing,
+    // and the refill votes run only when a slot is free
+    unsigned present = __reduce_or_sync(kFull, (1u << (ta & 7u)) | (1u << (tb & 7u)));
+    if (!exhausted && (present & (1u << T_FREE))) {
+      // ---- refill: new particles for the free slots (one atomicAdd per warp) ----
+      const unsigned fa = __ballot_sync(kFull, ta == T_FREE), fb = __ballot_sync(kFull, tb == T_FREE);
+      const unsigned nfree = (unsigned)(__popc(fa) + __popc(fb));
+      if (nfree >= (unsigned)kEvRefill) {
+        unsigned long long base = 0;
+        if (lane == 0) base = atomicAdd(&E.ctl->counter, (unsigned long long)nfree);
+        base = __shfl_sync(kFull, base, 0);
+        const unsigned long long avail = base < span ? (span - base < nfree ? span - base : nfree) : 0ull;
+        if (base + nfree >= span) exhausted = true;
+        const unsigned ra = (unsigned)__popc(fa & lt), rb = (unsigned)(__popc(fa) + __popc(fb & lt));
+        if (ta == T_FREE && ra < avail) {
+          K.ci(P_CS, sb + lane).z = (int32_t)(P.lo + (int64_t)(base + ra));
+          ta = T_BIRTH;
+        }
+        if (tb == T_FREE && rb < avail) {
+          K.ci(P_CS, sb + 32 + lane).z = (int32_t)(P.lo + (int64_t)(base + rb));
+          tb = T_BIRTH;
+        }
+        if (avail > 0ull) present |= 1u << T_BIRTH;
       }
     }
-    if (!__any_sync(kFull, ta != T_FREE || tb != T_FREE)) {
+    if (!(present & 0xfu)) {                   // every slot free
       if (exhausted) break;
       continue;
     }
     // ---- Listing 2: all collisions, then all facets, then all census, then the births ----
-    // the event types present in the warp's slots (one REDUX): absent types cost nothing
-    const unsigned present = __reduce_or_sync(kFull, (1u << (ta & 7u)) | (1u << (tb & 7u)));
-#if NT_EV_COMPACT
-    // queues compacted per slot half: ballot + popc ranks, any lane may take any slot
+    // Lane-paired per-type queues: a type's events run in at most two rounds -- round 1 one
+    // event of every lane holding one, round 2 the second of lanes holding two -- so a round
+    // touches slot k or k + 32 only: conflict-free shared-memory accesses.  Only the present
+    // types are visited (find-first-set over the REDUX), in Listing 2's order.
 #pragma unroll 1
-    for (uint32_t T = 0; T < 4; ++T) {
-      if (!(present & (1u << T))) continue;
-#pragma unroll 1
-      for (int h = 0; h < 2; ++h) {
-        const uint32_t ty = h ? tb : ta;
-        const bool mine = (ty & 7u) == T;
-        const unsigned m = __ballot_sync(kFull, mine);
-        if (m == 0u) continue;
-        const int n = __popc(m);
-        if (mine) wq[__popc(m & lt)] = (uint8_t)(32 * h + lane);
-        __syncwarp();
-        if (lane < n) {
-          const int s = sb + wq[lane];
-          const uint32_t tys = s_type[s];
-          uint32_t nt;
-          if (T == T_COLL) nt = K.collision(s, tys);
-          else if (T == T_FACET) nt = K.facet(s, tys);
-          else if (T == T_CENSUS) nt = K.census(s, tys);
-          else nt = K.birth(s);
-          s_type[s] = (uint8_t)nt;
-        }
-        __syncwarp();
-      }
-    }
-#else
-    // lane-paired queues: lane k owns slots k and k + 32; a type's events run in at most two
-    // rounds, the second only for lanes holding two of them
-#if NT_EV_FFS
-#pragma unroll 1
-    for (unsigned pm = present & 0xfu; pm != 0u; pm &= pm - 1u) {   // present types, in order
+    for (unsigned pm = present & 0xfu; pm != 0u; pm &= pm - 1u) {
       const uint32_t T = (uint32_t)(__ffs(pm) - 1);
-#else
-#pragma unroll 1
-    for (uint32_t T = 0; T < 4; ++T) {
-      if (!(present & (1u << T))) continue;
-#endif
       bool pa = (ta & 7u) == T, pb = (tb & 7u) == T;
-#if NT_EV_DOWHILE
-      // (the type is present, so round 1 always runs: test for another round at the end)
 #pragma unroll 1
-      do {
-#else
-#pragma unroll 1
-      while (__any_sync(kFull, pa || pb)) {
-#endif
+      do {                                      // (the type is present: round 1 always runs)
         if (pa || pb) {
           const bool first = pa;
           const int s = sb + (first ? lane : 32 + lane);
@@ -659,17 +613,8 @@ __global__ void __launch_bounds__(kEvBlock, 1) ev_loop_kernel(const __grid_const
           else nt = K.birth(s);
           if (first) { ta = nt; pa = false; } else { tb = nt; pb = false; }
         }
-#if NT_EV_DOWHILE
       } while (__any_sync(kFull, pa || pb));
-#else
-      }
-#endif
     }
-#if !NT_EV_REGTYPES
-    s_type[sb + lane] = (uint8_t)ta;
-    s_type[sb + 32 + lane] = (uint8_t)tb;
-#endif
-#endif
   }
   if (lane == 0 && iter > 0) atomicMax(&E.ctl->iter, iter);
 

@@ -7,6 +7,9 @@ ROOT=$(cd "$(dirname "$0")/../.." && pwd)
 PKG=$ROOT/paper_conf_cluster_martineaum17_b200
 NCCL=$(python -c "import nvidia.nccl as n, os; print(list(n.__path__)[0])")
 mkdir -p $PKG/lib/variants $ROOT/build/variants
+# the variants link against the other objects of a full build (build/ is not shipped to the
+# GPU box: rebuild it there when missing)
+ls $ROOT/build/nt_api.o > /dev/null 2>&1 || (cd $ROOT && python -m paper_conf_cluster_martineaum17_b200.build --force > /dev/null)
 for spec in "$@"; do
   name=${spec%%:*}; flags=${spec#*:}
   for src in nt_kernels nt_event; do
