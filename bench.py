@@ -191,7 +191,10 @@ def parse():
     ap.add_argument("--defer-below", type=int, default=0,
                     help="collision deferral threshold (0 default 8, 1 off, 33 park every collision)")
     ap.add_argument("--xs-search", type=int, default=0,
-                    help="0 bucketed binary search, 1 plain binary search, 2 cached-bin linear walk")
+                    help="0 direct bucket rows (one dependent load per lookup), 1 plain binary search, "
+                         "2 cached-bin linear walk, 3 bucket index alone (two dependent loads)")
+    ap.add_argument("--xs-l2-persist", type=int, default=0,
+                    help="1: L2 persisting access-policy window over the XS tables while tracking")
     ap.add_argument("--table-size", type=int, default=0,
                     help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
     ap.add_argument("--fused-consumers", type=int, default=0,
@@ -341,7 +344,8 @@ def main():
                          refill_min=a.refill_min, layout=a.layout, density_format=a.density_format,
                          tally_mode=a.tally_mode, defer_below=a.defer_below,
                          xs_search=a.xs_search, hot_window=hot_window(cfg),
-                         particle_layout=a.particle_layout, fused_consumers=a.fused_consumers)
+                         particle_layout=a.particle_layout, fused_consumers=a.fused_consumers,
+                         xs_l2_persist=a.xs_l2_persist)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)
@@ -453,7 +457,9 @@ def main():
                        "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED", "CAS-emulated fp64 add",
                                  "shared-memory hot window %s + RED" % (hot_window(cfg),)][a.tally_mode],
                        "defer_below": a.defer_below or 8,
-                       "xs_search": ["bucketed binary", "binary", "cached-bin walk"][a.xs_search],
+                       "xs_search": ["direct bucket rows", "binary", "cached-bin walk",
+                                     "bucket index"][a.xs_search],
+                       "xs_l2_persist": bool(a.xs_l2_persist),
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
                        "tables": [len(tables[0]), len(tables[2])],
                        "parallelism": f"dp{world} (particle id shards, tally NCCL allreduce)",

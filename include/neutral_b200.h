@@ -103,12 +103,18 @@ typedef struct {
                                   such particles -- mostly inside dense matter -- collide
                                   together.  Results are unchanged.  0 -> 8; 1 disables;
                                   at most 33 (33: park every collision)                    */
-    int32_t xs_search;         /* cross-section bin search: 0 a bucket
-                                  index over the keys' bit patterns narrows a binary search;
-                                  1 plain binary search over the table; 2 the paper's
-                                  cached-index search -- a linear walk from the particle's
-                                  previous bin (history mode, u8 block-map meshes; others
-                                  use 0).  All three return the same bin.                 */
+    int32_t xs_search;         /* cross-section bin search: 0 direct
+                                  bucket rows -- a bucket index over the keys' bit patterns
+                                  (about four buckets per key) whose every bucket stores the
+                                  three (key, value) pairs its energies can need, so a
+                                  lookup is one dependent 48 B load (built when every
+                                  bucket spans at most one key, else as 3); 1 plain binary
+                                  search over the table; 2 the paper's cached-index search
+                                  -- a linear walk from the particle's previous bin
+                                  (history mode, u8 block-map meshes; others use 3); 3 the
+                                  bucket index alone (the index pair, then the pairs: two
+                                  dependent loads; a binary search inside buckets holding
+                                  more than one key).  All four return the same bin.      */
     /* physics variants (DESIGN.md §4 R30-R32; the defaults are the paper's problem)      */
     int32_t boundary;          /* 0 reflective on all four sides; 1 vacuum: a
                                   facet on the mesh boundary ends the history (escape)     */
@@ -140,6 +146,13 @@ typedef struct {
                                   parked particles while the others still run phase 1
                                   (they join when their range is exhausted).  Results are
                                   unchanged.  u8 block-map meshes, default kernel options */
+    int32_t xs_l2_persist;     /* 1: while the tracking kernels run, an L2 access-policy
+                                  window on the context stream marks the cross-section
+                                  tables persisting (large lookup tables can
+                                  become the bottleneck), with a device-wide persisting
+                                  carve-out of up to the tables' size set at
+                                  nt_load_cross_sections and released at nt_destroy;
+                                  0: no window (default)                                  */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,
@@ -276,6 +289,9 @@ int64_t nt_debug_alloc_count(void);
  * tally buffers.  With x-slabs (decomposition 1) only the rank's columns plus a one-column
  * halo are stored, so this scales as 1/nranks.  -1 for a NULL context. */
 int64_t nt_debug_mesh_bytes(const nt_ctx *ctx);
+/* Which loaded tables have direct bucket rows (xs_search 0): bit 0 scatter, bit 1 capture;
+ * -1 for a NULL context. */
+int32_t nt_debug_xs_rows(const nt_ctx *ctx);
 /* out[2i], out[2i+1] = threefry2x64_20(ctr = {in[4i], in[4i+1]}, key = {in[4i+2], in[4i+3]}). */
 nt_status nt_debug_threefry(nt_ctx *ctx, const uint64_t *in, int64_t n, uint64_t *out);
 /* Microscopic XS from the loaded tables: out_s[i], out_a[i] at energies[i] (no clamp

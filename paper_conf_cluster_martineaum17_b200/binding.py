@@ -32,7 +32,7 @@ EXPORTS = ["nt_abi_version", "nt_build_info", "nt_status_string", "nt_options_de
            "nt_read_particles", "nt_write_particles", "nt_slab_record_bytes", "nt_slab_begin",
            "nt_slab_round", "nt_slab_export", "nt_slab_import", "nt_slab_end", "nt_particle_slots",
            "nt_debug_threefry", "nt_debug_xs", "nt_debug_alloc_count",
-           "nt_debug_mesh_bytes"]
+           "nt_debug_mesh_bytes", "nt_debug_xs_rows"]
 
 
 class NeutralError(RuntimeError):
@@ -55,7 +55,7 @@ class Options(C.Structure):
                 ("roulette", C.c_int32), ("decomposition", C.c_int32),
                 ("roulette_weight", C.c_double), ("hot_x0", C.c_int32), ("hot_y0", C.c_int32),
                 ("hot_nx", C.c_int32), ("hot_ny", C.c_int32), ("particle_layout", C.c_int32),
-                ("fused_consumers", C.c_int32)]
+                ("fused_consumers", C.c_int32), ("xs_l2_persist", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -122,6 +122,7 @@ def lib():
             "nt_debug_xs": ([vp, vp, i64, vp, vp], C.c_int),
             "nt_debug_alloc_count": ([], i64),
             "nt_debug_mesh_bytes": ([vp], i64),
+            "nt_debug_xs_rows": ([vp], C.c_int32),
         }
         for name, (args, res) in sigs.items():
             f = getattr(L, name)
@@ -189,7 +190,7 @@ class Tracker:
                  defer_below: int = 0, xs_search: int = 0, boundary: int = 0,
                  analog: int = 0, roulette: int = 0, roulette_weight: float = 0.0,
                  decomposition: int = 0, hot_window=(0, 0, 0, 0), particle_layout: int = 0,
-                 fused_consumers: int = 0):
+                 fused_consumers: int = 0, xs_l2_persist: int = 0):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -218,6 +219,7 @@ class Tracker:
         o.hot_x0, o.hot_y0, o.hot_nx, o.hot_ny = hot_window
         o.particle_layout = particle_layout
         o.fused_consumers = fused_consumers
+        o.xs_l2_persist = xs_l2_persist
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:
@@ -351,6 +353,10 @@ class Tracker:
     def mesh_bytes(self) -> int:
         """Device bytes held for the mesh (density + tally buffers)."""
         return int(lib().nt_debug_mesh_bytes(self._h))
+
+    def xs_rows(self) -> int:
+        """Bit mask of the loaded tables with direct bucket rows (1 scatter, 2 capture)."""
+        return int(lib().nt_debug_xs_rows(self._h))
 
     def debug_threefry(self, inputs: np.ndarray) -> np.ndarray:
         inp = np.ascontiguousarray(inputs, dtype=np.uint64).reshape(-1, 4)

@@ -99,7 +99,9 @@ struct nt_ctx {
   // tables
   DevBuf xs;
   size_t xs_bytes = 0;                   // bytes of xs in use (keys, values, indexes, pairs)
+  size_t xs_persist_bytes = 0;           // xs_l2_persist: the device's persisting L2 carve-out
   Tables tables{};
+  const double2* xs_row[2] = {nullptr, nullptr};   // direct bucket rows (xs_search 0), if built
   // particles
   int64_t n_total = 0, first_id = 0, n_local = 0;
   uint64_t seed = 0;
@@ -129,6 +131,54 @@ struct nt_ctx {
 };
 
 namespace {
+
+// The tables as the kernels see them under the xs_search option: 0 the direct bucket rows
+// where the loader could build them (else the bucket index), 1 no index (plain binary
+// search), 2 and 3 the bucket index (2's walk is a kernel instantiation).
+// xs_l2_persist: an L2 access-policy window marks the cross-section buffer persisting on the
+// context stream while the step's tracking kernels run (cleared afterwards, also on error
+// paths), so the table lines are not evicted by the tally and particle-store traffic.  The
+// device-wide persisting carve-out is sized at nt_load_cross_sections.
+struct XsWindow {
+  nt_ctx* c;
+  bool on = false;
+  explicit XsWindow(nt_ctx* ctx);
+  ~XsWindow();
+};
+
+static Tables xs_tables(const nt_ctx* c) {
+  Tables t = c->tables;
+  if (c->opt.xs_search == 1) {
+    t.s.nb = 0;
+    t.c.nb = 0;
+  } else if (c->opt.xs_search == 0) {
+    t.s.row = c->xs_row[0];
+    t.c.row = c->xs_row[1];
+  }
+  return t;
+}
+
+XsWindow::XsWindow(nt_ctx* ctx) : c(ctx) {
+  if (!c->opt.xs_l2_persist || c->xs_bytes == 0 || c->xs_persist_bytes == 0) return;
+  int maxwin = 0;
+  cudaDeviceGetAttribute(&maxwin, cudaDevAttrMaxAccessPolicyWindowSize, c->device);
+  cudaStreamAttrValue v{};
+  v.accessPolicyWindow.base_ptr = c->xs.p;
+  v.accessPolicyWindow.num_bytes = c->xs_bytes < (size_t)maxwin ? c->xs_bytes : (size_t)maxwin;
+  const double r = (double)c->xs_persist_bytes / (double)v.accessPolicyWindow.num_bytes;
+  v.accessPolicyWindow.hitRatio = (float)(r < 1.0 ? r : 1.0);
+  v.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+  v.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+  on = cudaStreamSetAttribute(c->stream, cudaStreamAttributeAccessPolicyWindow, &v) == cudaSuccess;
+  if (!on) cudaGetLastError();
+}
+
+XsWindow::~XsWindow() {
+  if (!on) return;
+  cudaStreamAttrValue v{};
+  v.accessPolicyWindow.num_bytes = 0;     // no window: later work on the stream is unaffected
+  cudaStreamSetAttribute(c->stream, cudaStreamAttributeAccessPolicyWindow, &v);
+}
 
 nt_status fail(nt_ctx* c, nt_status s, const char* fmt, ...) {
   if (c) {
@@ -271,7 +321,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.refill_min > 32) opt.refill_min = 32;
   if (opt.defer_below == 0) opt.defer_below = def.defer_below;
   if (opt.defer_below < 0 || opt.defer_below > 33) return NT_ERR_ARG;
-  if (opt.xs_search < 0 || opt.xs_search > 2) return NT_ERR_ARG;
+  if (opt.xs_search < 0 || opt.xs_search > 3) return NT_ERR_ARG;
   if (opt.boundary < 0 || opt.boundary > 1 || opt.analog_absorption < 0 ||
       opt.analog_absorption > 1 || opt.roulette < 0 || opt.roulette > 1)
     return NT_ERR_ARG;
@@ -285,6 +335,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
     return NT_ERR_ARG;
   if (opt.particle_layout < 0 || opt.particle_layout > 1) return NT_ERR_ARG;
   if (opt.fused_consumers < 0 || opt.fused_consumers > 8) return NT_ERR_ARG;
+  if (opt.xs_l2_persist < 0 || opt.xs_l2_persist > 1) return NT_ERR_ARG;
   if (opt.tally_mode == 3 && (opt.hot_x0 < 0 || opt.hot_y0 < 0 || opt.hot_nx < 1 || opt.hot_ny < 1 ||
                               (int64_t)opt.hot_nx * opt.hot_ny > kHotCells))
     return NT_ERR_ARG;
@@ -336,6 +387,10 @@ nt_status nt_destroy(nt_ctx* c) {
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
   if (c->evs) event_state_destroy(c->evs);
+  if (c->xs_persist_bytes) {            // xs_l2_persist: release the persisting lines and carve-out
+    cudaCtxResetPersistingL2Cache();
+    cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, 0);
+  }
   for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->tally_full, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
                     &c->sort_tmp, &c->backup, &c->stats_d, &c->aos})
@@ -566,7 +621,20 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
       kvh[t][2 * (size_t)j + 1] = h[2 * t + 1][q];
     }
   }
-  size_t off[8], total = 0;
+  // direct bucket rows (xs_search 0): bucket b -> the pairs idx[b], idx[b] + 1, idx[b] + 2,
+  // built only when every bucket spans at most one key (then the bin is idx[b] or idx[b] + 1)
+  std::vector<double> rows[2];
+  for (int t = 0; t < 2; ++t) {
+    const int64_t nb = nbk[t];
+    if (nb <= 0) continue;
+    bool ok = true;
+    for (int64_t b = 0; b < nb && ok; ++b) ok = idx[t][(size_t)b + 1] - idx[t][(size_t)b] <= 1u;
+    if (!ok) continue;
+    rows[t].resize((size_t)nb * 6);
+    for (int64_t b = 0; b < nb; ++b)
+      std::memcpy(&rows[t][(size_t)b * 6], &kvh[t][2 * (size_t)idx[t][(size_t)b]], 48);
+  }
+  size_t off[10], total = 0;
   for (int k = 0; k < 4; ++k) {
     off[k] = total;
     total += align256((size_t)len[k] * 8);
@@ -579,6 +647,10 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     off[6 + t] = total;
     total += align256(kvh[t].size() * 8);
   }
+  for (int t = 0; t < 2; ++t) {
+    off[8 + t] = total;
+    total += align256(rows[t].size() * 8);
+  }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k], (size_t)len[k] * 8,
@@ -589,15 +661,34 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
                                  cudaMemcpyHostToDevice, c->stream));
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[6 + t], kvh[t].data(), kvh[t].size() * 8,
                                cudaMemcpyHostToDevice, c->stream));
+    if (!rows[t].empty())
+      NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[8 + t], rows[t].data(), rows[t].size() * 8,
+                                 cudaMemcpyHostToDevice, c->stream));
   }
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   c->xs_bytes = total;
+  c->xs_persist_bytes = 0;
+  if (c->opt.xs_l2_persist) {
+    int maxp = 0;
+    cudaDeviceGetAttribute(&maxp, cudaDevAttrMaxPersistingL2CacheSize, c->device);
+    const size_t want = total < (size_t)maxp ? total : (size_t)maxp;
+    if (want > 0 && cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, want) == cudaSuccess) {
+      size_t got = 0;
+      cudaDeviceGetLimit(&got, cudaLimitPersistingL2CacheSize);
+      c->xs_persist_bytes = got;
+    } else {
+      cudaGetLastError();
+    }
+  }
   Table* T[2] = {&c->tables.s, &c->tables.c};
   for (int t = 0; t < 2; ++t) {
     T[t]->k = reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t]);
     T[t]->v = reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t + 1]);
     T[t]->idx = reinterpret_cast<const uint32_t*>(c->xs.as<char>() + off[4 + t]);
     T[t]->kv = reinterpret_cast<const double2*>(c->xs.as<char>() + off[6 + t]);
+    T[t]->row = nullptr;                 // selected per launch (xs_tables)
+    c->xs_row[t] = rows[t].empty() ? nullptr
+                                   : reinterpret_cast<const double2*>(c->xs.as<char>() + off[8 + t]);
     T[t]->n = (int32_t)len[2 * t];
     T[t]->nb = nbk[t];
     T[t]->shift = shift[t];
@@ -712,11 +803,7 @@ static TrackParams make_params(nt_ctx* c, double dt) {
   tp.mesh.wx = c->W;
   tp.mesh.wy = c->H;
   tp.mesh.ny = c->ny;
-  tp.xs = c->tables;
-  if (c->opt.xs_search == 1) {          // plain binary search over the whole table
-    tp.xs.s.nb = 0;
-    tp.xs.c.nb = 0;
-  }
+  tp.xs = xs_tables(c);
   tp.ph = c->ph;
   tp.p = c->p;
   tp.n = c->n_local;
@@ -1140,6 +1227,7 @@ nt_status nt_run_timestep(nt_ctx* c, double dt, nt_step_stats* stats) {
   const bool det = c->opt.deterministic != 0;
   const TrackParams tp = make_params(c, dt);
   {
+    XsWindow xw(c);
     const nt_status st = c->opt.decomposition == 1 ? run_slab_nccl(c, tp, launches)
                          : det ? run_det(c, tp, launches) : track_range(c, tp, false, launches);
     if (st != NT_OK) return st;
@@ -1363,6 +1451,11 @@ int64_t nt_debug_mesh_bytes(const nt_ctx* c) {
   return b;
 }
 
+int32_t nt_debug_xs_rows(const nt_ctx* c) {
+  if (!c) return -1;
+  return (c->xs_row[0] ? 1 : 0) | (c->xs_row[1] ? 2 : 0);
+}
+
 nt_status nt_debug_threefry(nt_ctx* c, const uint64_t* in, int64_t n, uint64_t* out) {
   if (!c || !in || !out || n < 0) return NT_ERR_ARG;
   cudaSetDevice(c->device);
@@ -1387,7 +1480,7 @@ nt_status nt_debug_xs(nt_ctx* c, const double* energies, int64_t n, double* out_
   NT_CUDA(c, a.ensure((size_t)n * 8 + 8));
   NT_CUDA(c, b.ensure((size_t)n * 16 + 16));
   NT_CUDA(c, copy_in(a.p, energies, (size_t)n * 8, c->stream));
-  launch_xs_debug(c->tables, a.as<double>(), n, b.as<double>(), b.as<double>() + n, c->stream);
+  launch_xs_debug(xs_tables(c), a.as<double>(), n, b.as<double>(), b.as<double>() + n, c->stream);
   NT_CUDA(c, cudaGetLastError());
   NT_CUDA(c, cudaMemcpyAsync(out_s, b.p, (size_t)n * 8, cudaMemcpyDefault, c->stream));
   NT_CUDA(c, cudaMemcpyAsync(out_a, b.as<double>() + n, (size_t)n * 8, cudaMemcpyDefault, c->stream));

@@ -112,6 +112,8 @@ struct Table {
   const double2* __restrict__ kv;   // (k[i], v[i]) interleaved, [n + 1] (last entry repeats
                                     // n - 1): one 48 B run holds the two bins a bucket spans
   const uint32_t* __restrict__ idx; // [nb + 1]
+  const double2* __restrict__ row;  // xs_search 0: per bucket b the three pairs kv[idx[b]],
+                                    // kv[idx[b] + 1], kv[idx[b] + 2] (48 B), or nullptr
   uint64_t base;
   int32_t n, nb, shift, pad;
   double kfirst, klast;             // k[0] and k[n-1], as kernel parameters (no load latency)
@@ -448,7 +450,26 @@ __device__ __forceinline__ double xs_end(const Table& T, XsPre r) {
   return v0 + t * (v1 - v0);
 }
 
+// Direct bucket rows (xs_search 0, the default): the loader copies, for every bucket b, the three pairs a
+// bucket spanning at most one key can need into row[3b .. 3b+2], and builds rows only when
+// every bucket spans at most one key.  Then the lookup is ONE dependent load (the 48 B row)
+// instead of two (the index pair, then the run): the index and the pairs are "staged" into
+// one L2-resident structure addressed by the energy's bits (scatter history 8.26 -> 7.42 ms,
+// scatter event 17.8 -> 15.4 ms; profiles/ab/r02_ab19_xs_rows.txt).  Same bin and the same
+// lerp expression as xs_end, hence the same result.
+__device__ __forceinline__ double xs_row(const Table& T, double e) {
+  const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
+  const double2* r = T.row + 3 * b;
+  const double2 a = __ldg(r), m = __ldg(r + 1), c = __ldg(r + 2);
+  const bool up = m.x <= e;
+  const double k0 = up ? m.x : a.x, v0 = up ? m.y : a.y;
+  const double k1 = up ? c.x : m.x, v1 = up ? c.y : m.y;
+  const double t = (e - k0) / (k1 - k0);
+  return v0 + t * (v1 - v0);
+}
+
 __device__ __forceinline__ double xs_lookup(const Table& T, double e) {
+  if (T.row != nullptr && e < T.klast) return xs_row(T, e);   // uniform branch (kernel param)
   return xs_end(T, xs_begin(T, e));
 }
 

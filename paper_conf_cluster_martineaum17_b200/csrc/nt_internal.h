@@ -73,8 +73,8 @@ void launch_inject(const InjectParams& ip, cudaStream_t s);
 // production u8 + block map only -- <= 72 registers (7 per SM).
 // tally_mode 1/2/3 (production u8 + block map only): warp-aggregated flushes / CAS-emulated
 // fp64 add / shared-memory hot window (tp.hot_*).
-// xs_search 2 (u8 + block map only): the cached-bin linear walk; 1 is a data change (the
-// caller passes tables without bucket index, nb = 0).
+// xs_search 2 (u8 + block map only): the cached-bin linear walk; 0, 1 and 3 are data
+// changes (the caller passes tables with direct rows / without bucket index / index only).
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
                     int xs_search, bool slab, cudaStream_t s);
 // particle_layout 1: copy the particle store SoA -> AoS (to_aos) or back, particles [0, n)
