@@ -193,6 +193,9 @@ def parse():
     ap.add_argument("--xs-search", type=int, default=0,
                     help="0 direct bucket rows (one dependent load per lookup), 1 plain binary search, "
                          "2 cached-bin linear walk, 3 bucket index alone (two dependent loads)")
+    ap.add_argument("--resume-prefetch", type=int, default=-1,
+                    help="history mode: 1 parked records + cp.async resume ring, 0 particle store + "
+                         "index queue, -1 the library default")
     ap.add_argument("--xs-l2-persist", type=int, default=0,
                     help="1: L2 persisting access-policy window over the XS tables while tracking")
     ap.add_argument("--table-size", type=int, default=0,
@@ -345,7 +348,8 @@ def main():
                          tally_mode=a.tally_mode, defer_below=a.defer_below,
                          xs_search=a.xs_search, hot_window=hot_window(cfg),
                          particle_layout=a.particle_layout, fused_consumers=a.fused_consumers,
-                         xs_l2_persist=a.xs_l2_persist)
+                         xs_l2_persist=a.xs_l2_persist,
+                         resume_prefetch=None if a.resume_prefetch < 0 else a.resume_prefetch)
     density = wl.density(cfg)
     tables = wl.tables(cfg)
     tr.init_mesh(cfg.nx, cfg.ny, cfg.width, cfg.height, density)

@@ -153,6 +153,13 @@ typedef struct {
                                   carve-out of up to the tables' size set at
                                   nt_load_cross_sections and released at nt_destroy;
                                   0: no window (default)                                  */
+    int32_t resume_prefetch;   /* history mode, production, default kernel options: 1 a
+                                  parked particle's state is written as a queue-ordered
+                                  144 B record, and the second launch streams the records
+                                  into a per-warp shared-memory ring with cp.async one
+                                  batch ahead of use (refills of resumed particles read
+                                  shared memory); 0 the state goes to the particle store
+                                  and a queue of indices.  Results are unchanged.         */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

@@ -55,7 +55,8 @@ class Options(C.Structure):
                 ("roulette", C.c_int32), ("decomposition", C.c_int32),
                 ("roulette_weight", C.c_double), ("hot_x0", C.c_int32), ("hot_y0", C.c_int32),
                 ("hot_nx", C.c_int32), ("hot_ny", C.c_int32), ("particle_layout", C.c_int32),
-                ("fused_consumers", C.c_int32), ("xs_l2_persist", C.c_int32)]
+                ("fused_consumers", C.c_int32), ("xs_l2_persist", C.c_int32),
+                ("resume_prefetch", C.c_int32)]
 
 
 class StepStats(C.Structure):
@@ -190,7 +191,7 @@ class Tracker:
                  defer_below: int = 0, xs_search: int = 0, boundary: int = 0,
                  analog: int = 0, roulette: int = 0, roulette_weight: float = 0.0,
                  decomposition: int = 0, hot_window=(0, 0, 0, 0), particle_layout: int = 0,
-                 fused_consumers: int = 0, xs_l2_persist: int = 0):
+                 fused_consumers: int = 0, xs_l2_persist: int = 0, resume_prefetch: int | None = None):
         L = lib()
         o = Options()
         L.nt_options_default(C.byref(o))
@@ -220,6 +221,8 @@ class Tracker:
         o.particle_layout = particle_layout
         o.fused_consumers = fused_consumers
         o.xs_l2_persist = xs_l2_persist
+        if resume_prefetch is not None:          # None: the library default
+            o.resume_prefetch = resume_prefetch
         h = C.c_void_p()
         st = L.nt_create(C.byref(o), C.byref(h))
         if st != NT_OK:

@@ -109,6 +109,8 @@ struct nt_ctx {
   DevBuf aos;                            // particle_layout 1: AoS records during the step
   Soa p{};
   int32_t* defer_q = nullptr;            // regime-parking queue (in soa)
+  DevBuf park_rec;                       // resume_prefetch: queue-ordered parked records
+  int64_t park_cap = 0;
   // x-slab decomposition (decomposition 1)
   int64_t n_cap = 0;                     // particle-store capacity (n_total with slabs)
   int32_t slab_lo = 0, slab_hi = 0;      // owned mesh columns
@@ -286,6 +288,7 @@ nt_status nt_options_default(nt_options* opt) {
   opt->det_batch = 65536;
   opt->refill_min = 4;
   opt->defer_below = 8;
+  opt->resume_prefetch = 1;
   return NT_OK;
 }
 
@@ -336,6 +339,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.particle_layout < 0 || opt.particle_layout > 1) return NT_ERR_ARG;
   if (opt.fused_consumers < 0 || opt.fused_consumers > 8) return NT_ERR_ARG;
   if (opt.xs_l2_persist < 0 || opt.xs_l2_persist > 1) return NT_ERR_ARG;
+  if (opt.resume_prefetch < 0 || opt.resume_prefetch > 1) return NT_ERR_ARG;
   if (opt.tally_mode == 3 && (opt.hot_x0 < 0 || opt.hot_y0 < 0 || opt.hot_nx < 1 || opt.hot_ny < 1 ||
                               (int64_t)opt.hot_nx * opt.hot_ny > kHotCells))
     return NT_ERR_ARG;
@@ -393,7 +397,7 @@ nt_status nt_destroy(nt_ctx* c) {
   }
   for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->tally_full, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
-                    &c->sort_tmp, &c->backup, &c->stats_d, &c->aos})
+                    &c->sort_tmp, &c->backup, &c->stats_d, &c->aos, &c->park_rec})
     b->release();
   if (c->stats_h) cudaFreeHost(c->stats_h);
   for (auto& ev : c->ev)
@@ -623,16 +627,14 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   }
   // direct bucket rows (xs_search 0): bucket b -> the pairs idx[b], idx[b] + 1, idx[b] + 2,
   // built only when every bucket spans at most one key (then the bin is idx[b] or idx[b] + 1)
-  std::vector<double> rows[2];
+  // (checked here, copied on the device from the interleaved pairs: no extra H2D bytes)
+  int64_t nrows[2] = {0, 0};
   for (int t = 0; t < 2; ++t) {
     const int64_t nb = nbk[t];
     if (nb <= 0) continue;
     bool ok = true;
     for (int64_t b = 0; b < nb && ok; ++b) ok = idx[t][(size_t)b + 1] - idx[t][(size_t)b] <= 1u;
-    if (!ok) continue;
-    rows[t].resize((size_t)nb * 6);
-    for (int64_t b = 0; b < nb; ++b)
-      std::memcpy(&rows[t][(size_t)b * 6], &kvh[t][2 * (size_t)idx[t][(size_t)b]], 48);
+    if (ok) nrows[t] = nb;
   }
   size_t off[10], total = 0;
   for (int k = 0; k < 4; ++k) {
@@ -649,7 +651,7 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   }
   for (int t = 0; t < 2; ++t) {
     off[8 + t] = total;
-    total += align256(rows[t].size() * 8);
+    total += align256((size_t)nrows[t] * 48);
   }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
@@ -661,9 +663,10 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
                                  cudaMemcpyHostToDevice, c->stream));
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[6 + t], kvh[t].data(), kvh[t].size() * 8,
                                cudaMemcpyHostToDevice, c->stream));
-    if (!rows[t].empty())
-      NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[8 + t], rows[t].data(), rows[t].size() * 8,
-                                 cudaMemcpyHostToDevice, c->stream));
+    if (nrows[t] > 0)
+      launch_xs_rows(reinterpret_cast<const double2*>(c->xs.as<char>() + off[6 + t]),
+                     reinterpret_cast<const uint32_t*>(c->xs.as<char>() + off[4 + t]), nrows[t],
+                     reinterpret_cast<double2*>(c->xs.as<char>() + off[8 + t]), c->stream);
   }
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   c->xs_bytes = total;
@@ -687,7 +690,7 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     T[t]->idx = reinterpret_cast<const uint32_t*>(c->xs.as<char>() + off[4 + t]);
     T[t]->kv = reinterpret_cast<const double2*>(c->xs.as<char>() + off[6 + t]);
     T[t]->row = nullptr;                 // selected per launch (xs_tables)
-    c->xs_row[t] = rows[t].empty() ? nullptr
+    c->xs_row[t] = nrows[t] == 0 ? nullptr
                                    : reinterpret_cast<const double2*>(c->xs.as<char>() + off[8 + t]);
     T[t]->n = (int32_t)len[2 * t];
     T[t]->nb = nbk[t];
@@ -721,6 +724,14 @@ static cudaError_t alloc_soa(nt_ctx* c, int64_t n) {
   c->free_q = reinterpret_cast<int32_t*>(q); q += b4;
   c->p.gid = reinterpret_cast<int64_t*>(q); q += b8;
   c->p.status = reinterpret_cast<uint8_t*>(q);
+  // resume_prefetch: one record per particle at most (a particle is parked once per step),
+  // plus a batch of slack so the last batch's copies stay inside the buffer
+  if (c->opt.resume_prefetch && c->opt.mode != NT_MODE_EVENT && !c->opt.deterministic) {
+    const int64_t cap = ((int64_t)N + kRingB + 3) / 4 * 4;
+    e = c->park_rec.ensure((size_t)cap * (kParkF64 * 8 + kParkU32 * 4));
+    if (e != cudaSuccess) return e;
+    c->park_cap = cap;
+  }
   return cudaSuccess;
 }
 
@@ -918,9 +929,23 @@ static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uin
     NT_CUDA(c, cudaGetLastError());
     return NT_OK;
   }
+  // resume_prefetch: record parking + the phase-2 ring, default kernel options only (the
+  // conditions mirror the kernel selection in nt_kernels.cu history_fn)
+  const bool ring = c->opt.resume_prefetch && c->park_cap > 0 && !det && !slab && !src_count &&
+                    !var && !aos && c->dens_fmt == kDensU8 && c->blk_n > 0 &&
+                    c->opt.tally_mode == 0 && c->opt.xs_search != 2 && c->opt.ctas_per_sm < 7;
   for (int ph = 1; ph <= 2; ++ph) {
     TrackParams p = bp;
     p.phase = ph;
+    int g = grid;
+    if (ring) {
+      p.park_rec = c->park_rec.as<double>();
+      p.park_cap = c->park_cap;
+      if (ph == 2) {                 // the ring's shared memory may lower the residency
+        const int per_sm = history_ring_ctas_per_sm(c->tiled != 0);
+        if (per_sm > 0 && per_sm * c->sm_count < g) g = per_sm * c->sm_count;
+      }
+    }
     if (slab) {
       p.slab_lo = c->slab_lo;
       p.slab_hi = c->slab_hi;
@@ -940,7 +965,7 @@ static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uin
       p.park_count = qlen;
       p.park_coll_below = c->opt.defer_below;
     }
-    launch_history(p, det, grid, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, slab,
+    launch_history(p, det, g, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, slab,
                    c->stream);
     ++launches;
   }

@@ -333,6 +333,16 @@ __device__ __forceinline__ uint32_t dens_load_blk(const Mesh& M, const uint8_t* 
 }
 
 // Cross-CTA hand-over within one launch (fused phases): volatile / L2-only accesses.
+// cp.async (Ampere+ LDGSTS): 16 bytes global -> shared, L2 only (.cg), completion tracked per
+// thread by commit groups
+__device__ __forceinline__ void cp_async16(void* smem, const void* gmem) {
+  const unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
+  asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" :: "r"(sa), "l"(gmem) : "memory");
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+__device__ __forceinline__ void cp_async_wait_all() { asm volatile("cp.async.wait_all;" ::: "memory"); }
+__device__ __forceinline__ void cp_async_wait_group1() { asm volatile("cp.async.wait_group 1;" ::: "memory"); }
+
 __device__ __forceinline__ int32_t ld_volatile(const int32_t* p) {
   return *reinterpret_cast<const volatile int32_t*>(p);
 }

@@ -28,6 +28,11 @@ struct TrackParams {
   const unsigned long long* resume_count;
   int32_t* park_q;            // out-queue of parked local indices
   unsigned long long* park_count;
+  // resume_prefetch (kQ kernels): parks write queue-ordered records (kParkF64 f64 columns,
+  // then kParkU32 u32 columns, park_cap entries each) instead of the particle store + queue
+  // index; phase 2 streams them into a per-warp shared-memory ring with cp.async
+  double* park_rec;
+  int64_t park_cap;
   // fused phases (fused_consumers > 0): one launch; CTAs [0, coll_ctas) start as consumers
   // of park_q (entries published as index + 1 after a fence), the others produce (phase 1)
   // and turn consumer when their range is exhausted
@@ -87,6 +92,11 @@ void launch_slab_pack(const TrackParams& tp, const int32_t* out_q, int64_t n, Sl
 void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32_t* free_slots,
                         int64_t n_free, int64_t base, int32_t* arr_q, cudaStream_t s);
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally);
+// direct bucket rows (xs_search 0): row[3b .. 3b+2] = kv[idx[b] .. idx[b]+2], b < nb
+void launch_xs_rows(const double2* kv, const uint32_t* idx, int64_t nb, double2* row,
+                    cudaStream_t s);
+// resident CTAs per SM of the resume_prefetch kernel with its ring (phase 2)
+int history_ring_ctas_per_sm(bool tiled);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
                       unsigned long long n, double* tally, cudaStream_t s);
 void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s);
@@ -106,6 +116,13 @@ void launch_stats_to_f64(const unsigned long long* su, const double* sf, double*
                          cudaStream_t s);
 
 constexpr int kHistoryBlock = 128;
+// resume ring (history kernel, resume_prefetch): a parked record is 15 f64 (x, y, ox, oy,
+// exn, eyn, E, w, n_mfp, census distance, acc, dstep, sigma_t, p_a, H) + 6 u32 (cx, cy, ctr,
+// facets, collisions, local index) = 144 B; claims and copies move batches of kRingB
+// records, and each warp holds two batches (one being consumed, one in flight).
+constexpr int kParkF64 = 15, kParkU32 = 6, kRingB = 12;
+constexpr int kRingHalfBytes = kRingB * (kParkF64 * 8 + kParkU32 * 4);     // 1728
+constexpr int kRingCtaBytes = 2 * kRingHalfBytes * (kHistoryBlock / 32);   // 13824
 constexpr int kHotCells = 2048;     // tally_mode 3: cells of the shared-memory hot window (16 KB)
 // history kernel: events a lane may run between two warp votes (refill checks); the A/B
 // sweep in profiles/ab/r01_ab4_history_variants.md chose 256

@@ -91,8 +91,14 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 // 2 the fp64 add emulated with a 64-bit compare-and-swap loop (how fp64 atomics were done
 // before native ones); 3 a per-CTA shared-memory copy of a hot window of cells
 // (privatisation), merged into the tally with one RED per cell at the end.
+//
+// kQ (resume_prefetch): a park writes the particle's register state as a queue-ordered record
+// (TrackParams::park_rec) instead of the particle store + a queue index, and the resume
+// phase streams those records into a per-warp shared-memory ring with cp.async, one batch
+// ahead of use, so a refill of parked particles costs shared-memory loads instead of a
+// dependent chain of global loads (queue index, then the state, then the XS lookups).
 template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, int kTally, bool kXsWalk,
-          bool kVar, bool kSlab, bool kAoS = false, bool kFused = false>
+          bool kVar, bool kSlab, bool kAoS = false, bool kFused = false, bool kQ = false>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
 history_kernel(const __grid_constant__ TrackParams P) {
   // particle-store field f of local particle idx: structure of arrays, or -- the
@@ -104,6 +110,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
   static_assert(!(kTally == 3 && kSlab), "hot window: replicated meshes only");
   static_assert(!(kAoS && kSlab), "AoS particle store: replicated meshes only");
   static_assert(!(kFused && (kSlab || kDet || kAoS)), "fused phases: production, replicated, SoA");
+  static_assert(!(kQ && (kSlab || kDet || kAoS || kFused || kXsWalk)),
+                "resume ring: production, replicated, SoA, two launches, table lookups");
   // Statistics: u32 counters per warp in shared memory (native shared atomics); f64 sums in
   // per-thread slots in global memory (touched only when a history ends), so the CTA keeps
   // almost no shared memory and the L1 stays free for the density / edge gathers.
@@ -238,6 +246,25 @@ history_kernel(const __grid_constant__ TrackParams P) {
   // takes a new particle.  Used for regime parking (status 2, park_q) and, with x-slabs,
   // for emigrants (status 4, out_q).
   auto park_to = [&](uint8_t st, int32_t* q, unsigned long long* qn) {
+    if constexpr (kQ) {
+      // the register state as record k of the queue-ordered park buffer (status stays 1)
+      const unsigned am = __activemask();
+      const int ld = __ffs(am) - 1;
+      unsigned long long k = 0;
+      if (lane == ld) k = atomicAdd(qn, (unsigned long long)__popc(am));
+      k = __shfl_sync(am, k, ld) + (unsigned long long)__popc(am & lt_mask);
+      const int64_t C = P.park_cap;
+      double* f = P.park_rec + k;
+      uint32_t* u = reinterpret_cast<uint32_t*>(P.park_rec + kParkF64 * C) + k;
+      f[0] = x; f[C] = y; f[2 * C] = ox; f[3 * C] = oy; f[4 * C] = exn; f[5 * C] = eyn;
+      f[6 * C] = e; f[7 * C] = w; f[8 * C] = mfp; f[9 * C] = dcen; f[10 * C] = acc;
+      f[11 * C] = dstep; f[12 * C] = m.st; f[13 * C] = m.pa; f[14 * C] = m.H;
+      u[0] = (uint32_t)cx; u[C] = (uint32_t)cy; u[2 * C] = ctr; u[3 * C] = nf; u[4 * C] = nc;
+      u[5 * C] = (uint32_t)i;
+      (void)st; (void)q;
+      active = false;
+      return;
+    }
     (*PP(x, i)) = x;
     (*PP(y, i)) = y;
     (*PP(ox, i)) = ox;
@@ -280,6 +307,63 @@ history_kernel(const __grid_constant__ TrackParams P) {
     if (ox == 0.0) { exn = d_inf(); iox = d_inf(); }
     if (oy == 0.0) { eyn = d_inf(); ioy = d_inf(); }
   };
+
+  // ---- resume ring (kQ, phase 2): per warp two halves of kRingB records in shared memory ----
+  // rh: the half being consumed (rpos of rcnt records used); the other half receives the
+  // batch claimed at the previous swap (fcnt records, cp.async in flight); cb_raw (lane 0)
+  // is the next batch's claim, consumed at the next swap -- so neither the claim's atomic
+  // nor the copies stall a refill.
+  extern __shared__ __align__(16) unsigned char dsm[];
+  unsigned char* ring = dsm + (size_t)wid * 2 * kRingHalfBytes;
+  // ring state packed in one register (live through phase 1 too): bit 0 rh, bits 1-7 rpos,
+  // 8-15 rcnt, 16-23 fcnt; cb_raw keeps the claim's low word (positions < 2^31)
+  uint32_t rstate = 0;
+  uint32_t cb_raw = 0;
+  auto rvalid = [&](unsigned long long b) -> int {
+    return b < span2 ? (int)(span2 - b < (unsigned long long)kRingB ? span2 - b : kRingB) : 0;
+  };
+  // all 32 lanes: copy records [b, b + kRingB) into half hf (16-byte chunks, coalesced)
+  auto ring_issue = [&](unsigned long long b, int hf) __attribute__((always_inline)) {
+    const int64_t C = P.park_cap;
+    unsigned char* hb = ring + hf * kRingHalfBytes;
+    constexpr int kF = kParkF64 * (kRingB / 2), kU = kParkU32 * (kRingB / 4);
+    for (int ck = lane; ck < kF + kU; ck += 32) {
+      const void* src;
+      unsigned char* dst;
+      if (ck < kF) {
+        const int col = ck / (kRingB / 2), part = ck % (kRingB / 2);
+        src = P.park_rec + col * C + (int64_t)b + 2 * part;
+        dst = hb + col * (kRingB * 8) + part * 16;
+      } else {
+        const int c2 = ck - kF, col = c2 / (kRingB / 4), part = c2 % (kRingB / 4);
+        src = reinterpret_cast<const uint32_t*>(P.park_rec + kParkF64 * C) + col * C + (int64_t)b + 4 * part;
+        dst = hb + kParkF64 * kRingB * 8 + col * (kRingB * 4) + part * 16;
+      }
+      cp_async16(dst, src);
+    }
+    cp_async_commit();
+  };
+  if constexpr (kQ) {
+    if (resume) {
+      unsigned long long b0 = 0;
+      if (lane == 0) b0 = atomicAdd(P.counter, (unsigned long long)kRingB);
+      b0 = __shfl_sync(kFull, b0, 0);
+      const int rcnt = rvalid(b0);
+      if (rcnt > 0) ring_issue(b0, 0);
+      unsigned long long b1 = 0;
+      if (lane == 0) b1 = atomicAdd(P.counter, (unsigned long long)kRingB);
+      b1 = __shfl_sync(kFull, b1, 0);
+      const int fcnt = rvalid(b1);
+      if (fcnt > 0) {
+        ring_issue(b1, 1);
+        if (lane == 0) cb_raw = (uint32_t)atomicAdd(P.counter, (unsigned long long)kRingB);
+      }
+      if (fcnt > 0) cp_async_wait_group1();   // batch b0 has landed (b1 may be in flight)
+      else cp_async_wait_all();
+      __syncwarp();
+      rstate = ((uint32_t)rcnt << 8) | ((uint32_t)fcnt << 16);
+    }
+  }
 
   for (;;) {
     if constexpr (kFused) {
@@ -344,7 +428,56 @@ history_kernel(const __grid_constant__ TrackParams P) {
     }
     // ---- refill idle lanes with new particles: one atomic per warp ----
     const unsigned idle = __ballot_sync(kFull, !active);
-    if (!consumer && !exhausted && idle != 0u && (__popc(idle) >= P.refill_min || idle == kFull)) {
+    if (kQ && resume) {
+      if (!exhausted && idle != 0u && (__popc(idle) >= P.refill_min || idle == kFull)) {
+        int rh = (int)(rstate & 1u), rpos = (int)((rstate >> 1) & 127u);
+        int rcnt = (int)((rstate >> 8) & 255u), fcnt = (int)((rstate >> 16) & 255u);
+        unsigned need = idle;
+        while (need != 0u) {
+          if (rpos == rcnt) {                  // the consumed half is used up: swap
+            if (fcnt == 0) { exhausted = true; break; }
+            cp_async_wait_all();
+            __syncwarp();
+            rh ^= 1;
+            rpos = 0;
+            rcnt = fcnt;
+            const unsigned long long cb = __shfl_sync(kFull, cb_raw, 0);
+            fcnt = rvalid(cb);
+            if (fcnt > 0) {
+              ring_issue(cb, rh ^ 1);
+              if (lane == 0) cb_raw = (uint32_t)atomicAdd(P.counter, (unsigned long long)kRingB);
+            }
+          }
+          const int take = min(rcnt - rpos, __popc(need));
+          const int rank = __popc(need & lt_mask);
+          const bool mine = ((need >> lane) & 1u) && rank < take;
+          if (mine) {
+            const int r = rpos + rank;
+            const unsigned char* hb = ring + rh * kRingHalfBytes;
+            const double* f = reinterpret_cast<const double*>(hb) + r;
+            const uint32_t* u = reinterpret_cast<const uint32_t*>(hb + kParkF64 * kRingB * 8) + r;
+            x = f[0]; y = f[kRingB]; ox = f[2 * kRingB]; oy = f[3 * kRingB];
+            exn = f[4 * kRingB]; eyn = f[5 * kRingB]; e = f[6 * kRingB]; w = f[7 * kRingB];
+            mfp = f[8 * kRingB]; dcen = f[9 * kRingB]; acc = f[10 * kRingB];
+            dstep = f[11 * kRingB]; m.st = f[12 * kRingB]; m.pa = f[13 * kRingB];
+            m.H = f[14 * kRingB];
+            cx = (int32_t)u[0]; cy = (int32_t)u[kRingB]; ctr = u[2 * kRingB];
+            nf = u[3 * kRingB]; nc = u[4 * kRingB]; i = (int32_t)u[5 * kRingB];
+            iox = 1.0 / ox;
+            ioy = 1.0 / oy;
+            if (ox == 0.0) iox = d_inf();
+            if (oy == 0.0) ioy = d_inf();
+            active = true;
+            res = true;
+            cidx = cidx_of(cx, cy);
+            draw = dload(cx, cy, cidx);
+          }
+          rpos += take;
+          need &= ~__ballot_sync(kFull, mine);
+        }
+        rstate = (uint32_t)rh | ((uint32_t)rpos << 1) | ((uint32_t)rcnt << 8) | ((uint32_t)fcnt << 16);
+      }
+    } else if (!consumer && !exhausted && idle != 0u && (__popc(idle) >= P.refill_min || idle == kFull)) {
       const int leader = __ffs(idle) - 1;
       unsigned long long base = 0;
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
@@ -758,7 +891,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
 #define NT_HIST_MINB 6   // resident CTAs per SM the default kernel is compiled for (A/B ab11)
 #endif
 template <bool kDet, bool kTiled, bool kVar>
-static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos, bool fused) {
+static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos, bool fused,
+                        bool q = false) {
   if (fmt == kDensU8) {
     if (!blk) return (void*)history_kernel<kDet, kDensU8, kTiled, false, 6, 0, false, kVar, false>;
     if constexpr (!kVar) {
@@ -769,6 +903,8 @@ static void* history_fn(int fmt, bool blk, int minb, int tally, int xs, bool aos
         if (tally == 1) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 1, false, false, false>;
         if (tally == 2) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 2, false, false, false>;
         if (tally == 3) return (void*)history_kernel<kDet, kDensU8, kTiled, true, 6, 3, false, false, false>;
+        // resume ring (resume_prefetch): the default kernel with record parking
+        if (q) return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, 0, false, false, false, false, false, true>;
         // fused phases: the default kernel otherwise (nt_api.cu history_fused mirrors this)
         if (fused) return (void*)history_kernel<kDet, kDensU8, kTiled, true, NT_HIST_MINB, 0, false, false, false, false, true>;
       }
@@ -791,27 +927,40 @@ static void* history_slab_fn(int fmt, bool blk) {
 
 template <bool kVar>
 static void* history_select_v(bool det, int fmt, bool tiled, bool blk, int minb, int tally, int xs,
-                              bool aos, bool fused) {
+                              bool aos, bool fused, bool q) {
   if (det) return tiled ? history_fn<true, true, kVar>(fmt, blk, minb, tally, xs, aos, false)
                         : history_fn<true, false, kVar>(fmt, blk, minb, tally, xs, aos, false);
-  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, tally, xs, aos, fused)
-               : history_fn<false, false, kVar>(fmt, blk, minb, tally, xs, aos, fused);
+  return tiled ? history_fn<false, true, kVar>(fmt, blk, minb, tally, xs, aos, fused, q)
+               : history_fn<false, false, kVar>(fmt, blk, minb, tally, xs, aos, fused, q);
 }
 
 static void* history_select(bool det, int fmt, bool tiled, bool blk, int minb, int tally, int xs,
-                            bool var, bool slab = false, bool aos = false, bool fused = false) {
+                            bool var, bool slab = false, bool aos = false, bool fused = false,
+                            bool q = false) {
   if (slab) return tiled ? history_slab_fn<true>(fmt, blk) : history_slab_fn<false>(fmt, blk);
-  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, tally, xs, false, false)
-             : history_select_v<false>(det, fmt, tiled, blk, minb, tally, xs, aos, fused);
+  return var ? history_select_v<true>(det, fmt, tiled, blk, minb, tally, xs, false, false, false)
+             : history_select_v<false>(det, fmt, tiled, blk, minb, tally, xs, aos, fused, q);
 }
 
 void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tally_mode,
                     int xs_search, bool slab, cudaStream_t s) {
   const bool var = tp.ph.vacuum || tp.ph.analog || tp.ph.roulette;
+  const bool q = tp.park_rec != nullptr;     // resume_prefetch (the host checked the conditions)
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode, xs_search, var, slab, tp.aos != nullptr, tp.coll_ctas > 0);
+                            tally_mode, xs_search, var, slab, tp.aos != nullptr, tp.coll_ctas > 0, q);
   void* args[] = {const_cast<TrackParams*>(&tp)};
-  cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, 0, s);
+  // the resume phase of a kQ kernel holds the record ring in dynamic shared memory (phase 1
+  // launches without it, keeping the larger L1 for the density and edge gathers)
+  const size_t dyn = (q && tp.resume_q != nullptr) ? (size_t)kRingCtaBytes : 0;
+  cudaLaunchKernel(fn, dim3(grid), dim3(kHistoryBlock), args, dyn, s);
+}
+
+int history_ring_ctas_per_sm(bool tiled) {
+  int n = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(
+      &n, history_select(false, kDensU8, tiled, true, 6, 0, 0, false, false, false, false, true),
+      kHistoryBlock, kRingCtaBytes);
+  return n;
 }
 
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally) {
@@ -954,6 +1103,22 @@ __global__ void threefry_debug_kernel(const uint64_t* __restrict__ in, int64_t n
 void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStream_t s) {
   if (n <= 0) return;
   threefry_debug_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(in, n, out);
+}
+
+__global__ void xs_rows_kernel(const double2* __restrict__ kv, const uint32_t* __restrict__ idx,
+                               int64_t nb, double2* __restrict__ row) {
+  const int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (b >= nb) return;
+  const double2* src = kv + idx[b];
+  row[3 * b] = src[0];
+  row[3 * b + 1] = src[1];
+  row[3 * b + 2] = src[2];
+}
+
+void launch_xs_rows(const double2* kv, const uint32_t* idx, int64_t nb, double2* row,
+                    cudaStream_t s) {
+  if (nb <= 0) return;
+  xs_rows_kernel<<<(unsigned)((nb + 255) / 256), 256, 0, s>>>(kv, idx, nb, row);
 }
 
 __global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, int64_t n,

@@ -160,6 +160,25 @@ def test_parity_fused_phases(nt, orc, cfgname, fused):
         assert np.all(gp["status"] <= 1)
 
 
+@pytest.mark.parametrize("resume_prefetch", [0, 1])
+@pytest.mark.parametrize("cfgname", ["tiny_csp", "small_csp", "small_scatter", "tiny_split", "tiny_mosaic",
+                                     "tiny_mid", "tiny_hotspot"])
+def test_parity_resume_prefetch(nt, orc, cfgname, resume_prefetch):
+    """Production history mode with parked particles as queue-ordered records streamed by a
+    cp.async ring (1) or the particle store + index queue (0): same per-particle results,
+    tally within the production bar, every parked particle resumed once (batches of 12
+    records, ragged last batch; defer_below 33 parks every collision)."""
+    cfg = wl.CONFIGS[cfgname]
+    for defer_below in (8, 33):
+        gt, gp, (gs,) = _gpu_run(nt, cfg, deterministic=False, resume_prefetch=resume_prefetch,
+                                 defer_below=defer_below)
+        ot, op, (os_,) = orc.run(cfg)
+        compare_particles(gp, op)
+        compare_tally(gt, ot, rtol=1e-6, floor=1e-12)
+        compare_stats(gs, os_, rtol=1e-9)
+        assert np.all(gp["status"] <= 1)
+
+
 @pytest.mark.parametrize("cfgname", ["tiny_csp", "small_csp", "small_scatter", "tiny_split", "tiny_mosaic"])
 def test_parity_aos_particle_layout(nt, orc, cfgname):
     """particle_layout 1 (AoS records while the history kernel runs): same
