@@ -158,8 +158,10 @@ typedef struct {
                                   144 B record, and the second launch streams the records
                                   into a per-warp shared-memory ring with cp.async one
                                   batch ahead of use (refills of resumed particles read
-                                  shared memory); 0 the state goes to the particle store
-                                  and a queue of indices.  Results are unchanged.         */
+                                  shared memory); 0 (default) the state goes to the
+                                  particle store and a queue of indices.  Results are
+                                  unchanged.  (Measured: 1 is 2% slower on csp and split,
+                                  DESIGN.md §8.)                                          */
 } nt_options;
 
 /* Statistics of one timestep (sums over the particles this rank -- or, when nranks > 1,

@@ -288,7 +288,6 @@ nt_status nt_options_default(nt_options* opt) {
   opt->det_batch = 65536;
   opt->refill_min = 4;
   opt->defer_below = 8;
-  opt->resume_prefetch = 1;
   return NT_OK;
 }
 

@@ -97,6 +97,9 @@ void launch_inject(const InjectParams& ip, cudaStream_t s) {
 // phase streams those records into a per-warp shared-memory ring with cp.async, one batch
 // ahead of use, so a refill of parked particles costs shared-memory loads instead of a
 // dependent chain of global loads (queue index, then the state, then the XS lookups).
+// Measured and rejected as the default (csp 27.0 -> 27.5 ms, split 104.7 -> 107.0 ms,
+// profiles/ab/r02_ab20_resume_ring.txt): the resumed phase is not refill-bound -- its time
+// goes to the streaming tail of particles scattered back out of dense matter.
 template <bool kDet, int kFmt, bool kTiled, bool kBlk, int kMinB, int kTally, bool kXsWalk,
           bool kVar, bool kSlab, bool kAoS = false, bool kFused = false, bool kQ = false>
 __global__ void __launch_bounds__(kHistoryBlock, kMinB)
@@ -812,6 +815,8 @@ history_kernel(const __grid_constant__ TrackParams P) {
     // Each lane runs up to kInnerEvents events between two warp votes; the per-lane bound
     // lim = min(events so far + kInnerEvents, max_events) also enforces the event cap (R27),
     // whose kill is handled by event(true) once the bound is the cap.
+    // (with the resume ring's cheap refills, 4-64 events per vote in the resumed phase were
+    // measured too: all slower, csp +0.9-2.6%, split +1-9%; profiles/ab/r02_ab20_resume_ring.txt)
     constexpr uint32_t inner = (uint32_t)kInnerEvents;
     auto run_lane = [&]() __attribute__((always_inline)) {
       if (active) {

@@ -49,7 +49,7 @@ def test_identity_calls(L):
     assert L.nt_options_default(C.byref(o)) == 0
     assert o.nranks == 1 and o.A == 1.0 and o.e_min == 1.0 and o.w_min == 1e-3
     assert o.max_events_per_history == 10**9 and o.det_batch == 65536 and o.refill_min == 4
-    assert o.defer_below == 8 and o.resume_prefetch == 1 and o.xs_search == 0
+    assert o.defer_below == 8 and o.resume_prefetch == 0 and o.xs_search == 0
 
 
 def test_struct_layouts_match_header():
