@@ -23,6 +23,18 @@ namespace nt {
 
 __device__ __forceinline__ double d_inf() { return __longlong_as_double(0x7ff0000000000000ll); }
 
+#ifndef NT_TIMELINE
+#define NT_TIMELINE 0    // dev variant: per-warp start / range-exhausted / end globaltimer stamps
+#endif
+#if NT_TIMELINE
+__device__ unsigned long long g_tl[2][8192][3];
+__device__ __forceinline__ unsigned long long gtimer() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+  return t;
+}
+#endif
+
 // ---------------------------------------------------------------------------------------
 // Mesh edges: edge(i) = (i*W)/n  (DESIGN.md §3 MESH)
 __global__ void edges_kernel(double* ex, int32_t nx, double W, double* ey, int32_t ny,
@@ -207,6 +219,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
 
   bool active = false, exhausted = false;
   int32_t i = 0;                 // local particle index (< 2^31)
+#if NT_TIMELINE
+  const int tl_w = (int)((blockIdx.x * kHistoryBlock + threadIdx.x) >> 5);
+  const int tl_p = P.phase == 2 ? 1 : 0;
+  if ((threadIdx.x & 31) == 0 && tl_w < 8192) { g_tl[tl_p][tl_w][0] = gtimer(); g_tl[tl_p][tl_w][1] = 0; }
+#endif
   // register-resident history state
   double x = 0, y = 0, ox = 0, oy = 0, iox = 0, ioy = 0, e = 0, w = 0, mfp = 0, dcen = 0;
   typename DensRaw<kFmt>::type draw = 0;  // density (code) of the current cell, as loaded
@@ -486,6 +503,9 @@ history_kernel(const __grid_constant__ TrackParams P) {
       if (lane == leader) base = atomicAdd(P.counter, (unsigned long long)__popc(idle));
       base = __shfl_sync(kFull, base, leader);
       if (base + (unsigned long long)__popc(idle) >= span2) {
+#if NT_TIMELINE
+        if (!exhausted && lane == 0 && tl_w < 8192) g_tl[tl_p][tl_w][1] = gtimer();
+#endif
         exhausted = true;
       }
       if (!active) {
@@ -554,7 +574,12 @@ history_kernel(const __grid_constant__ TrackParams P) {
         consumer = true;
         continue;
       }
-      if (exhausted) break;
+      if (exhausted) {
+#if NT_TIMELINE
+        if (lane == 0 && tl_w < 8192) g_tl[tl_p][tl_w][2] = gtimer();
+#endif
+        break;
+      }
       continue;
     }
 
@@ -952,7 +977,7 @@ void launch_history(const TrackParams& tp, bool det, int grid, int minb, int tal
   const bool var = tp.ph.vacuum || tp.ph.analog || tp.ph.roulette;
   const bool q = tp.park_rec != nullptr;     // resume_prefetch (the host checked the conditions)
   void* fn = history_select(det, tp.mesh.fmt, tp.mesh.tiled != 0, tp.mesh.blk != nullptr, minb,
-                            tally_mode, xs_search, var, slab, tp.aos != nullptr, tp.coll_ctas > 0, q);
+                            tally_mode, xs_search, var, slab, tp.aos != nullptr, tp.park_taken != nullptr, q);
   void* args[] = {const_cast<TrackParams*>(&tp)};
   // the resume phase of a kQ kernel holds the record ring in dynamic shared memory (phase 1
   // launches without it, keeping the larger L1 for the density and edge gathers)
@@ -1119,6 +1144,12 @@ __global__ void xs_rows_kernel(const double2* __restrict__ kv, const uint32_t* _
   row[3 * b + 1] = src[1];
   row[3 * b + 2] = src[2];
 }
+
+#if NT_TIMELINE
+extern "C" int nt_dev_timeline(unsigned long long* out) {   // [2][8192][3]
+  return (int)cudaMemcpyFromSymbol(out, g_tl, sizeof(g_tl));
+}
+#endif
 
 void launch_xs_rows(const double2* kv, const uint32_t* idx, int64_t nb, double2* row,
                     cudaStream_t s) {
