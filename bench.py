@@ -201,7 +201,8 @@ def parse():
     ap.add_argument("--table-size", type=int, default=0,
                     help="experiment: scatter table keys (capture = 3/4 of it); 0 = the config's")
     ap.add_argument("--fused-consumers", type=int, default=0,
-                    help="history mode: fuse the parking phases, k consumer CTAs per SM (0: two launches)")
+                    help="history mode: fuse the parking phases (k > 0: k-1 dedicated consumer CTAs per SM, "
+                         "the other warps resume parked particles once the range is exhausted; 0: two launches)")
     ap.add_argument("--particle-layout", type=int, default=0,
                     help="0 structure of arrays (default), 1 AoS records while tracking (ablation)")
     ap.add_argument("--json-out", default=None)
@@ -455,7 +456,7 @@ def main():
             "config": {"workload": cfg.name, "mode": a.mode, "nx": cfg.nx, "ny": cfg.ny,
                        "layout": "tiled4x4" if a.layout == 0 else "row-major",
                        "particle_store": ["SoA", "AoS (ablation)"][a.particle_layout],
-                       "phases": (f"fused, {a.fused_consumers} consumer CTA(s)/SM" if a.fused_consumers
+                       "phases": (f"fused, {a.fused_consumers - 1} dedicated consumer CTA(s)/SM" if a.fused_consumers
                                   else "two launches (park, resume)"),
                        "density_format": ["codes+block map", "f64", "codes"][a.density_format],
                        "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED", "CAS-emulated fp64 add",

@@ -142,10 +142,12 @@ typedef struct {
                                   production tally, default kernel; others use 0)          */
     int32_t fused_consumers;   /* history mode, production: 0 runs the parked collisions in
                                   a second launch after phase 1 (the default); k > 0 fuses
-                                  both phases into one launch in which k CTAs per SM resume
-                                  parked particles while the others still run phase 1
-                                  (they join when their range is exhausted).  Results are
-                                  unchanged.  u8 block-map meshes, default kernel options */
+                                  both phases into one launch: k - 1 CTAs per SM resume
+                                  parked particles from the start, and every other warp
+                                  turns to them as soon as the particle range is exhausted
+                                  (its idle lanes resume parked particles while its last
+                                  own histories still run).  Results are unchanged.  u8
+                                  block-map meshes, default kernel options                */
     int32_t xs_l2_persist;     /* 1: while the tracking kernels run, an L2 access-policy
                                   window on the context stream marks the cross-section
                                   tables persisting (large lookup tables can

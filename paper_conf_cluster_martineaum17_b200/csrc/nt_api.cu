@@ -579,7 +579,6 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     }
   }
   // bucket indexes over the IEEE bit patterns of the (positive) keys
-  std::vector<uint32_t> idx[2];
   uint64_t base[2] = {0, 0};
   int32_t shift[2] = {0, 0}, nbk[2] = {0, 0};
   for (int t = 0; t < 2; ++t) {
@@ -598,43 +597,14 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     int s = 0;
     while ((range >> s) >= (uint64_t)target) ++s;
     const int64_t nb = (int64_t)(range >> s) + 1;
-    idx[t].resize((size_t)nb + 1);
-    // bin of each bucket's first value, max{i in [0, n-2] : k[i] <= v}: the values increase
-    // with b, so one merge-like sweep over the keys (O(nb + n)) instead of a search each
-    int64_t lo = 0;
-    for (int64_t b = 0; b <= nb; ++b) {
-      const uint64_t bits = b0 + ((uint64_t)b << s);
-      double v;
-      if (bits >= 0x7ff0000000000000ull) v = INFINITY; else std::memcpy(&v, &bits, 8);
-      while (lo < n - 2 && k[lo + 1] <= v) ++lo;
-      idx[t][(size_t)b] = (uint32_t)lo;
-    }
     base[t] = b0;
     shift[t] = s;
     nbk[t] = (int32_t)nb;
   }
-  // interleaved (key, value) pairs, one padding pair (a copy of the last) at the end
-  std::vector<double> kvh[2];
-  for (int t = 0; t < 2; ++t) {
-    const int64_t n = len[2 * t];
-    kvh[t].resize(2 * ((size_t)n + 1));
-    for (int64_t j = 0; j <= n; ++j) {
-      const int64_t q = j < n ? j : n - 1;
-      kvh[t][2 * (size_t)j] = h[2 * t][q];
-      kvh[t][2 * (size_t)j + 1] = h[2 * t + 1][q];
-    }
-  }
-  // direct bucket rows (xs_search 0): bucket b -> the pairs idx[b], idx[b] + 1, idx[b] + 2,
-  // built only when every bucket spans at most one key (then the bin is idx[b] or idx[b] + 1)
-  // (checked here, copied on the device from the interleaved pairs: no extra H2D bytes)
-  int64_t nrows[2] = {0, 0};
-  for (int t = 0; t < 2; ++t) {
-    const int64_t nb = nbk[t];
-    if (nb <= 0) continue;
-    bool ok = true;
-    for (int64_t b = 0; b < nb && ok; ++b) ok = idx[t][(size_t)b + 1] - idx[t][(size_t)b] <= 1u;
-    if (ok) nrows[t] = nb;
-  }
+  // Device buffer: keys, values (as given), the bucket index [nb + 1], the interleaved
+  // (key, value) pairs [n + 1] and the direct bucket rows [nb] (xs_search 0).  Only the
+  // caller's four arrays cross PCIe; the index, pairs and rows are built on the device
+  // (xs_prepare: the index by a binary search per bucket, the same bins as a sweep).
   size_t off[10], total = 0;
   for (int k = 0; k < 4; ++k) {
     off[k] = total;
@@ -642,32 +612,36 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   }
   for (int t = 0; t < 2; ++t) {
     off[4 + t] = total;
-    total += align256(idx[t].size() * 4 + 4);
+    total += align256(((size_t)nbk[t] + 1) * 4 + 4);
   }
   for (int t = 0; t < 2; ++t) {
     off[6 + t] = total;
-    total += align256(kvh[t].size() * 8);
+    total += align256(((size_t)len[2 * t] + 1) * 16);
   }
   for (int t = 0; t < 2; ++t) {
     off[8 + t] = total;
-    total += align256((size_t)nrows[t] * 48);
+    total += align256((size_t)nbk[t] * 48);
   }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k], (size_t)len[k] * 8,
                                cudaMemcpyDefault, c->stream));
-  for (int t = 0; t < 2; ++t) {
-    if (!idx[t].empty())
-      NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[4 + t], idx[t].data(), idx[t].size() * 4,
-                                 cudaMemcpyHostToDevice, c->stream));
-    NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[6 + t], kvh[t].data(), kvh[t].size() * 8,
-                               cudaMemcpyHostToDevice, c->stream));
-    if (nrows[t] > 0)
-      launch_xs_rows(reinterpret_cast<const double2*>(c->xs.as<char>() + off[6 + t]),
-                     reinterpret_cast<const uint32_t*>(c->xs.as<char>() + off[4 + t]), nrows[t],
-                     reinterpret_cast<double2*>(c->xs.as<char>() + off[8 + t]), c->stream);
-  }
+  unsigned int* wide = reinterpret_cast<unsigned int*>(c->scratch.as<char>() + 128);  // [2]
+  NT_CUDA(c, cudaMemsetAsync(wide, 0, 8, c->stream));
+  for (int t = 0; t < 2; ++t)
+    launch_xs_prepare(reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t]),
+                      reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t + 1]),
+                      len[2 * t], base[t], shift[t], nbk[t],
+                      reinterpret_cast<uint32_t*>(c->xs.as<char>() + off[4 + t]),
+                      reinterpret_cast<double2*>(c->xs.as<char>() + off[6 + t]),
+                      reinterpret_cast<double2*>(c->xs.as<char>() + off[8 + t]), wide + t, c->stream);
+  unsigned int hw[2] = {1, 1};
+  NT_CUDA(c, cudaMemcpyAsync(hw, wide, 8, cudaMemcpyDeviceToHost, c->stream));
+  // direct bucket rows only where every bucket spans at most one key (then the bin is
+  // idx[b] or idx[b] + 1)
+  int64_t nrows[2] = {0, 0};
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
+  for (int t = 0; t < 2; ++t) nrows[t] = (nbk[t] > 0 && hw[t] == 0) ? nbk[t] : 0;
   c->xs_bytes = total;
   c->xs_persist_bytes = 0;
   if (c->opt.xs_l2_persist) {
@@ -916,7 +890,7 @@ static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uin
     p.park_q = c->defer_q;
     p.park_count = qlen;
     p.park_coll_below = c->opt.defer_below;
-    int coll = c->opt.fused_consumers * c->sm_count;
+    int coll = (c->opt.fused_consumers - 1) * c->sm_count;   // dedicated consumer CTAs
     if (coll >= grid) coll = grid - 1;
     p.coll_ctas = coll;
     p.n_prod = (uint32_t)(grid - coll) * (uint32_t)(kHistoryBlock / 32);

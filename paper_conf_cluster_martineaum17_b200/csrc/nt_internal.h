@@ -92,9 +92,12 @@ void launch_slab_pack(const TrackParams& tp, const int32_t* out_q, int64_t n, Sl
 void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32_t* free_slots,
                         int64_t n_free, int64_t base, int32_t* arr_q, cudaStream_t s);
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally);
-// direct bucket rows (xs_search 0): row[3b .. 3b+2] = kv[idx[b] .. idx[b]+2], b < nb
-void launch_xs_rows(const double2* kv, const uint32_t* idx, int64_t nb, double2* row,
-                    cudaStream_t s);
+// cross-section tables on the device: the interleaved pairs kv [n + 1], the bucket index
+// idx [nb + 1] (base, shift: the bucket of a bit pattern is (bits - base) >> shift) and the
+// direct bucket rows [nb] (xs_search 0); *wide |= 1 if a bucket spans more than one key
+void launch_xs_prepare(const double* k, const double* v, int64_t n, uint64_t base, int shift,
+                       int64_t nb, uint32_t* idx, double2* kv, double2* row, unsigned int* wide,
+                       cudaStream_t s);
 // resident CTAs per SM of the resume_prefetch kernel with its ring (phase 2)
 int history_ring_ctas_per_sm(bool tiled);
 void launch_det_apply(const unsigned long long* keys, const double* vals,

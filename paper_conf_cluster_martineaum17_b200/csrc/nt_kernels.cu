@@ -259,6 +259,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
   // a consumer lane holds at most one claimed queue position (pend, qpos) and is done (fin)
   // once every producer has finished and its claim lies beyond the final queue length.
   bool consumer = kFused && (int)blockIdx.x < P.coll_ctas;
+  // a producer warp turns consumer as soon as its particle range is exhausted, while its
+  // own (producer) lanes still run: their idle lanes resume parked particles instead of
+  // waiting for the warp's last history (the phase-1 tail).  prod_live: producer lanes may
+  // still park -- the warp counts itself done (prod_done) once none is left.
+  bool prod_live = kFused && !consumer;
   bool res = resume, pend = false, fin = false;
   uint32_t qpos = 0;
   // Park this lane: the state before its next event to the particle store (status st), the
@@ -387,6 +392,11 @@ history_kernel(const __grid_constant__ TrackParams P) {
 
   for (;;) {
     if constexpr (kFused) {
+      if (prod_live && consumer && !__any_sync(kFull, active && !res)) {
+        __threadfence();                     // this warp's parks are published
+        if (lane == 0) atomicAdd(P.prod_done, 1u);
+        prod_live = false;
+      }
       if (consumer) {
         // ---- consumer refill: claim queue positions for idle lanes, take published ones ----
         const unsigned want = __ballot_sync(kFull, !active && !pend && !fin);
@@ -507,6 +517,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
         if (!exhausted && lane == 0 && tl_w < 8192) g_tl[tl_p][tl_w][1] = gtimer();
 #endif
         exhausted = true;
+        if constexpr (kFused) consumer = true;   // mixed from here on (prod_live until done)
       }
       if (!active) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
@@ -567,13 +578,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       }
     }
     if (!__any_sync(kFull, active)) {
-      if (kFused && !consumer && exhausted) {
-        // this producer warp is done: count it, then resume parked particles too
-        __threadfence();
-        if (lane == 0) atomicAdd(P.prod_done, 1u);
-        consumer = true;
-        continue;
-      }
+      if (kFused && consumer) continue;    // the consumer block at the loop top decides
       if (exhausted) {
 #if NT_TIMELINE
         if (lane == 0 && tl_w < 8192) g_tl[tl_p][tl_w][2] = gtimer();
@@ -664,7 +669,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           fsum(SF_KILLED_E, w * e);
           fsum(SF_KILLED_W, w);
           outcome = 2;
-        } else if (coll && !(kFused && consumer) && __popc(__activemask()) < park_coll_below) {
+        } else if (coll && !(kFused && res) && __popc(__activemask()) < park_coll_below) {
           park_to(2u, P.park_q, P.park_count);
         } else if (coll) {
           // ---- collision (implicit capture + elastic scatter) ----
@@ -1135,26 +1140,60 @@ void launch_threefry_debug(const uint64_t* in, int64_t n, uint64_t* out, cudaStr
   threefry_debug_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(in, n, out);
 }
 
-__global__ void xs_rows_kernel(const double2* __restrict__ kv, const uint32_t* __restrict__ idx,
-                               int64_t nb, double2* __restrict__ row) {
-  const int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
-  if (b >= nb) return;
-  const double2* src = kv + idx[b];
-  row[3 * b] = src[0];
-  row[3 * b + 1] = src[1];
-  row[3 * b + 2] = src[2];
-}
-
 #if NT_TIMELINE
 extern "C" int nt_dev_timeline(unsigned long long* out) {   // [2][8192][3]
   return (int)cudaMemcpyFromSymbol(out, g_tl, sizeof(g_tl));
 }
 #endif
 
-void launch_xs_rows(const double2* kv, const uint32_t* idx, int64_t nb, double2* row,
-                    cudaStream_t s) {
+// ---- cross-section table preparation (nt_load_cross_sections) ----
+// interleaved (key, value) pairs [n + 1], the last pair repeated as padding
+__global__ void xs_pairs_kernel(const double* __restrict__ k, const double* __restrict__ v,
+                                int64_t n, double2* __restrict__ kv) {
+  const int64_t j = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (j > n) return;
+  const int64_t q = j < n ? j : n - 1;
+  kv[j] = make_double2(k[q], v[q]);
+}
+
+// bucket index: idx[b] = max{i in [0, n-2] : k[i] <= value with bits base + (b << shift)}
+// (+inf past the finite range), b in [0, nb]
+__global__ void xs_index_kernel(const double* __restrict__ k, int64_t n, uint64_t base, int shift,
+                                int64_t nb, uint32_t* __restrict__ idx) {
+  const int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (b > nb) return;
+  const uint64_t bits = base + ((uint64_t)b << shift);
+  const double v = bits >= 0x7ff0000000000000ull ? __longlong_as_double(0x7ff0000000000000ll)
+                                                 : __longlong_as_double((long long)bits);
+  int64_t lo = 0, hi = n - 1;                 // k[lo] <= v (k[0] is bucket 0's first value)
+  while (hi - lo > 1) {
+    const int64_t mid = (lo + hi) >> 1;
+    if (k[mid] <= v) lo = mid; else hi = mid;
+  }
+  idx[b] = (uint32_t)lo;
+}
+
+// direct bucket rows: row[3b .. 3b+2] = kv[idx[b] .. idx[b]+2]; *wide != 0 if some bucket
+// spans more than one key (then the rows are not used)
+__global__ void xs_rows_kernel(const double2* __restrict__ kv, const uint32_t* __restrict__ idx,
+                               int64_t nb, double2* __restrict__ row, unsigned int* wide) {
+  const int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (b >= nb) return;
+  const uint32_t i0 = idx[b];
+  if (idx[b + 1] - i0 > 1u) atomicOr(wide, 1u);
+  const double2* src = kv + i0;
+  row[3 * b] = src[0];
+  row[3 * b + 1] = src[1];
+  row[3 * b + 2] = src[2];
+}
+
+void launch_xs_prepare(const double* k, const double* v, int64_t n, uint64_t base, int shift,
+                       int64_t nb, uint32_t* idx, double2* kv, double2* row, unsigned int* wide,
+                       cudaStream_t s) {
+  xs_pairs_kernel<<<(unsigned)((n + 256) / 256), 256, 0, s>>>(k, v, n, kv);
   if (nb <= 0) return;
-  xs_rows_kernel<<<(unsigned)((nb + 255) / 256), 256, 0, s>>>(kv, idx, nb, row);
+  xs_index_kernel<<<(unsigned)((nb + 256) / 256), 256, 0, s>>>(k, n, base, shift, nb, idx);
+  xs_rows_kernel<<<(unsigned)((nb + 255) / 256), 256, 0, s>>>(kv, idx, nb, row, wide);
 }
 
 __global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, int64_t n,
