@@ -303,6 +303,10 @@ int64_t nt_debug_mesh_bytes(const nt_ctx *ctx);
 /* Which loaded tables have direct bucket rows (xs_search 0): bit 0 scatter, bit 1 capture;
  * -1 for a NULL context. */
 int32_t nt_debug_xs_rows(const nt_ctx *ctx);
+/* The density storage nt_init_mesh chose: 2 u8 material codes, 1 u16 codes, 0 the f64 map
+ * (-1 for a NULL context, or before nt_init_mesh); *n_distinct (if not NULL) = the number
+ * of distinct density values found (0 for the f64 format without codes). */
+int32_t nt_debug_density_format(const nt_ctx *ctx, int32_t *n_distinct);
 /* out[2i], out[2i+1] = threefry2x64_20(ctr = {in[4i], in[4i+1]}, key = {in[4i+2], in[4i+3]}). */
 nt_status nt_debug_threefry(nt_ctx *ctx, const uint64_t *in, int64_t n, uint64_t *out);
 /* Microscopic XS from the loaded tables: out_s[i], out_a[i] at energies[i] (no clamp

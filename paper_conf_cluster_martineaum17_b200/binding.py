@@ -32,7 +32,7 @@ EXPORTS = ["nt_abi_version", "nt_build_info", "nt_status_string", "nt_options_de
            "nt_read_particles", "nt_write_particles", "nt_slab_record_bytes", "nt_slab_begin",
            "nt_slab_round", "nt_slab_export", "nt_slab_import", "nt_slab_end", "nt_particle_slots",
            "nt_debug_threefry", "nt_debug_xs", "nt_debug_alloc_count",
-           "nt_debug_mesh_bytes", "nt_debug_xs_rows"]
+           "nt_debug_mesh_bytes", "nt_debug_xs_rows", "nt_debug_density_format"]
 
 
 class NeutralError(RuntimeError):
@@ -124,6 +124,7 @@ def lib():
             "nt_debug_alloc_count": ([], i64),
             "nt_debug_mesh_bytes": ([vp], i64),
             "nt_debug_xs_rows": ([vp], C.c_int32),
+            "nt_debug_density_format": ([vp, vp], C.c_int32),
         }
         for name, (args, res) in sigs.items():
             f = getattr(L, name)
@@ -356,6 +357,12 @@ class Tracker:
     def mesh_bytes(self) -> int:
         """Device bytes held for the mesh (density + tally buffers)."""
         return int(lib().nt_debug_mesh_bytes(self._h))
+
+    def density_format(self) -> tuple[str, int]:
+        """(storage nt_init_mesh chose: "u8" / "u16" / "f64", distinct density values found)."""
+        n = C.c_int32(0)
+        f = int(lib().nt_debug_density_format(self._h, C.byref(n)))
+        return {2: "u8", 1: "u16", 0: "f64"}.get(f, str(f)), int(n.value)
 
     def xs_rows(self) -> int:
         """Bit mask of the loaded tables with direct bucket rows (1 scatter, 2 capture)."""

@@ -77,6 +77,10 @@ struct nt_ctx {
   cudaStream_t stream = nullptr;
   bool own_stream = false;
   cudaEvent_t ev[6] = {};
+  cudaStream_t aux = nullptr;            // nt_init_mesh: checks chunks while the next uploads
+  cudaEvent_t chunk_ev[9] = {};
+  DevBuf dset;                           // distinct-value set (kDistinctSlots u64)
+  int32_t dens_distinct = 0;             // distinct density values found by nt_init_mesh
   ncclComm_t comm = nullptr;
   Phys ph{};
   // step statistics as doubles: [SU_COUNT u64 counts][SF_COUNT sums] (device, and a
@@ -365,6 +369,11 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
     c->own_stream = true;
   }
   for (auto& ev : c->ev) cudaEventCreate(&ev);
+  for (auto& ev : c->chunk_ev) cudaEventCreateWithFlags(&ev, cudaEventDisableTiming);
+  if (cudaStreamCreateWithFlags(&c->aux, cudaStreamNonBlocking) != cudaSuccess) {
+    nt_destroy(c);
+    return NT_ERR_CUDA;
+  }
   if (cudaHostAlloc(reinterpret_cast<void**>(&c->stats_h), (SU_COUNT + SF_COUNT) * sizeof(double),
                     cudaHostAllocDefault) != cudaSuccess ||
       c->stats_d.ensure((SU_COUNT + SF_COUNT) * sizeof(double)) != cudaSuccess) {
@@ -396,11 +405,14 @@ nt_status nt_destroy(nt_ctx* c) {
   }
   for (DevBuf* b : {&c->slab_buf, &c->slab_rbuf, &c->rho_code, &c->blk, &c->nd_tab, &c->enc_keys, &c->rho_st, &c->tally_rm, &c->tally_full, &c->rho, &c->tally, &c->tally_red, &c->ex, &c->ey, &c->xs, &c->soa,
                     &c->scratch, &c->slots, &c->rec_key, &c->rec_val, &c->rec_key2, &c->rec_val2,
-                    &c->sort_tmp, &c->backup, &c->stats_d, &c->aos, &c->park_rec})
+                    &c->sort_tmp, &c->backup, &c->stats_d, &c->aos, &c->park_rec, &c->dset})
     b->release();
   if (c->stats_h) cudaFreeHost(c->stats_h);
   for (auto& ev : c->ev)
     if (ev) cudaEventDestroy(ev);
+  for (auto& ev : c->chunk_ev)
+    if (ev) cudaEventDestroy(ev);
+  if (c->aux) cudaStreamDestroy(c->aux);
   if (c->comm) ncclCommDestroy(c->comm);
   if (c->own_stream && c->stream) cudaStreamDestroy(c->stream);
   delete c;
@@ -454,33 +466,62 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   NT_CUDA(c, c->ex.ensure(((size_t)nx + 1) * 8));
   NT_CUDA(c, c->ey.ensure(((size_t)ny + 1) * 8));
   NT_CUDA(c, c->scratch.ensure(1024));
-  if (nxs == nx)
-    NT_CUDA(c, cudaMemcpyAsync(c->rho.p, density, (size_t)cells * 8, cudaMemcpyDefault, c->stream));
-  else
+  // Upload in chunks on the context stream; each chunk is validated and its distinct values
+  // collected (check_distinct_kernel) on the aux stream while the next chunk is copied, so
+  // the device work hides under the H2D transfer.
+  const bool codes = c->opt.density_format == 0 || c->opt.density_format == 2;
+  unsigned long long* bad = reinterpret_cast<unsigned long long*>(c->scratch.as<char>() + 160);  // [3]
+  NT_CUDA(c, c->dset.ensure((size_t)kDistinctSlots * 8));
+  unsigned long long* dset = c->dset.as<unsigned long long>();
+  NT_CUDA(c, cudaMemsetAsync(bad, 0, 24, c->stream));
+  NT_CUDA(c, cudaMemsetAsync(dset, 0xff, (size_t)kDistinctSlots * 8, c->stream));
+  if (nxs == nx) {
+    constexpr int kChunks = 8;
+    const int64_t per = (cells + kChunks - 1) / kChunks;
+    for (int k = 0; k < kChunks; ++k) {
+      const int64_t a = (int64_t)k * per, n = a < cells ? (cells - a < per ? cells - a : per) : 0;
+      if (n <= 0) break;
+      NT_CUDA(c, cudaMemcpyAsync(c->rho.as<double>() + a, density + a, (size_t)n * 8, cudaMemcpyDefault, c->stream));
+      NT_CUDA(c, cudaEventRecord(c->chunk_ev[k], c->stream));
+      NT_CUDA(c, cudaStreamWaitEvent(c->aux, c->chunk_ev[k], 0));
+      if (codes) NT_CUDA(c, launch_check_distinct(c->rho.as<double>() + a, n, bad, dset, c->aux));
+      else NT_CUDA(c, launch_density_check(c->rho.as<double>() + a, n, bad, c->aux));
+    }
+    NT_CUDA(c, cudaEventRecord(c->chunk_ev[8], c->aux));
+    NT_CUDA(c, cudaStreamWaitEvent(c->stream, c->chunk_ev[8], 0));
+  } else {
     NT_CUDA(c, cudaMemcpy2DAsync(c->rho.p, (size_t)nxs * 8, density + x0, (size_t)nx * 8,
                                  (size_t)nxs * 8, (size_t)ny, cudaMemcpyDefault, c->stream));
-  unsigned long long* bad = c->scratch.as<unsigned long long>();
-  NT_CUDA(c, cudaMemsetAsync(bad, 0, 16, c->stream));
-  NT_CUDA(c, launch_density_check(c->rho.as<double>(), cells, bad, c->stream));
-  // distinct density values (for the lossless encoding)
-  int fmt = kDensF64, nu = 0;
-  if (c->opt.density_format == 0 || c->opt.density_format == 2) {
-    size_t tmp = 0;
-    NT_CUDA(c, c->enc_keys.ensure((size_t)cells * 16));
-    unsigned long long* k0 = c->enc_keys.as<unsigned long long>();
-    unsigned long long* k1 = k0 + cells;
-    int* d_count = reinterpret_cast<int*>(c->scratch.as<char>() + 8);
-    NT_CUDA(c, density_distinct(c->rho.as<double>(), cells, k0, k1, nullptr, tmp, d_count, c->stream));
-    NT_CUDA(c, c->sort_tmp.ensure(tmp));
-    NT_CUDA(c, density_distinct(c->rho.as<double>(), cells, k0, k1, c->sort_tmp.p, tmp, d_count, c->stream));
+    if (codes) NT_CUDA(c, launch_check_distinct(c->rho.as<double>(), cells, bad, dset, c->stream));
+    else NT_CUDA(c, launch_density_check(c->rho.as<double>(), cells, bad, c->stream));
   }
-  unsigned long long hb[2] = {0, 0};
-  NT_CUDA(c, cudaMemcpyAsync(hb, bad, 16, cudaMemcpyDeviceToHost, c->stream));
+  unsigned long long hb[3] = {0, 0, 0};
+  NT_CUDA(c, cudaMemcpyAsync(hb, bad, 24, cudaMemcpyDeviceToHost, c->stream));
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   if (hb[0] != 0)
     return fail(c, NT_ERR_ARG, "%llu density values are not finite and >= 0", hb[0]);
-  if (c->opt.density_format == 0 || c->opt.density_format == 2) {
-    nu = (int)(hb[1] & 0xffffffffu);
+  // distinct density values (for the lossless encoding): sorted from the set, or -- more
+  // than kDistinctSlots / 2 of them -- by sorting every cell's bit pattern
+  int fmt = kDensF64, nu = 0;
+  if (codes) {
+    if (hb[2] == 0) {
+      nu = (int)hb[1];
+      NT_CUDA(c, c->enc_keys.ensure((size_t)kDistinctSlots * 8));
+      NT_CUDA(c, launch_distinct_sort(dset, c->enc_keys.as<unsigned long long>(), c->stream));
+    } else {
+      size_t tmp = 0;
+      NT_CUDA(c, c->enc_keys.ensure((size_t)cells * 16));
+      unsigned long long* k0 = c->enc_keys.as<unsigned long long>();
+      unsigned long long* k1 = k0 + cells;
+      int* d_count = reinterpret_cast<int*>(c->scratch.as<char>() + 8);
+      NT_CUDA(c, density_distinct(c->rho.as<double>(), cells, k0, k1, nullptr, tmp, d_count, c->stream));
+      NT_CUDA(c, c->sort_tmp.ensure(tmp));
+      NT_CUDA(c, density_distinct(c->rho.as<double>(), cells, k0, k1, c->sort_tmp.p, tmp, d_count, c->stream));
+      int hn = 0;
+      NT_CUDA(c, cudaMemcpyAsync(&hn, d_count, 4, cudaMemcpyDeviceToHost, c->stream));
+      NT_CUDA(c, cudaStreamSynchronize(c->stream));
+      nu = hn;
+    }
     if (nu <= 256) fmt = kDensU8;
     else if (nu <= 65536) fmt = kDensU16;
   }
@@ -523,6 +564,7 @@ nt_status nt_init_mesh(nt_ctx* c, int32_t nx, int32_t ny, double width, double h
   NT_CUDA(c, cudaGetLastError());
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   c->dens_fmt = fmt;
+  c->dens_distinct = nu;
   c->dens_codes = nu;
   c->blk_shift = blk_shift;
   c->blk_nbx = blk_nbx;
@@ -618,9 +660,14 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     off[6 + t] = total;
     total += align256(((size_t)len[2 * t] + 1) * 16);
   }
+  // rows only while they stay comfortably L2-resident (the scatter sweep: 2^20-key tables
+  // give 100+ MB of rows per table, and the rows then lose to the 4 B bucket index)
+  constexpr int64_t kRowsMaxBytes = 32ll << 20;
+  int64_t nrow_alloc[2] = {0, 0};
   for (int t = 0; t < 2; ++t) {
+    nrow_alloc[t] = (int64_t)nbk[t] * 48 <= kRowsMaxBytes ? nbk[t] : 0;
     off[8 + t] = total;
-    total += align256((size_t)nbk[t] * 48);
+    total += align256((size_t)nrow_alloc[t] * 48);
   }
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
@@ -631,7 +678,7 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   for (int t = 0; t < 2; ++t)
     launch_xs_prepare(reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t]),
                       reinterpret_cast<const double*>(c->xs.as<char>() + off[2 * t + 1]),
-                      len[2 * t], base[t], shift[t], nbk[t],
+                      len[2 * t], base[t], shift[t], nbk[t], nrow_alloc[t] > 0,
                       reinterpret_cast<uint32_t*>(c->xs.as<char>() + off[4 + t]),
                       reinterpret_cast<double2*>(c->xs.as<char>() + off[6 + t]),
                       reinterpret_cast<double2*>(c->xs.as<char>() + off[8 + t]), wide + t, c->stream);
@@ -641,7 +688,7 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
   // idx[b] or idx[b] + 1)
   int64_t nrows[2] = {0, 0};
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
-  for (int t = 0; t < 2; ++t) nrows[t] = (nbk[t] > 0 && hw[t] == 0) ? nbk[t] : 0;
+  for (int t = 0; t < 2; ++t) nrows[t] = (nrow_alloc[t] > 0 && hw[t] == 0) ? nbk[t] : 0;
   c->xs_bytes = total;
   c->xs_persist_bytes = 0;
   if (c->opt.xs_l2_persist) {
@@ -1447,6 +1494,12 @@ int64_t nt_debug_mesh_bytes(const nt_ctx* c) {
   for (const DevBuf* d : {&c->rho, &c->tally, &c->tally_red, &c->rho_code, &c->blk, &c->rho_st})
     b += (int64_t)d->bytes;
   return b;
+}
+
+int32_t nt_debug_density_format(const nt_ctx* c, int32_t* n_distinct) {
+  if (!c || c->stage < ST_MESH) return -1;
+  if (n_distinct) *n_distinct = c->dens_distinct;
+  return c->dens_fmt;
 }
 
 int32_t nt_debug_xs_rows(const nt_ctx* c) {

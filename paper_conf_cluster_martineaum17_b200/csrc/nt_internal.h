@@ -94,10 +94,10 @@ void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally);
 // cross-section tables on the device: the interleaved pairs kv [n + 1], the bucket index
 // idx [nb + 1] (base, shift: the bucket of a bit pattern is (bits - base) >> shift) and the
-// direct bucket rows [nb] (xs_search 0); *wide |= 1 if a bucket spans more than one key
+// direct bucket rows [nb] (xs_search 0; if rows); *wide |= 1 if a bucket spans more than one key
 void launch_xs_prepare(const double* k, const double* v, int64_t n, uint64_t base, int shift,
-                       int64_t nb, uint32_t* idx, double2* kv, double2* row, unsigned int* wide,
-                       cudaStream_t s);
+                       int64_t nb, bool rows, uint32_t* idx, double2* kv, double2* row,
+                       unsigned int* wide, cudaStream_t s);
 // resident CTAs per SM of the resume_prefetch kernel with its ring (phase 2)
 int history_ring_ctas_per_sm(bool tiled);
 void launch_det_apply(const unsigned long long* keys, const double* vals,
@@ -136,6 +136,15 @@ constexpr int kInnerEvents = 256;   // (also best for the parked-particle phase:
 namespace nt {
 // Mesh preparation (nt_kernels.cu).
 cudaError_t launch_density_check(const double* rho, int64_t n, unsigned long long* bad,
+                                 cudaStream_t s);
+// Validation + distinct values in one pass (a chunk of the density): bad[0] += invalid
+// values, distinct bit patterns into the open-addressing set (kDistinctSlots u64, all ones =
+// empty), bad[1] += patterns inserted, bad[2] = 1 once the set is half full.
+constexpr int kDistinctSlots = 4096;
+cudaError_t launch_check_distinct(const double* rho, int64_t n, unsigned long long* bad,
+                                  unsigned long long* set, cudaStream_t s);
+// The set's patterns sorted into uniq[0, count) (count <= kDistinctSlots / 2).
+cudaError_t launch_distinct_sort(const unsigned long long* set, unsigned long long* uniq,
                                  cudaStream_t s);
 // Sort the density bit patterns (k0 -> k1) and write the distinct ones to k0, their count to
 // *d_count.  temp == nullptr: query temp_bytes.

@@ -1188,12 +1188,12 @@ __global__ void xs_rows_kernel(const double2* __restrict__ kv, const uint32_t* _
 }
 
 void launch_xs_prepare(const double* k, const double* v, int64_t n, uint64_t base, int shift,
-                       int64_t nb, uint32_t* idx, double2* kv, double2* row, unsigned int* wide,
-                       cudaStream_t s) {
+                       int64_t nb, bool rows, uint32_t* idx, double2* kv, double2* row,
+                       unsigned int* wide, cudaStream_t s) {
   xs_pairs_kernel<<<(unsigned)((n + 256) / 256), 256, 0, s>>>(k, v, n, kv);
   if (nb <= 0) return;
   xs_index_kernel<<<(unsigned)((nb + 256) / 256), 256, 0, s>>>(k, n, base, shift, nb, idx);
-  xs_rows_kernel<<<(unsigned)((nb + 255) / 256), 256, 0, s>>>(kv, idx, nb, row, wide);
+  if (rows) xs_rows_kernel<<<(unsigned)((nb + 255) / 256), 256, 0, s>>>(kv, idx, nb, row, wide);
 }
 
 __global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, int64_t n,

@@ -85,6 +85,54 @@ __global__ void nd_table_kernel(const unsigned long long* __restrict__ uniq, int
   if (k < nu) tab[k] = __longlong_as_double((long long)uniq[k]) * cn;
 }
 
+// Validation + distinct density values in one pass over a chunk (nt_init_mesh, while the
+// next chunk is still being copied): bad[0] counts values not finite and >= 0; every valid
+// value's bit pattern is inserted into an open-addressing set (kDistinctSlots slots, empty =
+// all ones, which no valid density has); bad[1] counts the distinct patterns inserted and
+// bad[2] != 0 once the set is half full (the caller then falls back to the sorting path).
+__global__ void check_distinct_kernel(const double* __restrict__ rho, int64_t n,
+                                      unsigned long long* bad, unsigned long long* set) {
+  unsigned long long nbad = 0;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n;
+       i += (int64_t)gridDim.x * blockDim.x) {
+    const double v = rho[i];
+    if (!(v >= 0.0) || !isfinite(v)) { ++nbad; continue; }
+    const unsigned long long b = (unsigned long long)__double_as_longlong(v);
+    unsigned h = (unsigned)((b * 0x9E3779B97F4A7C15ull) >> 52) & (kDistinctSlots - 1);
+    for (int probe = 0; probe < kDistinctSlots; ++probe) {
+      const unsigned long long cur = ld_volatile(set + h);
+      if (cur == b) break;
+      if (cur == ~0ull) {
+        if (ld_volatile(bad + 2)) break;            // overflowed: the sort path takes over
+        const unsigned long long old = atomicCAS(set + h, ~0ull, b);
+        if (old == ~0ull) {
+          if (atomicAdd(bad + 1, 1ull) + 1 >= (unsigned long long)(kDistinctSlots / 2)) atomicExch(bad + 2, 1ull);
+          break;
+        }
+        if (old == b) break;
+      }
+      h = (h + 1) & (kDistinctSlots - 1);
+    }
+  }
+  for (int o = 16; o > 0; o >>= 1) nbad += __shfl_xor_sync(kFull, nbad, o);
+  if ((threadIdx.x & 31) == 0 && nbad) atomicAdd(bad, nbad);
+}
+
+// The set's patterns in increasing order: uniq[rank] (one block; <= kDistinctSlots / 2 keys).
+__global__ void distinct_sort_kernel(const unsigned long long* __restrict__ set,
+                                     unsigned long long* __restrict__ uniq) {
+  __shared__ unsigned long long s[kDistinctSlots];
+  for (int k = threadIdx.x; k < kDistinctSlots; k += blockDim.x) s[k] = set[k];
+  __syncthreads();
+  for (int k = threadIdx.x; k < kDistinctSlots; k += blockDim.x) {
+    const unsigned long long b = s[k];
+    if (b == ~0ull) continue;
+    int rank = 0;
+    for (int j = 0; j < kDistinctSlots; ++j) rank += (s[j] != ~0ull && s[j] < b) ? 1 : 0;
+    uniq[rank] = b;
+  }
+}
+
 static unsigned grid_for(int64_t n) {
   const int64_t b = (n + 255) / 256;
   return (unsigned)(b > 148 * 32 ? 148 * 32 : (b < 1 ? 1 : b));
@@ -93,6 +141,18 @@ static unsigned grid_for(int64_t n) {
 cudaError_t launch_density_check(const double* rho, int64_t n, unsigned long long* bad,
                                  cudaStream_t s) {
   density_check_kernel<<<grid_for(n), 256, 0, s>>>(rho, n, bad);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_check_distinct(const double* rho, int64_t n, unsigned long long* bad,
+                                  unsigned long long* set, cudaStream_t s) {
+  if (n > 0) check_distinct_kernel<<<grid_for(n), 256, 0, s>>>(rho, n, bad, set);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_distinct_sort(const unsigned long long* set, unsigned long long* uniq,
+                                 cudaStream_t s) {
+  distinct_sort_kernel<<<1, 1024, 0, s>>>(set, uniq);
   return cudaGetLastError();
 }
 

@@ -146,3 +146,24 @@ def test_two_ranks_nccl(nt, orc, tmp_path, cfgname, decomposition):
             out[k][g] = p[k][keep]
     assert np.all(seen == 1)
     compare_particles(out, op)
+
+
+@pytest.mark.parametrize("n_distinct", [1, 2, 255, 256, 257, 2047, 2048, 5000, 70000])
+def test_density_distinct_values_and_format(nt, n_distinct):
+    """nt_init_mesh counts the distinct density values while the upload runs (a hashed set,
+    falling back to sorting every cell's bit pattern past 2047 values) and picks the lossless
+    u8 (<= 256) / u16 (<= 65536) material codes or the f64 map.  (That the codes
+    reproduce the density exactly is covered by the parity tests on tiny_levels, u16, and
+    small_random, f64.)"""
+    rng = np.random.default_rng(n_distinct)
+    nx, ny = 301, 297                            # ragged, several upload chunks
+    levels = np.unique(rng.uniform(1e-3, 5.0, n_distinct * 2))[:n_distinct]
+    assert len(levels) == n_distinct
+    rho = levels[rng.integers(0, n_distinct, nx * ny)]
+    rho[:n_distinct] = levels[: min(n_distinct, nx * ny)]   # every level present
+    t = nt.Tracker(density_format=0)
+    t.init_mesh(nx, ny, 1.0, 1.0, rho)
+    fmt, nd = t.density_format()
+    t.close()
+    want = "u8" if n_distinct <= 256 else ("u16" if n_distinct <= 65536 else "f64")
+    assert fmt == want and nd == n_distinct
