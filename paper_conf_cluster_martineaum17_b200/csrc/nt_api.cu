@@ -984,7 +984,6 @@ static nt_status track_phases(nt_ctx* c, const TrackParams& bp_in, bool det, uin
       p.park_q = c->defer_q;
       p.park_count = qlen;
       p.park_coll_below = c->opt.defer_below;
-      if (const char* ev = std::getenv("NT_TAIL_PARK")) p.tail_park_below = std::atoi(ev);   // DEV A/B
     }
     launch_history(p, det, g, c->opt.ctas_per_sm, c->opt.tally_mode, c->opt.xs_search, slab,
                    c->stream);

@@ -24,7 +24,6 @@ struct TrackParams {
   // history kernel regime parking
   int32_t phase;              // 1: track [lo, hi) (resume_q null); 2: resume resume_q
   int32_t park_coll_below;    // park a colliding lane while fewer lanes of its warp collide
-  int32_t tail_park_below;    // phase 1, range exhausted: park a warp's lanes once fewer are active
   const int32_t* resume_q;
   const unsigned long long* resume_count;
   int32_t* park_q;            // out-queue of parked local indices

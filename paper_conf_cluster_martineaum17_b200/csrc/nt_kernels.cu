@@ -577,14 +577,6 @@ history_kernel(const __grid_constant__ TrackParams P) {
         }
       }
     }
-    // tail parking: once the phase-1 range is exhausted, a warp left with fewer than
-    // tail_park_below active lanes parks them for the resumed phase and ends
-    if constexpr (!kFused && !kSlab) {
-      if (exhausted && !resume && P.tail_park_below > 0) {
-        const int na = __popc(__ballot_sync(kFull, active));
-        if (na > 0 && na < P.tail_park_below && active) park_to(2u, P.park_q, P.park_count);
-      }
-    }
     if (!__any_sync(kFull, active)) {
       if (kFused && consumer) continue;    // the consumer block at the loop top decides
       if (exhausted) {
