@@ -49,6 +49,23 @@ MUTATIONS = {
         ("            acc += ((w * ds) * sig) * m.H;", "            acc += ((w * dcen * 0.5) * sig) * m.H;"),
     "collision does not advance the census timer":
         ("            dcen = dcen - dc;\n", ""),
+    "X-facet deposit flushed into the entered cell":
+        ("                or_flush(tally, nx, cx, cy, &acc, &dep, st);\n"
+         "                int at_boundary = ox > 0.0 ? cx == nx - 1 : cx == 0;\n"
+         "                if (at_boundary && pb->boundary) { escaped = 1; }\n"
+         "                else if (ox > 0.0) {\n"
+         "                    if (cx == nx - 1) { ox = -ox; iox = -iox; } else { cx += 1; }\n"
+         "                } else {\n"
+         "                    if (cx == 0) { ox = -ox; iox = -iox; } else { cx -= 1; }\n"
+         "                }\n",
+         "                int at_boundary = ox > 0.0 ? cx == nx - 1 : cx == 0;\n"
+         "                if (at_boundary && pb->boundary) { escaped = 1; }\n"
+         "                else if (ox > 0.0) {\n"
+         "                    if (cx == nx - 1) { ox = -ox; iox = -iox; } else { cx += 1; }\n"
+         "                } else {\n"
+         "                    if (cx == 0) { ox = -ox; iox = -iox; } else { cx -= 1; }\n"
+         "                }\n"
+         "                or_flush(tally, nx, cx, cy, &acc, &dep, st);\n"),
     "tie rule: facet axis tie -> X":
         ("        int axis_x = tx < ty;", "        int axis_x = tx <= ty;"),
 }
@@ -60,7 +77,7 @@ def main():
     a = ap.parse_args()
     tmp = Path(tempfile.mkdtemp(prefix="oracle_mut_"))
     ROOT = tmp / "repo"
-    shutil.copytree(REPO, ROOT, ignore=shutil.ignore_patterns(".git", "gpurun_out", "profiles", "build",
+    shutil.copytree(REPO, ROOT, ignore=shutil.ignore_patterns(".git", "gpurun_out", "build",
                                                               "__pycache__"))
     SRC = ROOT / "oracle" / "neutral_oracle.c"
     LIB = ROOT / "oracle" / "liboracle.so"
