@@ -73,6 +73,28 @@ def ncu_traffic(config: str, mode: str):
     return d.get(f"{config}/{mode}")
 
 
+def ncu_inst(config: str, mode: str):
+    """Warp instructions of the tracking kernel(s) per step from a committed ncu capture."""
+    p = ROOT / "profiles" / "ncu_inst.json"
+    if not p.exists():
+        return None
+    return json.loads(p.read_text()).get(f"{config}/{mode}")
+
+
+def issue_roofline(config: str, mode: str, kernel_ms: float, sm_mhz: float, sms: int):
+    """Instruction-issue bound: warp instructions per step (ncu, same workload) over the
+    kernel's live time, against 4 warp schedulers x 1 instruction per clock per SM at the
+    measured SM clock -- the ceiling of a collision-dominated (ALU) kernel."""
+    inst = ncu_inst(config, mode)
+    if not inst or not kernel_ms or not sm_mhz:
+        return None
+    achieved = inst / (kernel_ms / 1e3)
+    peak = sms * 4 * sm_mhz * 1e6
+    return {"bound": "alu", "achieved": achieved, "peak": peak, "unit": "warp inst/s", "frac": achieved / peak,
+            "inst_per_step": inst, "peak_source": f"{sms} SMs x 4 schedulers x {sm_mhz:.0f} MHz (measured clock)",
+            "inst_source": "smsp__inst_executed.sum, profiles/ncu_inst.json"}
+
+
 # ---- clocks sampled during the timed region ------------------------------------------------
 class ClockSampler:
     FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
@@ -436,6 +458,8 @@ def main():
                        "run_timestep + read_tally"}
     tr.close()
 
+    clk_sum = clk.summary()
+    sms = torch.cuda.get_device_properties(local).multi_processor_count
     extras = None
     if rank == 0 and world == 1 and not a.no_extras and a.config == "csp" and a.mode == "history":
         extras = {}
@@ -443,6 +467,10 @@ def main():
             key = f"{c}/{m}" + "".join(f"/{k}={v}" for k, v in o.items())
             try:
                 extras[key] = measure_extra(binding, torch, c, m, o, local)
+                if not o:                    # an ncu capture exists for the default options
+                    ir = issue_roofline(c, m, extras[key]["kernel_ms"], clk_sum.get("sm_mhz"), sms)
+                    if ir:
+                        extras[key]["issue_frac"] = ir["frac"]
             except Exception as ex:          # reported, never fatal for the headline
                 extras[key] = {"error": str(ex)[:200]}
 
@@ -501,11 +529,12 @@ def main():
                 "bound": "l2_red", "achieved": red_rate, "peak": red_peak, "unit": "RED/s",
                 "frac": red_rate / red_peak, "reds_per_launch": reds,
                 "peak_source": "measured: scripts/dev/red_microbench.cu (profiles/r01_v16_red_microbench.json)"},
+            "issue_roofline": issue_roofline(cfg.name, a.mode, track_ms, clk_sum.get("sm_mhz"), sms),
             "cpu_baseline": cpu,
             "extra_configs": extras,
             "e2e": e2e,
             "gpu_launches": launches,
-            "clocks": clk.summary(),
+            "clocks": clk_sum,
         }, a.json_out)
     if world > 1:
         dist.barrier()

@@ -51,6 +51,7 @@ def main():
     hdr, units, rows = raw[0], raw[1], raw[2:]
     lines = [f"# ncu summary: {Path(a.rep).name}", ""]
     traffic = 0.0      # summed over the captured launches (history phases 1 + 2 of one step)
+    inst = 0.0         # warp instructions issued, summed the same way (bench.py's issue roofline)
     for r in rows:
         d = dict(zip(hdr, r))
         u = dict(zip(hdr, units))
@@ -83,6 +84,7 @@ def main():
             return f * mult
         tr = num("dram__bytes_read.sum", 1) + num("dram__bytes_write.sum", 1)
         traffic += tr
+        inst += num("smsp__inst_executed.sum", 1)
         lines.append("")
         lines.append(f"DRAM traffic of this launch (read + write): {tr:.4g} B")
         lines.append("")
@@ -184,6 +186,10 @@ def main():
         p = Path(a.out).parent / "ncu_traffic.json"
         d = json.loads(p.read_text()) if p.exists() else {}
         d[a.traffic_key] = traffic
+        p.write_text(json.dumps(d, indent=1, sort_keys=True) + "\n")
+        p = Path(a.out).parent / "ncu_inst.json"
+        d = json.loads(p.read_text()) if p.exists() else {}
+        d[a.traffic_key] = inst
         p.write_text(json.dumps(d, indent=1, sort_keys=True) + "\n")
     print(f"wrote {a.out}")
 

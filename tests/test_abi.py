@@ -106,3 +106,14 @@ def test_bench_roofline_inputs():
     assert peak is not None and 1e10 < peak < 1e12
     s = {"n_facets": 10, "n_census": 2, "n_killed": 1, "n_alive_start": 3}
     assert bench.algorithmic_bytes(s) == 24 * 10 + 16 * 3 + 138 * 3
+
+
+def test_bench_issue_roofline():
+    """The ALU (instruction-issue) roofline of a collision-dominated config: committed ncu
+    instruction counts over the kernel time against SMs x 4 schedulers x clock."""
+    import bench
+    r = bench.issue_roofline("scatter", "history", 7.4, 1965.0, 148)
+    assert r is not None and r["bound"] == "alu"
+    assert r["peak"] == 148 * 4 * 1965e6
+    assert 0.3 < r["frac"] < 1.0
+    assert bench.issue_roofline("no_such_config", "history", 7.4, 1965.0, 148) is None
