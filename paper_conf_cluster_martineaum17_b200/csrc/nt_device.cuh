@@ -244,6 +244,15 @@ __device__ __forceinline__ void red_add_hint(double* a, double v, uint64_t pol) 
   asm volatile("red.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(a), "d"(v), "l"(pol));
 #endif
 }
+// Fire-and-forget adds to locations a single thread owns (a particle's ledgers, a thread's
+// statistic slots): no load on the critical path at the end of a history.  A thread's own
+// adds to one address apply in program order, so the sums round as the load-add-store did.
+__device__ __forceinline__ void red_add_f64(double* a, double v) {
+  asm volatile("red.global.add.f64 [%0], %1;" ::"l"(a), "d"(v));
+}
+__device__ __forceinline__ void red_add_u32(uint32_t* a, uint32_t v) {
+  asm volatile("red.global.add.u32 [%0], %1;" ::"l"(a), "r"(v));
+}
 // Warp-aggregated flush (tally_mode 1): the lanes executing this call that flush into the
 // same cell are grouped with __match_any_sync; the group's lowest lane adds the group's
 // values (its own first, then the others in lane order) and issues the one RED.  Lanes

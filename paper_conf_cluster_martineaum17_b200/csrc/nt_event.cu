@@ -120,7 +120,7 @@ struct EvKernel {
   __device__ int32_t pid(int s) { return ci(P_CS, s).z; }
 
   __device__ void cnt(int k, uint32_t v) { atomicAdd(s_u + k, (unsigned long long)v); }
-  __device__ void fsum(int k, double v) { sf[k * sstride] += v; }
+  __device__ void fsum(int k, double v) { red_add_f64(sf + k * sstride, v); }
 
   __device__ uint32_t cidx(int32_t cx, int32_t cy) { return (uint32_t)cell_index(P.mesh, cx, cy); }
 
@@ -177,13 +177,13 @@ struct EvKernel {
     P.p.e[pi] = v.e;
     P.p.w[pi] = v.w;
     P.p.mfp[pi] = v.mfp;
-    P.p.dep[pi] += v.dstep;
+    red_add_f64(P.p.dep + pi, v.dstep);         // the particle's ledgers: no load here
     P.p.cx[pi] = v.cx;
     P.p.cy[pi] = v.cy;
     P.p.ctr[pi] = v.ctr;
-    P.p.nfac[pi] += v.nf;
-    P.p.ncol[pi] += v.nc;
-    if (alive) P.p.ncen[pi] += 1u; else P.p.status[pi] = 0u;
+    red_add_u32(P.p.nfac + pi, v.nf);
+    red_add_u32(P.p.ncol + pi, v.nc);
+    if (alive) red_add_u32(P.p.ncen + pi, 1u); else P.p.status[pi] = 0u;
     cnt(SU_FACETS, v.nf);
     cnt(SU_COLLISIONS, v.nc);
     fsum(SF_TALLY, v.dstep);

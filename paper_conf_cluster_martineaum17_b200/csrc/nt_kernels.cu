@@ -170,7 +170,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
 #if NT_SMEM_FSUM
   auto fsum = [&](int k, double v) { s_f[k][t] += v; };
 #else
-  auto fsum = [&](int k, double v) { sf[k * sstride] += v; };
+  auto fsum = [&](int k, double v) { red_add_f64(sf + k * sstride, v); };
 #endif
   s_wabs[t] = 0.0;
   const double* __restrict__ ndtab = (kFmt == kDensU8) ? s_nd : P.mesh.nd_tab;
@@ -824,14 +824,14 @@ history_kernel(const __grid_constant__ TrackParams P) {
           st_stream(PP(e, i), e, pol_stream);
           st_stream(PP(w, i), w, pol_stream);
           st_stream(PP(mfp, i), mfp, pol_stream);
-          st_stream(PP(dep, i), ld_stream(PP(dep, i), pol_stream) + dstep, pol_stream);
+          red_add_f64(PP(dep, i), dstep);           // the particle's ledgers: no load here
           st_stream(PP(cx, i), cx, pol_stream);
           st_stream(PP(cy, i), cy, pol_stream);
           st_stream(PP(ctr, i), ctr, pol_stream);
-          st_stream(PP(nfac, i), ld_stream(PP(nfac, i), pol_stream) + nf, pol_stream);
-          st_stream(PP(ncol, i), ld_stream(PP(ncol, i), pol_stream) + nc, pol_stream);
+          red_add_u32(PP(nfac, i), nf);
+          red_add_u32(PP(ncol, i), nc);
           if (outcome == 1) {
-            (*PP(ncen, i)) += 1u;
+            red_add_u32(PP(ncen, i), 1u);
             if (res) (*PP(status, i)) = 1u;              // was parked (2)
           } else {
             (*PP(status, i)) = 0u;
