@@ -352,6 +352,11 @@ __device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commi
 __device__ __forceinline__ void cp_async_wait_all() { asm volatile("cp.async.wait_all;" ::: "memory"); }
 __device__ __forceinline__ void cp_async_wait_group1() { asm volatile("cp.async.wait_group 1;" ::: "memory"); }
 
+__device__ __forceinline__ uint32_t ld_volatile_u8(const uint8_t* p) {
+  uint32_t v;
+  asm volatile("ld.volatile.global.u8 %0, [%1];" : "=r"(v) : "l"(p));
+  return v;
+}
 __device__ __forceinline__ int32_t ld_volatile(const int32_t* p) {
   return *reinterpret_cast<const volatile int32_t*>(p);
 }

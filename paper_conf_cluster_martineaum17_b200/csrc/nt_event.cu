@@ -488,11 +488,16 @@ struct EvKernel {
   // ---- a new particle (local index in P_CS.z): its slot state and first event ----
   __device__ uint32_t birth(int s) {
     const int32_t pi = pid(s);
-    if (P.p.status[pi] != 1u) return T_FREE;
+    // the state loads go out with the status load (one round trip instead of two)
+    const uint32_t st_i = ld_volatile_u8(P.p.status + pi);
     St v;
-    v.ox = P.p.ox[pi]; v.oy = P.p.oy[pi];
-    v.e = P.p.e[pi];
-    v.cx = P.p.cx[pi]; v.cy = P.p.cy[pi];
+    v.ox = __ldcs(P.p.ox + pi); v.oy = __ldcs(P.p.oy + pi);
+    v.e = __ldcs(P.p.e + pi);
+    v.cx = __ldcs(P.p.cx + pi); v.cy = __ldcs(P.p.cy + pi);
+    v.x = __ldcs(P.p.x + pi); v.y = __ldcs(P.p.y + pi);
+    v.mfp = __ldcs(P.p.mfp + pi); v.w = __ldcs(P.p.w + pi);
+    v.ctr = __ldcs(P.p.ctr + pi);
+    if (st_i != 1u) return T_FREE;
     uint32_t nr = 0;
     const Mat m = refresh_xs(P.xs, ph, v.e, nr);
     if (nr) cnt(SU_XS_RANGE, nr);
@@ -502,15 +507,13 @@ struct EvKernel {
     v.ioy = 1.0 / v.oy;
     if (v.ox == 0.0) { v.exn = ev_inf(); v.iox = ev_inf(); }
     if (v.oy == 0.0) { v.eyn = ev_inf(); v.ioy = ev_inf(); }
-    v.x = P.p.x[pi]; v.y = P.p.y[pi];
-    v.mfp = P.p.mfp[pi]; v.dcen = speed(v.e, ph) * P.dt;
+    v.dcen = speed(v.e, ph) * P.dt;
     v.acc = 0.0; v.dstep = 0.0;
-    v.w = P.p.w[pi]; v.st = m.st; v.H = m.H; v.pa = m.pa;
+    v.st = m.st; v.H = m.H; v.pa = m.pa;
     bool u;
     v.nd = nd_of(v.cx, v.cy, u);
     v.uni = u ? T_UNIBIT : 0u;
     v.nf = 0u; v.nc = 0u;
-    v.ctr = P.p.ctr[pi];
     cnt(SU_ALIVE, 1u);
     c(P_XY, s) = make_double2(v.x, v.y);
     c(P_O, s) = make_double2(v.ox, v.oy);

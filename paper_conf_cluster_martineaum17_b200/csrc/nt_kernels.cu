@@ -523,18 +523,29 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
         if (my < span2) {
           i = resume ? P.resume_q[my] : (int32_t)(P.lo + (int64_t)my);
-          if ((*PP(status, i)) == (resume ? 2u : 1u)) {
+          // the state loads are issued together with the status load (one round trip to
+          // the particle store instead of two; a skipped particle's loads are wasted)
+          const uint32_t st_i = *PP(status, i);
+          x = ld_stream(PP(x, i), pol_stream);
+          y = ld_stream(PP(y, i), pol_stream);
+          ox = ld_stream(PP(ox, i), pol_stream);
+          oy = ld_stream(PP(oy, i), pol_stream);
+          e = ld_stream(PP(e, i), pol_stream);
+          w = ld_stream(PP(w, i), pol_stream);
+          mfp = ld_stream(PP(mfp, i), pol_stream);
+          cx = ld_stream(PP(cx, i), pol_stream);
+          cy = ld_stream(PP(cy, i), pol_stream);
+          ctr = ld_stream(PP(ctr, i), pol_stream);
+          if (resume) {              // the parked state
+            dcen = ld_stream(PP(dcen, i), pol_stream);
+            acc = ld_stream(PP(acc, i), pol_stream);
+            dstep = ld_stream(PP(dstep, i), pol_stream);
+            nf = ld_stream(PP(nf_s, i), pol_stream);
+            nc = ld_stream(PP(nc_s, i), pol_stream);
+            if constexpr (kDet) seq = ld_stream(PP(seq_s, i), pol_stream);
+          }
+          if (st_i == (resume ? 2u : 1u)) {
             active = true;
-            x = ld_stream(PP(x, i), pol_stream);
-            y = ld_stream(PP(y, i), pol_stream);
-            ox = ld_stream(PP(ox, i), pol_stream);
-            oy = ld_stream(PP(oy, i), pol_stream);
-            e = ld_stream(PP(e, i), pol_stream);
-            w = ld_stream(PP(w, i), pol_stream);
-            mfp = ld_stream(PP(mfp, i), pol_stream);
-            cx = ld_stream(PP(cx, i), pol_stream);
-            cy = ld_stream(PP(cy, i), pol_stream);
-            ctr = ld_stream(PP(ctr, i), pol_stream);
             res = resume;
             setup_loaded();
             if constexpr (kXsWalk) {
@@ -550,15 +561,9 @@ history_kernel(const __grid_constant__ TrackParams P) {
               nc = 0u;
               seq = 0u;
               cnt(SU_ALIVE, 1u);
-            } else {                 // the parked state (phase 1 counted the XS clamps)
+            } else {                 // parked (loaded above; phase 1 counted the XS clamps)
               uint32_t nr_dummy = 0;
               m = refresh_xs(P.xs, ph, e, nr_dummy);
-              dcen = (*PP(dcen, i));
-              acc = (*PP(acc, i));
-              dstep = (*PP(dstep, i));
-              nf = (*PP(nf_s, i));
-              nc = (*PP(nc_s, i));
-              if constexpr (kDet) seq = (*PP(seq_s, i));
             }
             // born (or resumed) outside this rank's slab: hand over before any event (and
             // before touching the density, which this rank holds for its columns only)
