@@ -85,6 +85,22 @@ struct Mesh {
 };
 
 constexpr uint32_t kBlkMixed = 255u;   // block-map entry: block holds more than one code
+
+// NT_CHECKS (dev variant, scripts/gpu_r02_chk.sh): device-side bounds checks of the indices
+// the kernels compute -- storage cells, table buckets, queue and ring positions -- run under
+// the GPU parity suite in place of compute-sanitizer (closed on this pool).
+#ifndef NT_CHECKS
+#define NT_CHECKS 0
+#endif
+#if NT_CHECKS
+#include <cassert>
+#define NT_CHECK(c) assert(c)
+#else
+#define NT_CHECK(c) ((void)0)
+#endif
+__device__ __forceinline__ uint32_t storage_cells(const Mesh& M) {
+  return M.tiled ? (uint32_t)M.strip * (uint32_t)((M.ny + 3) / 4) : (uint32_t)M.nx * (uint32_t)M.ny;
+}
 constexpr int kBlkMax = 16384;         // max block-map entries (bytes of shared memory)
 
 // Storage index of cell (cx, cy) in the tally and density arrays.  Tiled layout: 4x4-cell
@@ -439,6 +455,7 @@ __device__ __forceinline__ XsPre xs_begin(const Table& T, double e) {
     r.hi = T.n - 1;
   } else if (T.nb > 0) {
     const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
+    NT_CHECK(b < (uint64_t)T.nb);
     r.lo = (int32_t)xs_ldu(T.idx + b);
     r.hi = (int32_t)xs_ldu(T.idx + b + 1) + 1;
   } else {
@@ -483,6 +500,7 @@ __device__ __forceinline__ double xs_end(const Table& T, XsPre r) {
 // lerp expression as xs_end, hence the same result.
 __device__ __forceinline__ double xs_row(const Table& T, double e) {
   const uint64_t b = ((uint64_t)__double_as_longlong(e) - T.base) >> T.shift;
+  NT_CHECK(b < (uint64_t)T.nb);
   const double2* r = T.row + 3 * b;
   const double2 a = __ldg(r), m = __ldg(r + 1), c = __ldg(r + 2);
   const bool up = m.x <= e;

@@ -122,7 +122,11 @@ struct EvKernel {
   __device__ void cnt(int k, uint32_t v) { atomicAdd(s_u + k, (unsigned long long)v); }
   __device__ void fsum(int k, double v) { red_add_f64(sf + k * sstride, v); }
 
-  __device__ uint32_t cidx(int32_t cx, int32_t cy) { return (uint32_t)cell_index(P.mesh, cx, cy); }
+  __device__ uint32_t cidx(int32_t cx, int32_t cy) {
+    const uint32_t c = (uint32_t)cell_index(P.mesh, cx, cy);
+    NT_CHECK(c < storage_cells(P.mesh));
+    return c;
+  }
 
   __device__ double edge_x(int32_t k) { return __ldg(P.mesh.ex + k); }
   __device__ double edge_y(int32_t k) { return __ldg(P.mesh.ey + k); }

@@ -207,6 +207,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
   // stays inside a uniform block (more spills), and issuing the facet's edge and density
   // loads before its deposit arithmetic (csp +0.5%, split +2%).
   auto dload = [&](int32_t cx_, int32_t cy_, uint32_t ci_) {
+    NT_CHECK(ci_ < storage_cells(P.mesh));
     if constexpr (kBlk) {
       const int32_t lx = kSlab ? cx_ - P.mesh.x0 : cx_;
       uint32_t code = s_blk[(cy_ >> P.mesh.bshift) * P.mesh.nbx + (lx >> P.mesh.bshift)];
@@ -278,6 +279,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       unsigned long long k = 0;
       if (lane == ld) k = atomicAdd(qn, (unsigned long long)__popc(am));
       k = __shfl_sync(am, k, ld) + (unsigned long long)__popc(am & lt_mask);
+      NT_CHECK(k < (unsigned long long)P.park_cap);
       const int64_t C = P.park_cap;
       double* f = P.park_rec + k;
       uint32_t* u = reinterpret_cast<uint32_t*>(P.park_rec + kParkF64 * C) + k;
@@ -317,6 +319,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
       __threadfence();
       st_volatile(q + k, i + 1);
     } else {
+      NT_CHECK(k < (unsigned long long)P.n || q == P.out_q);
       q[k] = i;
     }
     active = false;
@@ -483,6 +486,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
           const bool mine = ((need >> lane) & 1u) && rank < take;
           if (mine) {
             const int r = rpos + rank;
+            NT_CHECK(r < kRingB);
             const unsigned char* hb = ring + rh * kRingHalfBytes;
             const double* f = reinterpret_cast<const double*>(hb) + r;
             const uint32_t* u = reinterpret_cast<const uint32_t*>(hb + kParkF64 * kRingB * 8) + r;
@@ -523,6 +527,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
         const unsigned long long my = base + (unsigned long long)__popc(idle & lt_mask);
         if (my < span2) {
           i = resume ? P.resume_q[my] : (int32_t)(P.lo + (int64_t)my);
+          NT_CHECK(i >= 0 && (int64_t)i < P.n);
           // the state loads are issued together with the status load (one round trip to
           // the particle store instead of two; a skipped particle's loads are wasted)
           const uint32_t st_i = *PP(status, i);
@@ -631,6 +636,7 @@ history_kernel(const __grid_constant__ TrackParams P) {
         int outcome = 0;                      // 0 continue, 1 census, 2 dead
         auto flush = [&]() {
           const uint32_t cell = cidx;                // storage index of the current cell
+          NT_CHECK(cell < storage_cells(P.mesh) && (uint32_t)i < (uint32_t)P.n);
           if constexpr (kDet) {
             const unsigned long long slot = atomicAdd(P.rec_count, 1ull);
             if (slot < P.rec_cap) {

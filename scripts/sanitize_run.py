@@ -48,6 +48,15 @@ def main():
             t.close()
             n += 1
             print(f"{name} history fused={fused}: ok", flush=True)
+        # resume ring (cp.async into shared memory) and the bucket-index-only XS search
+        for opts in ({"resume_prefetch": 1, "defer_below": 33}, {"xs_search": 3}, {"xs_search": 1}):
+            t = binding.setup(cfg, mode="history", **opts)
+            t.run_timestep(cfg.dt)
+            compare_particles(t.read_particles(), op)
+            compare_tally(t.read_tally(), ot, rtol=1e-6, floor=1e-12)
+            t.close()
+            n += 1
+            print(f"{name} history {opts}: ok", flush=True)
     # x-slabs (caller-driven exchange, 2 contexts)
     cfg = wl.CONFIGS["tiny_csp"].with_(n_particles=300)
     ts = [binding.setup(cfg, first_id=lo, n_local=k, rank=r, nranks=2, decomposition=1)
