@@ -213,8 +213,9 @@ def parse():
     ap.add_argument("--defer-below", type=int, default=0,
                     help="collision deferral threshold (0 default 8, 1 off, 33 park every collision)")
     ap.add_argument("--xs-search", type=int, default=0,
-                    help="0 direct bucket rows (one dependent load per lookup), 1 plain binary search, "
-                         "2 cached-bin linear walk, 3 bucket index alone (two dependent loads)")
+                    help="0 unionised grid (one index and one 96 B row for both tables) + direct rows, "
+                         "1 plain binary search, 2 cached-bin linear walk, 3 bucket index alone (two "
+                         "dependent loads), 4 direct bucket rows per table (one dependent load per lookup)")
     ap.add_argument("--resume-prefetch", type=int, default=-1,
                     help="history mode: 1 parked records + cp.async resume ring, 0 particle store + "
                          "index queue, -1 the library default")
@@ -496,8 +497,8 @@ def main():
                        "tally": ["fp64 RED per flush", "warp-aggregated fp64 RED", "CAS-emulated fp64 add",
                                  "shared-memory hot window %s + RED" % (hot_window(cfg),)][a.tally_mode],
                        "defer_below": a.defer_below or 8,
-                       "xs_search": ["direct bucket rows", "binary", "cached-bin walk",
-                                     "bucket index"][a.xs_search],
+                       "xs_search": ["unionised grid + direct rows", "binary", "cached-bin walk",
+                                     "bucket index", "direct bucket rows"][a.xs_search],
                        "xs_l2_persist": bool(a.xs_l2_persist),
                        "particles_per_gpu": n_per, "global_particles": n_total, "dt": cfg.dt,
                        "tables": [len(tables[0]), len(tables[2])],

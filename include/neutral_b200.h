@@ -103,18 +103,24 @@ typedef struct {
                                   such particles -- mostly inside dense matter -- collide
                                   together.  Results are unchanged.  0 -> 8; 1 disables;
                                   at most 33 (33: park every collision)                    */
-    int32_t xs_search;         /* cross-section bin search: 0 direct
-                                  bucket rows -- a bucket index over the keys' bit patterns
-                                  (about four buckets per key) whose every bucket stores the
-                                  three (key, value) pairs its energies can need, so a
-                                  lookup is one dependent 48 B load (built when every
-                                  bucket spans at most one key, else as 3); 1 plain binary
+    int32_t xs_search;         /* cross-section bin search: 0 (default)
+                                  the unionised grid of 4 where built, else the direct rows
+                                  of 4 per table; 4 direct bucket rows -- a bucket index
+                                  over the keys' bit patterns (about four buckets per key)
+                                  whose every bucket stores the three (key, value) pairs
+                                  its energies can need, so a lookup is one dependent 48 B
+                                  load (built when every bucket spans at most one key,
+                                  else as 3); 1 plain binary
                                   search over the table; 2 the paper's cached-index search
                                   -- a linear walk from the particle's previous bin
                                   (history mode, u8 block-map meshes; others use 3); 3 the
                                   bucket index alone (the index pair, then the pairs: two
                                   dependent loads; a binary search inside buckets holding
-                                  more than one key).  All four return the same bin.      */
+                                  more than one key).  The unionised grid (0): one bucket
+                                  index over both tables whose rows hold both tables' pairs
+                                  (96 B), one bucket computation and one row per refresh
+                                  (built when every bucket spans at most one key of each
+                                  table).  All five return the same bin.                  */
     /* physics variants (DESIGN.md §4 R30-R32; the defaults are the paper's problem)      */
     int32_t boundary;          /* 0 reflective on all four sides; 1 vacuum: a
                                   facet on the mesh boundary ends the history (escape)     */
@@ -301,7 +307,7 @@ int64_t nt_debug_alloc_count(void);
  * halo are stored, so this scales as 1/nranks.  -1 for a NULL context. */
 int64_t nt_debug_mesh_bytes(const nt_ctx *ctx);
 /* Which loaded tables have direct bucket rows (xs_search 0): bit 0 scatter, bit 1 capture;
- * -1 for a NULL context. */
+ * bit 2: the unionised grid (xs_search 4) was built; -1 for a NULL context. */
 int32_t nt_debug_xs_rows(const nt_ctx *ctx);
 /* The density storage nt_init_mesh chose: 2 u8 material codes, 1 u16 codes, 0 the f64 map
  * (-1 for a NULL context, or before nt_init_mesh); *n_distinct (if not NULL) = the number

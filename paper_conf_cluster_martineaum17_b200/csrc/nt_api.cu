@@ -105,7 +105,8 @@ struct nt_ctx {
   size_t xs_bytes = 0;                   // bytes of xs in use (keys, values, indexes, pairs)
   size_t xs_persist_bytes = 0;           // xs_l2_persist: the device's persisting L2 carve-out
   Tables tables{};
-  const double2* xs_row[2] = {nullptr, nullptr};   // direct bucket rows (xs_search 0), if built
+  const double2* xs_row[2] = {nullptr, nullptr};   // direct bucket rows (xs_search 0, 4), if built
+  const double2* xs_urow = nullptr;                 // unionised grid rows (xs_search 0), if built
   // particles
   int64_t n_total = 0, first_id = 0, n_local = 0;
   uint64_t seed = 0;
@@ -138,9 +139,10 @@ struct nt_ctx {
 
 namespace {
 
-// The tables as the kernels see them under the xs_search option: 0 the direct bucket rows
-// where the loader could build them (else the bucket index), 1 no index (plain binary
-// search), 2 and 3 the bucket index (2's walk is a kernel instantiation).
+// The tables as the kernels see them under the xs_search option: 0 the unionised grid and
+// the direct bucket rows where the loader could build them (else the bucket index), 1 no
+// index (plain binary search), 2 and 3 the bucket index (2's walk is a kernel
+// instantiation), 4 the direct bucket rows per table.
 // xs_l2_persist: an L2 access-policy window marks the cross-section buffer persisting on the
 // context stream while the step's tracking kernels run (cleared afterwards, also on error
 // paths), so the table lines are not evicted by the tally and particle-store traffic.  The
@@ -157,7 +159,11 @@ static Tables xs_tables(const nt_ctx* c) {
   if (c->opt.xs_search == 1) {
     t.s.nb = 0;
     t.c.nb = 0;
-  } else if (c->opt.xs_search == 0) {
+  } else if (c->opt.xs_search == 4) {     // direct rows per table only
+    t.s.row = c->xs_row[0];
+    t.c.row = c->xs_row[1];
+  } else if (c->opt.xs_search == 0) {     // unionised grid, the direct rows where it does not apply
+    t.urow = c->xs_urow;
     t.s.row = c->xs_row[0];
     t.c.row = c->xs_row[1];
   }
@@ -327,7 +333,7 @@ nt_status nt_create(const nt_options* opt_in, nt_ctx** out) {
   if (opt.refill_min > 32) opt.refill_min = 32;
   if (opt.defer_below == 0) opt.defer_below = def.defer_below;
   if (opt.defer_below < 0 || opt.defer_below > 33) return NT_ERR_ARG;
-  if (opt.xs_search < 0 || opt.xs_search > 3) return NT_ERR_ARG;
+  if (opt.xs_search < 0 || opt.xs_search > 4) return NT_ERR_ARG;
   if (opt.boundary < 0 || opt.boundary > 1 || opt.analog_absorption < 0 ||
       opt.analog_absorption > 1 || opt.roulette < 0 || opt.roulette > 1)
     return NT_ERR_ARG;
@@ -644,10 +650,31 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     nbk[t] = (int32_t)nb;
   }
   // Device buffer: keys, values (as given), the bucket index [nb + 1], the interleaved
-  // (key, value) pairs [n + 1] and the direct bucket rows [nb] (xs_search 0).  Only the
+  // (key, value) pairs [n + 1] and the direct bucket rows [nb] (xs_search 0, 4).  Only the
   // caller's four arrays cross PCIe; the index, pairs and rows are built on the device
   // (xs_prepare: the index by a binary search per bucket, the same bins as a sweep).
-  size_t off[10], total = 0;
+  // unionised grid over both tables (xs_search 0): one bucketing, fine enough for the
+  // denser table, over the union of both key ranges
+  uint64_t ubase = 0;
+  int32_t ushift = 0;
+  int64_t unb = 0;
+  if (nbk[0] > 0 && nbk[1] > 0) {
+    uint64_t a0, a1, c0, c1;
+    std::memcpy(&a0, &h[0][0], 8);
+    std::memcpy(&a1, &h[0][len[0] - 1], 8);
+    std::memcpy(&c0, &h[2][0], 8);
+    std::memcpy(&c1, &h[2][len[2] - 1], 8);
+    const uint64_t lo = a0 < c0 ? a0 : c0, hi = a1 > c1 ? a1 : c1;
+    int64_t target = 4 * (len[0] > len[2] ? len[0] : len[2]);
+    if (target > (1ll << 22)) target = 1ll << 22;
+    int sh = 0;
+    while (((hi - lo) >> sh) >= (uint64_t)target) ++sh;
+    ubase = lo;
+    ushift = sh;
+    unb = (int64_t)((hi - lo) >> sh) + 1;
+    if (unb * 96 > (32ll << 20)) unb = 0;      // as the rows: only while it stays L2-resident
+  }
+  size_t off[11], total = 0;
   for (int k = 0; k < 4; ++k) {
     off[k] = total;
     total += align256((size_t)len[k] * 8);
@@ -669,6 +696,8 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
     off[8 + t] = total;
     total += align256((size_t)nrow_alloc[t] * 48);
   }
+  off[10] = total;
+  total += align256((size_t)unb * 96);
   NT_CUDA(c, c->xs.ensure(total));
   for (int k = 0; k < 4; ++k)
     NT_CUDA(c, cudaMemcpyAsync(c->xs.as<char>() + off[k], h[k], (size_t)len[k] * 8,
@@ -682,13 +711,26 @@ nt_status nt_load_cross_sections(nt_ctx* c, const double* sk, const double* sv, 
                       reinterpret_cast<uint32_t*>(c->xs.as<char>() + off[4 + t]),
                       reinterpret_cast<double2*>(c->xs.as<char>() + off[6 + t]),
                       reinterpret_cast<double2*>(c->xs.as<char>() + off[8 + t]), wide + t, c->stream);
-  unsigned int hw[2] = {1, 1};
-  NT_CUDA(c, cudaMemcpyAsync(hw, wide, 8, cudaMemcpyDeviceToHost, c->stream));
+  NT_CUDA(c, cudaMemsetAsync(wide + 2, 0, 4, c->stream));
+  launch_xs_urows(reinterpret_cast<const double*>(c->xs.as<char>() + off[0]),
+                  reinterpret_cast<const double2*>(c->xs.as<char>() + off[6]), len[0],
+                  reinterpret_cast<const double*>(c->xs.as<char>() + off[2]),
+                  reinterpret_cast<const double2*>(c->xs.as<char>() + off[7]), len[2],
+                  ubase, ushift, unb, reinterpret_cast<double2*>(c->xs.as<char>() + off[10]),
+                  wide + 2, c->stream);
+  unsigned int hw[3] = {1, 1, 1};
+  NT_CUDA(c, cudaMemcpyAsync(hw, wide, 12, cudaMemcpyDeviceToHost, c->stream));
   // direct bucket rows only where every bucket spans at most one key (then the bin is
   // idx[b] or idx[b] + 1)
   int64_t nrows[2] = {0, 0};
   NT_CUDA(c, cudaStreamSynchronize(c->stream));
   for (int t = 0; t < 2; ++t) nrows[t] = (nrow_alloc[t] > 0 && hw[t] == 0) ? nbk[t] : 0;
+  c->xs_urow = (unb > 0 && hw[2] == 0) ? reinterpret_cast<const double2*>(c->xs.as<char>() + off[10]) : nullptr;
+  c->tables.urow = nullptr;                 // selected per launch (xs_tables)
+  c->tables.ubase = ubase;
+  c->tables.ushift = ushift;
+  c->tables.unb = (int32_t)unb;
+  c->tables.ulast = h[0][len[0] - 1] < h[2][len[2] - 1] ? h[0][len[0] - 1] : h[2][len[2] - 1];
   c->xs_bytes = total;
   c->xs_persist_bytes = 0;
   if (c->opt.xs_l2_persist) {
@@ -1504,7 +1546,7 @@ int32_t nt_debug_density_format(const nt_ctx* c, int32_t* n_distinct) {
 
 int32_t nt_debug_xs_rows(const nt_ctx* c) {
   if (!c) return -1;
-  return (c->xs_row[0] ? 1 : 0) | (c->xs_row[1] ? 2 : 0);
+  return (c->xs_row[0] ? 1 : 0) | (c->xs_row[1] ? 2 : 0) | (c->xs_urow ? 4 : 0);
 }
 
 nt_status nt_debug_threefry(nt_ctx* c, const uint64_t* in, int64_t n, uint64_t* out) {

@@ -128,7 +128,7 @@ struct Table {
   const double2* __restrict__ kv;   // (k[i], v[i]) interleaved, [n + 1] (last entry repeats
                                     // n - 1): one 48 B run holds the two bins a bucket spans
   const uint32_t* __restrict__ idx; // [nb + 1]
-  const double2* __restrict__ row;  // xs_search 0: per bucket b the three pairs kv[idx[b]],
+  const double2* __restrict__ row;  // xs_search 0/4: per bucket b the three pairs kv[idx[b]],
                                     // kv[idx[b] + 1], kv[idx[b] + 2] (48 B), or nullptr
   uint64_t base;
   int32_t n, nb, shift, pad;
@@ -138,6 +138,13 @@ struct Table {
 struct Tables {
   Table s;   // scatter
   Table c;   // capture
+  // xs_search 0, unionised grid: one bucket index over both tables' keys (bucket b covers
+  // the bit patterns [ubase + (b << ushift), ...)); row b = the three scatter pairs, then the
+  // three capture pairs its energies can need (96 B), or urow == nullptr
+  const double2* __restrict__ urow;
+  uint64_t ubase;
+  int32_t ushift, unb;
+  double ulast;               // min(klast of both tables): energies below it use urow
 };
 
 // Sub-expressions of DESIGN.md §3 that depend only on run constants.  Each is computed
@@ -491,7 +498,7 @@ __device__ __forceinline__ double xs_end(const Table& T, XsPre r) {
   return v0 + t * (v1 - v0);
 }
 
-// Direct bucket rows (xs_search 0, the default): the loader copies, for every bucket b, the three pairs a
+// Direct bucket rows (xs_search 4, and 0 where the unionised grid does not apply): the loader copies, for every bucket b, the three pairs a
 // bucket spanning at most one key can need into row[3b .. 3b+2], and builds rows only when
 // every bucket spans at most one key.  Then the lookup is ONE dependent load (the 48 B row)
 // instead of two (the index pair, then the run): the index and the pairs are "staged" into
@@ -543,12 +550,31 @@ __device__ __forceinline__ MatPre refresh_begin(const Tables& T, double e) {
   return p;
 }
 
+// one row of the unionised grid: the same bin selection and lerp as xs_row, per table
+__device__ __forceinline__ double xs_urow_lerp(const double2* r, double e) {
+  const double2 a = __ldg(r), m = __ldg(r + 1), c = __ldg(r + 2);
+  const bool up = m.x <= e;
+  const double k0 = up ? m.x : a.x, v0 = up ? m.y : a.y;
+  const double k1 = up ? c.x : m.x, v1 = up ? c.y : m.y;
+  const double t = (e - k0) / (k1 - k0);
+  return v0 + t * (v1 - v0);
+}
+
 __device__ __forceinline__ Mat refresh_xs(const Tables& T, const Phys& ph, double e,
                                           uint32_t& nrange) {
   const double es = clamp_count(e, T.s, nrange);
   const double ea = clamp_count(e, T.c, nrange);
-  const double ss = xs_lookup(T.s, es);
-  const double sa = xs_lookup(T.c, ea);
+  double ss, sa;
+  if (T.urow != nullptr && es == ea && es < T.ulast) {     // uniform branch on T.urow
+    const uint64_t b = ((uint64_t)__double_as_longlong(es) - T.ubase) >> T.ushift;
+    NT_CHECK(b < (uint64_t)T.unb);
+    const double2* r = T.urow + 6 * b;
+    ss = xs_urow_lerp(r, es);
+    sa = xs_urow_lerp(r + 3, ea);
+  } else {
+    ss = xs_lookup(T.s, es);
+    sa = xs_lookup(T.c, ea);
+  }
   const double t = ss + sa;
   Mat m;
   m.st = t * kBarn;

@@ -94,10 +94,15 @@ void launch_slab_unpack(const Soa& p, const SlabRec* src, int64_t n, const int32
 int history_max_ctas_per_sm(bool det, int fmt, bool tiled, bool blk, int minb, int tally);
 // cross-section tables on the device: the interleaved pairs kv [n + 1], the bucket index
 // idx [nb + 1] (base, shift: the bucket of a bit pattern is (bits - base) >> shift) and the
-// direct bucket rows [nb] (xs_search 0; if rows); *wide |= 1 if a bucket spans more than one key
+// direct bucket rows [nb] (xs_search 0, 4; if rows); *wide |= 1 if a bucket spans more than one key
 void launch_xs_prepare(const double* k, const double* v, int64_t n, uint64_t base, int shift,
                        int64_t nb, bool rows, uint32_t* idx, double2* kv, double2* row,
                        unsigned int* wide, cudaStream_t s);
+// unionised grid (xs_search 0): row[6b .. 6b+5] = the scatter then capture pairs of union
+// bucket b (nb buckets over bits base + (b << shift)); *wide |= 1 if unusable
+void launch_xs_urows(const double* ks, const double2* kvs, int64_t ns, const double* kc,
+                     const double2* kvc, int64_t nc, uint64_t base, int shift, int64_t nb,
+                     double2* row, unsigned int* wide, cudaStream_t s);
 // resident CTAs per SM of the resume_prefetch kernel with its ring (phase 2)
 int history_ring_ctas_per_sm(bool tiled);
 void launch_det_apply(const unsigned long long* keys, const double* vals,

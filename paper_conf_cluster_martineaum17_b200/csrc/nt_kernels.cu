@@ -1198,6 +1198,46 @@ __global__ void xs_rows_kernel(const double2* __restrict__ kv, const uint32_t* _
   row[3 * b + 2] = src[2];
 }
 
+// unionised grid (xs_search 0): per bucket of the union index, each table's three pairs
+// (scatter then capture); *wide != 0 if some bucket spans more than one key of a table
+__device__ __forceinline__ int64_t xs_bin_of(const double* __restrict__ k, int64_t n, double v) {
+  if (!(k[0] <= v)) return 0;                 // below the table: its first bin (e is clamped)
+  int64_t lo = 0, hi = n - 1;
+  while (hi - lo > 1) {
+    const int64_t mid = (lo + hi) >> 1;
+    if (k[mid] <= v) lo = mid; else hi = mid;
+  }
+  return lo;
+}
+__device__ __forceinline__ double xs_bucket_value(uint64_t base, int shift, int64_t b) {
+  const uint64_t bits = base + ((uint64_t)b << shift);
+  return bits >= 0x7ff0000000000000ull ? __longlong_as_double(0x7ff0000000000000ll)
+                                       : __longlong_as_double((long long)bits);
+}
+__global__ void xs_urow_kernel(const double* __restrict__ ks, const double2* __restrict__ kvs, int64_t ns,
+                               const double* __restrict__ kc, const double2* __restrict__ kvc, int64_t nc,
+                               uint64_t base, int shift, int64_t nb, double2* __restrict__ row,
+                               unsigned int* wide) {
+  const int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  if (b >= nb) return;
+  const double v0 = xs_bucket_value(base, shift, b), v1 = xs_bucket_value(base, shift, b + 1);
+  const int64_t s0 = xs_bin_of(ks, ns, v0), s1 = xs_bin_of(ks, ns, v1);
+  const int64_t c0 = xs_bin_of(kc, nc, v0), c1 = xs_bin_of(kc, nc, v1);
+  if (s1 - s0 > 1 || c1 - c0 > 1) atomicOr(wide, 1u);
+  for (int j = 0; j < 3; ++j) {
+    row[6 * b + j] = kvs[s0 + j];
+    row[6 * b + 3 + j] = kvc[c0 + j];
+  }
+}
+
+void launch_xs_urows(const double* ks, const double2* kvs, int64_t ns, const double* kc,
+                     const double2* kvc, int64_t nc, uint64_t base, int shift, int64_t nb,
+                     double2* row, unsigned int* wide, cudaStream_t s) {
+  if (nb <= 0) return;
+  xs_urow_kernel<<<(unsigned)((nb + 255) / 256), 256, 0, s>>>(ks, kvs, ns, kc, kvc, nc, base, shift,
+                                                               nb, row, wide);
+}
+
 void launch_xs_prepare(const double* k, const double* v, int64_t n, uint64_t base, int shift,
                        int64_t nb, bool rows, uint32_t* idx, double2* kv, double2* row,
                        unsigned int* wide, cudaStream_t s) {
@@ -1214,6 +1254,12 @@ __global__ void xs_debug_kernel(const Tables T, const double* __restrict__ e, in
   uint32_t dummy = 0;
   const double es = clamp_count(e[i], T.s, dummy);
   const double ea = clamp_count(e[i], T.c, dummy);
+  if (T.urow != nullptr && es == ea && es < T.ulast) {       // the unionised grid (xs_search 0)
+    const uint64_t b = ((uint64_t)__double_as_longlong(es) - T.ubase) >> T.ushift;
+    os[i] = xs_urow_lerp(T.urow + 6 * b, es);
+    oa[i] = xs_urow_lerp(T.urow + 6 * b + 3, ea);
+    return;
+  }
   os[i] = xs_lookup(T.s, es);
   oa[i] = xs_lookup(T.c, ea);
 }

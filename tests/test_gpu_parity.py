@@ -52,7 +52,7 @@ def test_threefry_words_bit_exact(nt, orc):
         assert tuple(int(v) for v in o) == orc.threefry2x64_20(*[int(v) for v in row])
 
 
-@pytest.mark.parametrize("xs_search", [0, 1, 3])
+@pytest.mark.parametrize("xs_search", [0, 1, 3, 4])
 @pytest.mark.parametrize("cfgname", ["csp", "tiny_csp"])
 def test_xs_lookup_matches_oracle(nt, orc, cfgname, xs_search):
     cfg = wl.CONFIGS[cfgname]
@@ -64,15 +64,15 @@ def test_xs_lookup_matches_oracle(nt, orc, cfgname, xs_search):
     es = np.concatenate([np.exp(rng.uniform(np.log(1e-5), np.log(2e7), 3000)), sk[:50], sk[-50:],
                          ck[::997], [sk[0], sk[-1], 1.0, 1e6]])
     gs, ga = t.debug_xs(es)
-    if xs_search == 0 and cfgname == "csp":
-        assert t.xs_rows() == 3            # the paper tables get direct rows
+    if xs_search in (0, 4) and cfgname == "csp":
+        assert t.xs_rows() == 7            # the paper tables get direct rows and the union grid
     t.close()
     for e, a, b in zip(es, gs, ga):
         assert a == orc.xs_lookup(sk, sv, e)
         assert b == orc.xs_lookup(ck, cv, e)
 
 
-@pytest.mark.parametrize("xs_search", [0, 3])
+@pytest.mark.parametrize("xs_search", [0, 3, 4])
 def test_xs_random_tables(nt, orc, xs_search):
     rng = np.random.default_rng(9)
     for n in [2, 3, 5, 17, 64, 1000]:
@@ -231,7 +231,7 @@ def test_parity_collision_deferral(nt, orc, cfgname, defer_below):
     assert np.all(gp["status"] <= 1)
 
 
-@pytest.mark.parametrize("xs_search", [1, 2, 3])
+@pytest.mark.parametrize("xs_search", [1, 2, 3, 4])
 @pytest.mark.parametrize("cfgname", ["small_scatter", "small_csp", "tiny_split", "small_mosaic", "tiny_A12"])
 def test_parity_xs_search_strategies(nt, orc, cfgname, xs_search):
     """Plain binary search (1), the paper's cached-index linear walk (2) and the
