@@ -88,6 +88,30 @@ def test_xs_random_tables(nt, orc, xs_search):
             assert b == orc.xs_lookup(k, v[::-1].copy(), e)
 
 
+@pytest.mark.parametrize("xs_search", [0, 4])
+def test_xs_tables_with_different_ranges(nt, orc, xs_search):
+    """The unionised grid (0) over two tables with different, partly overlapping key ranges
+    and densities: energies inside both ranges use the union rows, energies clamped by one
+    table fall back to the per-table rows -- every lookup equals the oracle's binary search
+    (P:252-265)."""
+    rng = np.random.default_rng(21)
+    ks = np.geomspace(1e-3, 1e3, 700)
+    kc = np.geomspace(1e-1, 1e5, 3000)
+    vs = rng.uniform(1.0, 3.0, ks.size)
+    vc = rng.uniform(0.1, 9.0, kc.size)
+    t = nt.Tracker(xs_search=xs_search)
+    t.init_mesh(4, 4, 1.0, 1.0, np.ones(16))
+    t.load_cross_sections(ks, vs, kc, vc)
+    es = np.concatenate([np.exp(rng.uniform(np.log(1e-4), np.log(1e6), 4000)), ks, kc[::7],
+                         [1e-3, 1e-1, 1e3, 1e5, np.nextafter(1e3, 0), np.nextafter(1e-1, 1)]])
+    gs, ga = t.debug_xs(es)
+    assert t.xs_rows() & 4                      # the union grid was built
+    t.close()
+    for e, a, b in zip(es, gs, ga):        # each table clamps the energy into its own range
+        assert a == orc.xs_lookup(ks, vs, min(max(e, ks[0]), ks[-1]))
+        assert b == orc.xs_lookup(kc, vc, min(max(e, kc[0]), kc[-1]))
+
+
 @pytest.mark.parametrize("cfgname", ["tiny_csp", "csp", "split"])
 def test_inject_matches_oracle(nt, orc, cfgname):
     cfg = wl.CONFIGS[cfgname].with_(n_particles=5000)
