@@ -159,7 +159,9 @@ typedef struct {
                                   tables persisting (large lookup tables can
                                   become the bottleneck), with a device-wide persisting
                                   carve-out of up to the tables' size set at
-                                  nt_load_cross_sections and released at nt_destroy;
+                                  nt_load_cross_sections and released at nt_destroy (the
+                                  limit is device-wide, and a window the caller had set on
+                                  the same stream is replaced, then cleared);
                                   0: no window (default)                                  */
     int32_t resume_prefetch;   /* history mode, production, default kernel options: 1 a
                                   parked particle's state is written as a queue-ordered
